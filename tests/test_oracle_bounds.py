@@ -1,0 +1,48 @@
+"""Pins for the bounds (oracle/bounds.py): closed forms and LP cross-checks."""
+import pytest
+
+from oracle import bounds
+
+T_THR = {"POTRF": 3.0, "TRSM": 1.2, "SYRK": 1.1, "GEMM": 2.0}
+T_LAT = {"POTRF": 5.0, "TRSM": 2.0, "SYRK": 1.5, "GEMM": 3.0}
+
+
+@pytest.mark.parametrize("N", [1, 2, 4, 10, 20])
+def test_mixed_dominates(N):
+    for M in (1, 2, 8):
+        a = bounds.area(N, T_THR, M)
+        c = bounds.chain(N, T_LAT)
+        m = bounds.mixed(N, T_THR, T_LAT, M)
+        assert m >= a and m >= c and m == max(a, c)
+        assert bounds.critical_path(N, T_LAT) >= c
+
+
+@pytest.mark.parametrize("N", [2, 5, 12])
+def test_lp_single_resource_equals_closed_form(N):
+    T = {"gpu": T_THR}
+    for M in (1, 3):
+        lp = bounds.lp_area_mixed(N, T, {"gpu": M}, mixed_chain=False)
+        assert abs(lp - bounds.area(N, T_THR, M)) < 1e-9 * lp
+        lpm = bounds.lp_area_mixed(N, T, {"gpu": M}, mixed_chain=True)
+        assert abs(lpm - max(bounds.area(N, T_THR, M), bounds.chain(N, T_THR))) < 1e-9 * lpm
+
+
+def test_lp_related_platform_closed_form():
+    """'Related' platform (L791-797): GPU exactly K times faster on every kernel ->
+    area = W_cpu / (M_cpu + K M_gpu)."""
+    N, K, Mc, Mg = 8, 7.0, 9, 3
+    Tc = {"POTRF": 1.0, "TRSM": 3.0, "SYRK": 3.0, "GEMM": 6.0}
+    Tg = {t: v / K for t, v in Tc.items()}
+    W = bounds.area(N, Tc, 1)
+    lp = bounds.lp_area_mixed(N, {"cpu": Tc, "gpu": Tg}, {"cpu": Mc, "gpu": Mg}, mixed_chain=False)
+    assert abs(lp - W / (Mc + K * Mg)) < 1e-9 * lp
+
+
+def test_critical_path_unit_weights():
+    assert bounds.critical_path(7, {k: 1.0 for k in T_THR}) == 3 * 7 - 2
+
+
+def test_gemm_peak():
+    # R_G = 2 nb^3 / T_G; bound = (n^3/3) / (M R_G)
+    n, nb = 9600, 960
+    assert abs(bounds.gemm_peak(n, nb, 2.0, 1) - (n ** 3 / 3) / (2 * nb ** 3 / 2.0)) < 1e-9
