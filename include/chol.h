@@ -1,0 +1,154 @@
+/*
+ * chol.h -- C-ABI of the B200-native tiled FP64 Cholesky library (libchol_b200.so).
+ *
+ * What it computes (Agullo et al., HCW 2015, /root/reference/PAPER.md):
+ *   "the Cholesky decomposition of a dense, symmetric, and positive-definite
+ *    double-precision matrix A, into the product L L^T, where L is lower
+ *    triangular and has positive diagonal elements" (L135-138; A = L L^T,
+ *    L166-168), by the tiled right-looking algorithm of Algorithm 1 (L172-181):
+ *    the matrix is an N x N grid of nb x nb tiles (L183-186) and four tile
+ *    kernels -- POTRF (L196-199), TRSM (L200-202), SYRK (L207-208) and GEMM
+ *    (L203-206) -- overwrite A_ij with L_ij in place (L209-211).  Tasks run as
+ *    soon as their direct data dependencies (L213-220) are met.
+ *
+ * Conventions: n = matrix order, nb = tile size,
+ * N = n / nb (the paper swaps the letters, reading R1).  All matrices are
+ * ROW-MAJOR: element (r, c) of X with leading dimension ld is X[r*ld + c].
+ *
+ * Status codes: every call returns int; 0 = OK, < 0 = error:
+ *   -1  n <= 0
+ *   -2  nb <= 0, n % nb != 0, or nb % 32 != 0 (kernel tile granularity)
+ *   -3  ngpus < 1, more GPUs than visible devices, or grid_p*grid_q != ngpus
+ *   -4  null or misaligned (not 8-byte aligned) pointer, or null plan
+ *   -5  lda / ldl < n
+ *   -6  bad options (unknown policy / executor / negative values)
+ *   -7  chol_trace before any chol_factor*, or tracing disabled
+ *   -8  operation not supported by this build (e.g. ngpus > 1 in one process)
+ *   -9  device out of memory while planning
+ *   -100 - e   CUDA runtime error e
+ *   -200 - e   NCCL error e
+ * A non-SPD input is NOT an error status: it is reported through *info.
+ *
+ * Thread safety: a plan may be used by one host thread at a time.
+ */
+#ifndef CHOL_B200_H
+#define CHOL_B200_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct chol_plan_s* chol_plan_t;
+
+/* Scheduling policies of the device-side task scheduler (§V-A,
+ * and the static rules of §V-C3). */
+enum {
+  CHOL_POLICY_DYNAMIC = 0,     /* dependency-ready FIFO, any worker (dmda analogue, L645-651) */
+  CHOL_POLICY_CP_PRIORITY = 1, /* ready tasks popped by bottom-level priority (dmdas / HEFT,
+                                  L652-660, L299-301) */
+  CHOL_POLICY_STATIC = 2       /* CP priority + static placement: POTRF and the TRSMs within
+                                  trsm_pin_distance tiles of the diagonal are pinned to the
+                                  latency workers; the other TRSMs and all SYRK/GEMM go to the
+                                  throughput workers (the paper's TRSM-distance rule,
+                                  L1019-1025, transposed to one GPU's two worker classes) */
+};
+
+/* Executors. */
+enum {
+  CHOL_EXEC_SCHEDULER = 0, /* one persistent scheduler kernel per GPU (default) */
+  CHOL_EXEC_HOST = 1       /* host-sequenced baseline: per k, POTRF / TRSM batch / update
+                              batch launches in Algorithm 1 order (no device scheduler) */
+};
+
+/* Options; a zero-initialised struct means "defaults". */
+typedef struct {
+  int policy;            /* CHOL_POLICY_* (default DYNAMIC) */
+  int trsm_pin_distance; /* STATIC only: TRSM_i_k with i-k <= d are pinned (0 = N, all) */
+  int latency_workers;   /* STATIC only: CTAs reserved for pinned tasks (0 = 8) */
+  int grid_p, grid_q;    /* 2D block-cyclic process grid (0,0 = 1 x ngpus) */
+  int trace;             /* 1 = record per-task t0/t1 (needed by chol_trace) */
+  int executor;          /* CHOL_EXEC_* */
+  int workers;           /* persistent CTAs (0 = one per SM) */
+} chol_opts_t;
+
+/* One trace record per task (Fig. 12). */
+typedef struct {
+  uint8_t type;    /* 0 POTRF, 1 TRSM, 2 SYRK, 3 GEMM */
+  uint8_t gpu;     /* rank / device that ran it */
+  uint16_t worker; /* SM id of the CTA that completed the task's last sub-task */
+  int32_t i, j, k; /* Fig. 1 indices: POTRF_k (i=j=k), TRSM_i_k (j=k), SYRK_j_k (i=j), GEMM_i_j_k */
+  uint64_t t0_ns;  /* first sub-task start, %globaltimer ns, relative to the factorization start */
+  uint64_t t1_ns;  /* last sub-task end */
+} chol_task_rec_t;
+
+/* Plan an n x n factorization in nb x nb tiles on ngpus GPUs (the devices
+ * 0..ngpus-1 of this process; this build supports ngpus == 1 here and
+ * multi-GPU through chol_plan_dist).  Allocates the tile store
+ * (N(N+1)/2 tiles, 8*nb*nb bytes each), the task tables and the scheduler
+ * state on the device.  *out receives the plan; free it with chol_destroy. */
+int chol_plan(int64_t n, int64_t nb, int ngpus, chol_plan_t* out);
+int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t* opts, chol_plan_t* out);
+
+/* Factor A = L L^T.  A (lda >= n) and L (ldl >= n) are caller-owned pointers to
+ * row-major n x n doubles, either device memory of the plan's GPU or host memory
+ * (pinned or pageable; detected with cudaPointerGetAttributes).  Only the lower
+ * triangle of A is read.  On return L holds the lower factor with its strictly
+ * upper part set to zero.  A == L with lda == ldl (in place) is allowed.
+ * Synchronous.  *info (host int) = 0 on success, or j > 0 if the leading minor of
+ * order j is not positive definite (1-based global column of the first pivot d
+ * with !(d > 0), NaN included); then columns < nb*floor((j-1)/nb) of L are valid
+ * and the rest is unspecified. */
+int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* L, int64_t ldl, int* info);
+
+/* Per-task trace of the last factorization (requires opts.trace = 1).
+ * Copies min(cap, #tasks) records into recs (host memory, may be NULL with
+ * cap = 0 to query), sets *nrecs to the number of tasks and *makespan_s to
+ * max t1 - min t0 in seconds. */
+int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int64_t* nrecs, double* makespan_s);
+
+int chol_destroy(chol_plan_t p);
+const char* chol_strerror(int status);
+
+/* ---- helpers for benchmarks / tests (not part of the paper's problem statement) ---- */
+
+/* Fill the plan's tile store in place with a seeded synthetic SPD matrix:
+ * family 0 = "uniform" (A_ij = u(i,j) + n [i==j]), family 1 = "integer"
+ * (A = L0 L0^T, exact), with the counter-based recipe of DESIGN.md
+ * "Input recipe" (same bits as the Python generator spdgen/). */
+int chol_generate(chol_plan_t p, uint64_t seed, int family);
+
+/* Copy a row-major matrix (host or device pointer) into / out of the tile store.
+ * chol_gather writes L with its strictly upper part zeroed. */
+int chol_scatter(chol_plan_t p, const double* A, int64_t lda);
+int chol_gather(chol_plan_t p, double* L, int64_t ldl);
+
+/* Factor the tile store in place (no layout conversion); *info as chol_factor. */
+int chol_factor_inplace(chol_plan_t p, int* info);
+
+/* Device time of the last factorization (CUDA events around the launches on the
+ * plan's stream) and of the last layout conversion (scatter + gather). */
+int chol_last_times(chol_plan_t p, double* factor_s, double* layout_s);
+
+/* The plan's CUDA stream (cudaStream_t) and tile size used by the kernels. */
+int chol_get_stream(chol_plan_t p, void** stream);
+int chol_get_info(chol_plan_t p, int64_t* n, int64_t* nb, int* block, int* workers, int* policy,
+                  int* executor);
+
+/* Run ONE tile task (type 0..3 with Fig. 1 indices i, j, k) on the tile store,
+ * alone on the GPU, `reps` times back to back (reps >= 1; for calibration the
+ * operands are simply re-used).  Returns the mean device time per run in *ms.
+ * Used by the per-kernel parity tests and the calibration of T_t^lat. */
+int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double* ms);
+
+/* Run `count` independent instances of tile task type `type` concurrently
+ * (count GEMMs / SYRKs / TRSMs on distinct output tiles of the store, POTRFs on
+ * distinct diagonal tiles) and return the device time per instance in *ms
+ * (throughput time T_t^thr, reading R9).  Overwrites the store. */
+int chol_run_batch(chol_plan_t p, int type, int count, int reps, double* ms);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* CHOL_B200_H */

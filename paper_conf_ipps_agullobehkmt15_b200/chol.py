@@ -1,0 +1,209 @@
+"""Thin ctypes binding of libchol_b200.so (include/chol.h) -- argument marshalling only.
+
+Every function has the C name and returns what the C call returns (status codes are
+turned into ``CholError`` exceptions).  Matrices are passed as raw pointers taken from
+torch tensors (``data_ptr()``, device or pinned host memory) or numpy arrays (host).
+There is no CPU fallback: if the CUDA library is missing this module raises on import.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libchol_b200.so")
+
+POLICY_DYNAMIC, POLICY_CP_PRIORITY, POLICY_STATIC = 0, 1, 2
+EXEC_SCHEDULER, EXEC_HOST = 0, 1
+POTRF, TRSM, SYRK, GEMM = 0, 1, 2, 3
+TYPE_NAMES = ("POTRF", "TRSM", "SYRK", "GEMM")
+
+
+class CholError(RuntimeError):
+    def __init__(self, status: int, what: str):
+        self.status = status
+        super().__init__(f"{what}: status {status} ({chol_strerror(status)})")
+
+
+class chol_opts_t(ctypes.Structure):
+    _fields_ = [("policy", ctypes.c_int), ("trsm_pin_distance", ctypes.c_int),
+                ("latency_workers", ctypes.c_int), ("grid_p", ctypes.c_int), ("grid_q", ctypes.c_int),
+                ("trace", ctypes.c_int), ("executor", ctypes.c_int), ("workers", ctypes.c_int)]
+
+
+class chol_task_rec_t(ctypes.Structure):
+    _fields_ = [("type", ctypes.c_uint8), ("gpu", ctypes.c_uint8), ("worker", ctypes.c_uint16),
+                ("i", ctypes.c_int32), ("j", ctypes.c_int32), ("k", ctypes.c_int32),
+                ("t0_ns", ctypes.c_uint64), ("t1_ns", ctypes.c_uint64)]
+
+
+def _load():
+    if not os.path.exists(LIB_PATH):
+        raise ImportError(f"{LIB_PATH} is missing: run __graft_entry__.build() (there is no CPU fallback)")
+    L = ctypes.CDLL(LIB_PATH)
+    P, i64, i32, u64, vp = ctypes.c_void_p, ctypes.c_int64, ctypes.c_int, ctypes.c_uint64, ctypes.c_void_p
+    dp = ctypes.POINTER(ctypes.c_double)
+    sig = {
+        "chol_plan": ([i64, i64, i32, ctypes.POINTER(P)], i32),
+        "chol_plan_ex": ([i64, i64, i32, ctypes.POINTER(chol_opts_t), ctypes.POINTER(P)], i32),
+        "chol_factor": ([P, vp, i64, vp, i64, ctypes.POINTER(i32)], i32),
+        "chol_trace": ([P, ctypes.POINTER(chol_task_rec_t), i64, ctypes.POINTER(i64), dp], i32),
+        "chol_destroy": ([P], i32),
+        "chol_strerror": ([i32], ctypes.c_char_p),
+        "chol_generate": ([P, u64, i32], i32),
+        "chol_scatter": ([P, vp, i64], i32),
+        "chol_gather": ([P, vp, i64], i32),
+        "chol_factor_inplace": ([P, ctypes.POINTER(i32)], i32),
+        "chol_last_times": ([P, dp, dp], i32),
+        "chol_get_stream": ([P, ctypes.POINTER(vp)], i32),
+        "chol_get_info": ([P, ctypes.POINTER(i64), ctypes.POINTER(i64), ctypes.POINTER(i32),
+                           ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(i32)], i32),
+        "chol_run_task": ([P, i32, i32, i32, i32, i32, dp], i32),
+        "chol_run_batch": ([P, i32, i32, i32, dp], i32),
+    }
+    for name, (args, res) in sig.items():
+        f = getattr(L, name)
+        f.argtypes = args
+        f.restype = res
+    return L
+
+
+_lib = _load()
+EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_destroy", "chol_strerror",
+            "chol_generate", "chol_scatter", "chol_gather", "chol_factor_inplace", "chol_last_times",
+            "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch")
+
+
+def _ptr(x) -> int:
+    """Raw address of a torch tensor / numpy array / int."""
+    if isinstance(x, int):
+        return x
+    if hasattr(x, "data_ptr"):
+        return x.data_ptr()
+    if hasattr(x, "ctypes"):
+        return x.ctypes.data
+    raise TypeError(f"cannot take a pointer of {type(x)}")
+
+
+def _check(st: int, what: str) -> None:
+    if st != 0:
+        raise CholError(st, what)
+
+
+def chol_strerror(status: int) -> str:
+    return _lib.chol_strerror(status).decode()
+
+
+def chol_plan(n: int, nb: int, ngpus: int = 1) -> int:
+    h = ctypes.c_void_p()
+    _check(_lib.chol_plan(n, nb, ngpus, ctypes.byref(h)), "chol_plan")
+    return h.value
+
+
+def chol_plan_ex(n: int, nb: int, ngpus: int = 1, **opts) -> int:
+    o = chol_opts_t(**opts)
+    h = ctypes.c_void_p()
+    _check(_lib.chol_plan_ex(n, nb, ngpus, ctypes.byref(o), ctypes.byref(h)), "chol_plan_ex")
+    return h.value
+
+
+def chol_factor(plan: int, A, lda: int, L, ldl: int) -> int:
+    info = ctypes.c_int(0)
+    _check(_lib.chol_factor(plan, _ptr(A), lda, _ptr(L), ldl, ctypes.byref(info)), "chol_factor")
+    return info.value
+
+
+def chol_factor_inplace(plan: int) -> int:
+    info = ctypes.c_int(0)
+    _check(_lib.chol_factor_inplace(plan, ctypes.byref(info)), "chol_factor_inplace")
+    return info.value
+
+
+def chol_trace(plan: int):
+    """Returns (records as a list of dicts, makespan in seconds)."""
+    n = ctypes.c_int64(0)
+    ms = ctypes.c_double(0.0)
+    _check(_lib.chol_trace(plan, None, 0, ctypes.byref(n), ctypes.byref(ms)), "chol_trace")
+    recs = (chol_task_rec_t * max(n.value, 1))()
+    _check(_lib.chol_trace(plan, recs, n.value, ctypes.byref(n), ctypes.byref(ms)), "chol_trace")
+    out = [{"type": r.type, "gpu": r.gpu, "worker": r.worker, "i": r.i, "j": r.j, "k": r.k,
+            "t0_ns": r.t0_ns, "t1_ns": r.t1_ns} for r in recs[:n.value]]
+    return out, ms.value
+
+
+def chol_destroy(plan: int) -> None:
+    _check(_lib.chol_destroy(plan), "chol_destroy")
+
+
+def chol_generate(plan: int, seed: int, family: int = 0) -> None:
+    _check(_lib.chol_generate(plan, seed, family), "chol_generate")
+
+
+def chol_scatter(plan: int, A, lda: int) -> None:
+    _check(_lib.chol_scatter(plan, _ptr(A), lda), "chol_scatter")
+
+
+def chol_gather(plan: int, L, ldl: int) -> None:
+    _check(_lib.chol_gather(plan, _ptr(L), ldl), "chol_gather")
+
+
+def chol_last_times(plan: int) -> tuple[float, float]:
+    f, l = ctypes.c_double(), ctypes.c_double()
+    _check(_lib.chol_last_times(plan, ctypes.byref(f), ctypes.byref(l)), "chol_last_times")
+    return f.value, l.value
+
+
+def chol_get_stream(plan: int) -> int:
+    s = ctypes.c_void_p()
+    _check(_lib.chol_get_stream(plan, ctypes.byref(s)), "chol_get_stream")
+    return s.value or 0
+
+
+def chol_get_info(plan: int) -> dict:
+    n, nb = ctypes.c_int64(), ctypes.c_int64()
+    bs, w, pol, ex = ctypes.c_int(), ctypes.c_int(), ctypes.c_int(), ctypes.c_int()
+    _check(_lib.chol_get_info(plan, ctypes.byref(n), ctypes.byref(nb), ctypes.byref(bs), ctypes.byref(w),
+                              ctypes.byref(pol), ctypes.byref(ex)), "chol_get_info")
+    return {"n": n.value, "nb": nb.value, "block": bs.value, "workers": w.value, "policy": pol.value,
+            "executor": ex.value}
+
+
+def chol_run_task(plan: int, type: int, i: int, j: int, k: int, reps: int = 1) -> float:
+    ms = ctypes.c_double()
+    _check(_lib.chol_run_task(plan, type, i, j, k, reps, ctypes.byref(ms)), "chol_run_task")
+    return ms.value
+
+
+def chol_run_batch(plan: int, type: int, count: int, reps: int = 1) -> float:
+    ms = ctypes.c_double()
+    _check(_lib.chol_run_batch(plan, type, count, reps, ctypes.byref(ms)), "chol_run_batch")
+    return ms.value
+
+
+class Plan:
+    """RAII wrapper: ``with Plan(n, nb, executor=EXEC_HOST) as p: info = p.factor(A, L)``."""
+
+    def __init__(self, n: int, nb: int, ngpus: int = 1, **opts):
+        self.n, self.nb = n, nb
+        self.h = chol_plan_ex(n, nb, ngpus, **opts)
+
+    def factor(self, A, L=None, lda: int | None = None, ldl: int | None = None) -> int:
+        L = A if L is None else L
+        return chol_factor(self.h, A, lda or self.n, L, ldl or self.n)
+
+    def close(self):
+        if self.h:
+            chol_destroy(self.h)
+            self.h = 0
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.close()
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
