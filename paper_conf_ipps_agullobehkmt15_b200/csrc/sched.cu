@@ -1,8 +1,483 @@
+// Device-side dependency-counting task scheduler (CHOL_EXEC_SCHEDULER).
+//
+// PAPER.md §II-B2 / §V-A (L283-306, L633-660): tasks of the Algorithm 1 DAG run as
+// soon as their direct data dependencies (L213-220) are satisfied; the policy decides
+// which ready task a free worker takes.  B200 form: ONE persistent kernel, one CTA
+// per SM ("worker").  Each task is a node with a dependency counter; when it becomes
+// ready all its CTA sub-tasks ("jobs") are appended to a device ready queue; a worker
+// pops a job, runs the tile op (tile_ops.cuh), and the worker that finishes a node's
+// last job decrements the successors' counters and enqueues those reaching zero.
+// POTRF_k is a chain of inner nodes (nested tiled Cholesky of the diagonal tile with
+// block BS: DIAG b -> PANEL b -> UPDATE b -> DIAG b+1 ...).
+//
+// Policies (include/chol.h): DYNAMIC = one FIFO; CP_PRIORITY = kBuckets FIFOs keyed by
+// the bottom-level of the task (HEFT/dmdas, L299-301, L655-660), a worker takes the
+// highest non-empty bucket; STATIC = CP_PRIORITY + POTRF and the TRSMs within
+// trsm_pin_distance of the diagonal are pinned to `latency_workers` dedicated CTAs
+// (the paper's TRSM-distance rule, L1019-1025).
+#include <algorithm>
+#include <climits>
+#include <cstring>
+#include <vector>
+
 #include "sched.h"
+#include "taskid.h"
+#include "tile_ops.cuh"
+
 namespace chol {
-struct SchedState { int workers; };
-int sched_create(SchedState** out, int64_t, int64_t, int, int, const chol_opts_t*, cudaStream_t) { *out = nullptr; return -8; }
-int sched_run(SchedState*, const CUtensorMap&, const StepParams&, cudaStream_t, int*) { return -8; }
-int sched_workers(const SchedState* st) { return st ? st->workers : 0; }
-void sched_destroy(SchedState* st) { delete st; }
+
+constexpr int kBuckets = 16;           // priority buckets per queue class
+constexpr int kQueues = 2 * kBuckets;  // [0, 16) normal, [16, 32) pinned
+constexpr int kQStride = 32;           // ints between queue heads (separate 128B lines)
+
+enum JobType : int16_t { J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4 };
+struct Job {
+  int16_t type, i, j, k, a, b, c, pad;
+};
+
+struct DevSched {
+  const Job* jobs;
+  const int* job_node;
+  int* node_deps;   // remaining predecessors
+  int* node_left;   // remaining jobs
+  const int* node_job_begin;
+  const int* node_job_count;
+  const int* succ_off;
+  const int* succ;
+  const int* node_paper;   // paper-level task id (taskid.h) for the trace
+  const int* node_queue;   // queue index
+  int* q_items;            // job id + 1 (0 = not yet written)
+  const int* q_base;       // start of each queue in q_items
+  int* q_head;             // kQueues * kQStride
+  int* q_tail;             // kQueues * kQStride
+  int* done_nodes;
+  int* finished;
+  int total_nodes;
+  int latency_workers;     // STATIC: CTAs [0, latency_workers) serve the pinned queues only
+  int policy;
+};
+
+// ------------------------------------------------------------------ device queue ops
+__device__ __forceinline__ int ld_volatile(const int* p) { return *reinterpret_cast<const volatile int*>(p); }
+
+__device__ __forceinline__ void push_node(const DevSched& d, int node) {
+  const int q = d.node_queue[node], cnt = d.node_job_count[node], jb = d.node_job_begin[node];
+  const int slot = atomicAdd(&d.q_tail[q * kQStride], cnt);
+  int* items = d.q_items + d.q_base[q] + slot;
+  for (int c = 0; c < cnt; ++c) items[c] = jb + c + 1;
+  __threadfence();
 }
+
+// Warp 0 pops one job (lane l inspects queue order[l]); returns job id or -1 if none.
+__device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, int lane) {
+  // queue inspected by this lane: highest priority = lowest lane
+  int q;
+  if (d.policy == 2 && latency_worker)
+    q = lane < kBuckets ? kBuckets + (kBuckets - 1 - lane) : -1;  // pinned only
+  else
+    q = lane < kBuckets ? (kBuckets - 1 - lane) : -1;             // normal only
+  for (int attempt = 0; attempt < 8; ++attempt) {
+    int h = 0;
+    bool avail = false;
+    if (q >= 0) {
+      h = ld_volatile(&d.q_head[q * kQStride]);
+      const int t = ld_volatile(&d.q_tail[q * kQStride]);
+      avail = h < t && ld_volatile(&d.q_items[d.q_base[q] + h]) != 0;
+    }
+    const unsigned m = __ballot_sync(0xffffffffu, avail);
+    if (!m) return -1;
+    const int src = __ffs(m) - 1;
+    int job = -1;
+    if (lane == src) {
+      if (atomicCAS(&d.q_head[q * kQStride], h, h + 1) == h) job = ld_volatile(&d.q_items[d.q_base[q] + h]) - 1;
+    }
+    job = __shfl_sync(0xffffffffu, job, src);
+    if (job >= 0) return job;
+  }
+  return -1;
+}
+
+template <int BS>
+__device__ __forceinline__ void run_job(Ctx<BS>& c, const Job& jb, int* info) {
+  switch (jb.type) {
+    case J_UPD: sub_update(c, jb.i, jb.j, jb.k, jb.a, jb.b); break;
+    case J_TRSM: sub_trsm(c, jb.i, jb.k, jb.a); break;
+    case J_DIAG: sub_potrf_diag(c, jb.k, jb.a, info); break;
+    case J_PANEL: sub_potrf_panel(c, jb.k, jb.a, jb.b); break;
+    case J_PUPD: sub_potrf_update(c, jb.k, jb.a, jb.b, jb.c); break;
+  }
+}
+
+template <int BS>
+__global__ void __launch_bounds__(kThreads, 1) k_sched(const __grid_constant__ CUtensorMap map, StepParams sp,
+                                                       DevSched d) {
+  __shared__ int s_job, s_skip;
+  __shared__ uint64_t s_t0;
+  auto c = make_ctx<BS>(&map, sp.tiles, sp.nb, sp.N);
+  const bool latency_worker = d.policy == 2 && (int)blockIdx.x < d.latency_workers;
+  const int tid = threadIdx.x;
+  while (true) {
+    if (c.warp == 0) {
+      int job = -1;
+      unsigned backoff = 32;
+      while (true) {
+        job = try_pop(d, latency_worker, c.lane);
+        if (job >= 0) break;
+        if (ld_volatile(d.finished)) break;
+        __nanosleep(backoff);
+        backoff = backoff < 1024 ? backoff * 2 : 1024;
+      }
+      if (c.lane == 0) {
+        __threadfence();  // acquire: the job's inputs were published before it was enqueued
+        s_job = job;
+        s_skip = ld_volatile(sp.info) != INT_MAX;
+        s_t0 = sp.tr_base ? globaltimer_ns() - *sp.tr_base : 0;
+      }
+    }
+    __syncthreads();
+    const int job = s_job;
+    if (job < 0) break;
+    const Job jb = d.jobs[job];
+    if (!s_skip) run_job(c, jb, sp.info);
+    __threadfence();      // this job's global writes are complete at L2 ...
+    fence_proxy_async();  // ... and ordered before later async-proxy (TMA) accesses
+    __syncthreads();
+    if (tid == 0) {
+      __threadfence();  // release this job's global writes
+      const int node = d.job_node[job];
+      if (sp.tr_t0) {
+        const uint64_t t_end = globaltimer_ns() - *sp.tr_base;
+        const int pt = d.node_paper[node];
+        atomicMin(reinterpret_cast<unsigned long long*>(sp.tr_t0 + pt), (unsigned long long)s_t0);
+        atomicMax(reinterpret_cast<unsigned long long*>(sp.tr_t1 + pt),
+                  (unsigned long long)((t_end << 16) | smid()));
+      }
+      if (atomicSub(&d.node_left[node], 1) == 1) {
+        __threadfence();
+        for (int e = d.succ_off[node]; e < d.succ_off[node + 1]; ++e) {
+          const int s = d.succ[e];
+          if (atomicSub(&d.node_deps[s], 1) == 1) push_node(d, s);
+        }
+        if (atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
+          __threadfence();
+          atomicExch(d.finished, 1);
+        }
+      }
+    }
+  }
+}
+
+__global__ void k_sched_init(DevSched d, const int* roots, int nroots) {
+  for (int r = 0; r < nroots; ++r) push_node(d, roots[r]);
+}
+
+// ------------------------------------------------------------------ host planner
+struct SchedState {
+  int64_t N = 0, nb = 0;
+  int bs = 0, workers = 0, nnodes = 0, njobs = 0, nroots = 0;
+  chol_opts_t opts{};
+  DevSched d{};
+  // device buffers
+  void* dev_static = nullptr;   // jobs, job_node, CSR, node tables (read-only)
+  void* dev_dynamic = nullptr;  // counters, queues (reset per run)
+  size_t dyn_bytes = 0;
+  void* dev_pristine = nullptr; // initial node_deps / node_left
+  size_t pristine_bytes = 0;
+  int* roots = nullptr;
+};
+
+namespace {
+
+struct Builder {
+  int64_t N;
+  int nbb, policy, pin_d;
+  std::vector<Job> jobs;
+  std::vector<int> job_node, deps, jbeg, jcnt, paper, ptype, pk, pi;
+  std::vector<std::vector<int>> succ;
+
+  int add_node(int paper_id, int type, int i, int k) {
+    const int id = (int)deps.size();
+    deps.push_back(0);
+    jbeg.push_back((int)jobs.size());
+    jcnt.push_back(0);
+    paper.push_back(paper_id);
+    ptype.push_back(type);
+    pi.push_back(i);
+    pk.push_back(k);
+    succ.emplace_back();
+    return id;
+  }
+  void add_job(int node, Job j) {
+    jobs.push_back(j);
+    job_node.push_back(node);
+    ++jcnt[node];
+  }
+  void edge(int a, int b) {
+    succ[a].push_back(b);
+    ++deps[b];
+  }
+};
+
+}  // namespace
+
+int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts,
+                 cudaStream_t s) {
+  auto* st = new SchedState();
+  st->N = N;
+  st->nb = nb;
+  st->bs = bs;
+  st->opts = *opts;
+  const int nbb = (int)(nb / bs);
+  Builder B{N, nbb, opts->policy, opts->trsm_pin_distance > 0 ? opts->trsm_pin_distance : (int)N};
+
+  // ---- nodes and jobs, Algorithm 1 order
+  std::vector<int> first_node(n_tasks(N)), last_node(n_tasks(N));
+  for (int k = 0; k < N; ++k) {
+    const int pid = (int)id_potrf(N, k);
+    int prev = -1;
+    for (int b = 0; b < nbb; ++b) {
+      const int dn = B.add_node(pid, T_POTRF, k, k);
+      B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+      if (prev >= 0) B.edge(prev, dn);
+      if (b == 0) first_node[pid] = dn;
+      prev = dn;
+      const int m = nbb - 1 - b;
+      if (m > 0) {
+        const int pn = B.add_node(pid, T_POTRF, k, k);
+        for (int r = b + 1; r < nbb; ++r)
+          B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
+        B.edge(prev, pn);
+        const int un = B.add_node(pid, T_POTRF, k, k);
+        for (int r = b + 1; r < nbb; ++r)
+          for (int q = b + 1; q <= r; ++q)
+            B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
+        B.edge(pn, un);
+        prev = un;
+      }
+    }
+    last_node[pid] = prev;
+    for (int i = k + 1; i < N; ++i) {
+      const int tid = (int)id_trsm(N, i, k);
+      const int n = B.add_node(tid, T_TRSM, i, k);
+      for (int sl = 0; sl < nbb; ++sl)
+        B.add_job(n, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
+      first_node[tid] = last_node[tid] = n;
+    }
+    for (int j = k + 1; j < N; ++j) {
+      const int sid = (int)id_syrk(N, j, k);
+      const int n = B.add_node(sid, T_SYRK, j, k);
+      for (int bm = 0; bm < nbb; ++bm)
+        for (int bn = 0; bn <= bm; ++bn)
+          B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
+      first_node[sid] = last_node[sid] = n;
+      for (int i = j + 1; i < N; ++i) {
+        const int gid = (int)id_gemm(N, i, j, k);
+        const int g = B.add_node(gid, T_GEMM, i, k);
+        for (int bm = 0; bm < nbb; ++bm)
+          for (int bn = 0; bn < nbb; ++bn)
+            B.add_job(g, Job{J_UPD, (int16_t)i, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
+        first_node[gid] = last_node[gid] = g;
+      }
+    }
+  }
+
+  // ---- task edges: direct data dependencies from tile read/write sets in program
+  // order (L213-220): each task depends on the last writer of every tile it touches.
+  {
+    std::vector<int> last_writer((size_t)N * (N + 1) / 2, -1);
+    auto touch = [&](int task, int64_t tile, std::vector<int>& preds) {
+      const int w = last_writer[tile];
+      if (w >= 0 && std::find(preds.begin(), preds.end(), w) == preds.end()) preds.push_back(w);
+    };
+    std::vector<int> preds;
+    auto visit = [&](int task, std::initializer_list<int64_t> reads, int64_t write) {
+      preds.clear();
+      for (int64_t t : reads) touch(task, t, preds);
+      touch(task, write, preds);
+      for (int p : preds) B.edge(last_node[p], first_node[task]);
+      last_writer[write] = task;
+    };
+    for (int k = 0; k < N; ++k) {
+      visit((int)id_potrf(N, k), {tile_index(k, k)}, tile_index(k, k));
+      for (int i = k + 1; i < N; ++i) visit((int)id_trsm(N, i, k), {tile_index(k, k), tile_index(i, k)}, tile_index(i, k));
+      for (int j = k + 1; j < N; ++j) {
+        visit((int)id_syrk(N, j, k), {tile_index(j, k), tile_index(j, j)}, tile_index(j, j));
+        for (int i = j + 1; i < N; ++i)
+          visit((int)id_gemm(N, i, j, k), {tile_index(i, k), tile_index(j, k), tile_index(i, j)}, tile_index(i, j));
+      }
+    }
+  }
+
+  // ---- priorities: bottom-level over the node DAG with per-type weights
+  // (latency estimates in microseconds; reading R13), quantised into kBuckets.
+  const int nnodes = (int)B.deps.size();
+  // POTRF is 3*nbb inner nodes: each gets a share of the POTRF latency
+  const double w_type[4] = {300.0 / (3.0 * nbb), 300.0, 80.0, 80.0};
+  std::vector<double> bl(nnodes, 0.0);
+  for (int v = nnodes - 1; v >= 0; --v) {  // node creation order is topological
+    double tail = 0.0;
+    for (int s2 : B.succ[v]) tail = std::max(tail, bl[s2]);
+    bl[v] = w_type[B.ptype[v]] + tail;
+  }
+  const double blmax = *std::max_element(bl.begin(), bl.end()) + 1e-9;
+  std::vector<int> node_queue(nnodes, 0);
+  for (int v = 0; v < nnodes; ++v) {
+    int bucket = 0;
+    if (opts->policy != CHOL_POLICY_DYNAMIC) bucket = std::min(kBuckets - 1, (int)(kBuckets * bl[v] / blmax));
+    bool pinned = false;
+    if (opts->policy == CHOL_POLICY_STATIC) {
+      if (B.ptype[v] == T_POTRF) pinned = true;
+      if (B.ptype[v] == T_TRSM && B.pi[v] - B.pk[v] <= B.pin_d) pinned = true;
+    }
+    node_queue[v] = bucket + (pinned ? kBuckets : 0);
+  }
+
+  // ---- queue capacities
+  std::vector<int> qcap(kQueues, 0), qbase(kQueues, 0);
+  for (int v = 0; v < nnodes; ++v) qcap[node_queue[v]] += B.jcnt[v];
+  for (int q = 1; q < kQueues; ++q) qbase[q] = qbase[q - 1] + qcap[q - 1];
+
+  std::vector<int> succ_off(nnodes + 1, 0), succ;
+  for (int v = 0; v < nnodes; ++v) {
+    succ_off[v + 1] = succ_off[v] + (int)B.succ[v].size();
+    succ.insert(succ.end(), B.succ[v].begin(), B.succ[v].end());
+  }
+  std::vector<int> roots;
+  for (int v = 0; v < nnodes; ++v)
+    if (B.deps[v] == 0) roots.push_back(v);
+
+  st->nnodes = nnodes;
+  st->njobs = (int)B.jobs.size();
+  st->nroots = (int)roots.size();
+
+  // ---- device layout: static (read-only) part
+  auto align = [](size_t x) { return (x + 255) & ~size_t(255); };
+  size_t off = 0;
+  const size_t o_jobs = off; off = align(off + B.jobs.size() * sizeof(Job));
+  const size_t o_jnode = off; off = align(off + B.job_node.size() * 4);
+  const size_t o_jbeg = off; off = align(off + nnodes * 4);
+  const size_t o_jcnt = off; off = align(off + nnodes * 4);
+  const size_t o_soff = off; off = align(off + (nnodes + 1) * 4);
+  const size_t o_succ = off; off = align(off + std::max<size_t>(succ.size(), 1) * 4);
+  const size_t o_paper = off; off = align(off + nnodes * 4);
+  const size_t o_nq = off; off = align(off + nnodes * 4);
+  const size_t o_qbase = off; off = align(off + kQueues * 4);
+  const size_t o_roots = off; off = align(off + std::max<size_t>(roots.size(), 1) * 4);
+  const size_t static_bytes = off;
+  std::vector<char> h(static_bytes, 0);
+  memcpy(h.data() + o_jobs, B.jobs.data(), B.jobs.size() * sizeof(Job));
+  memcpy(h.data() + o_jnode, B.job_node.data(), B.job_node.size() * 4);
+  memcpy(h.data() + o_jbeg, B.jbeg.data(), nnodes * 4);
+  memcpy(h.data() + o_jcnt, B.jcnt.data(), nnodes * 4);
+  memcpy(h.data() + o_soff, succ_off.data(), (nnodes + 1) * 4);
+  if (!succ.empty()) memcpy(h.data() + o_succ, succ.data(), succ.size() * 4);
+  memcpy(h.data() + o_paper, B.paper.data(), nnodes * 4);
+  memcpy(h.data() + o_nq, node_queue.data(), nnodes * 4);
+  memcpy(h.data() + o_qbase, qbase.data(), kQueues * 4);
+  if (!roots.empty()) memcpy(h.data() + o_roots, roots.data(), roots.size() * 4);
+
+  // dynamic part: node_deps, node_left, q_items, q_head, q_tail, done, finished
+  size_t doff = 0;
+  const size_t d_deps = doff; doff = align(doff + nnodes * 4);
+  const size_t d_left = doff; doff = align(doff + nnodes * 4);
+  const size_t pristine = doff;  // [0, pristine) is restored from the pristine copy
+  const size_t d_items = doff; doff = align(doff + (size_t)st->njobs * 4);
+  const size_t d_head = doff; doff = align(doff + kQueues * kQStride * 4);
+  const size_t d_tail = doff; doff = align(doff + kQueues * kQStride * 4);
+  const size_t d_done = doff; doff = align(doff + 4);
+  const size_t d_fin = doff; doff = align(doff + 4);
+  std::vector<char> hp(pristine, 0);
+  memcpy(hp.data() + d_deps, B.deps.data(), nnodes * 4);
+  memcpy(hp.data() + d_left, B.jcnt.data(), nnodes * 4);
+
+  cudaError_t e;
+  if ((e = cudaMalloc(&st->dev_static, static_bytes)) || (e = cudaMalloc(&st->dev_dynamic, doff)) ||
+      (e = cudaMalloc(&st->dev_pristine, pristine))) {
+    cudaGetLastError();
+    sched_destroy(st);
+    return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
+  }
+  if ((e = cudaMemcpy(st->dev_static, h.data(), static_bytes, cudaMemcpyHostToDevice)) ||
+      (e = cudaMemcpy(st->dev_pristine, hp.data(), pristine, cudaMemcpyHostToDevice))) {
+    sched_destroy(st);
+    return -100 - (int)e;
+  }
+  st->dyn_bytes = doff;
+  st->pristine_bytes = pristine;
+  char* S = static_cast<char*>(st->dev_static);
+  char* D = static_cast<char*>(st->dev_dynamic);
+  DevSched& d = st->d;
+  d.jobs = reinterpret_cast<const Job*>(S + o_jobs);
+  d.job_node = reinterpret_cast<const int*>(S + o_jnode);
+  d.node_job_begin = reinterpret_cast<const int*>(S + o_jbeg);
+  d.node_job_count = reinterpret_cast<const int*>(S + o_jcnt);
+  d.succ_off = reinterpret_cast<const int*>(S + o_soff);
+  d.succ = reinterpret_cast<const int*>(S + o_succ);
+  d.node_paper = reinterpret_cast<const int*>(S + o_paper);
+  d.node_queue = reinterpret_cast<const int*>(S + o_nq);
+  d.q_base = reinterpret_cast<const int*>(S + o_qbase);
+  st->roots = reinterpret_cast<int*>(S + o_roots);
+  d.node_deps = reinterpret_cast<int*>(D + d_deps);
+  d.node_left = reinterpret_cast<int*>(D + d_left);
+  d.q_items = reinterpret_cast<int*>(D + d_items);
+  d.q_head = reinterpret_cast<int*>(D + d_head);
+  d.q_tail = reinterpret_cast<int*>(D + d_tail);
+  d.done_nodes = reinterpret_cast<int*>(D + d_done);
+  d.finished = reinterpret_cast<int*>(D + d_fin);
+  d.total_nodes = nnodes;
+  d.policy = opts->policy;
+  d.latency_workers = opts->policy == CHOL_POLICY_STATIC ? (opts->latency_workers > 0 ? opts->latency_workers : 8) : 0;
+
+  // ---- workers: one CTA per SM (all co-resident)
+  int per_sm = 0;
+  const int smem = smem_bytes(bs);
+  cudaError_t ea = cudaSuccess;
+  switch (bs) {
+    case 96: ea = cudaFuncSetAttribute(k_sched<96>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<96>, kThreads, smem); break;
+    case 64: ea = cudaFuncSetAttribute(k_sched<64>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<64>, kThreads, smem); break;
+    case 32: ea = cudaFuncSetAttribute(k_sched<32>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<32>, kThreads, smem); break;
+  }
+  if (ea || per_sm < 1) {
+    sched_destroy(st);
+    return ea ? -100 - (int)ea : -8;
+  }
+  st->workers = opts->workers > 0 ? std::min(opts->workers, sms * per_sm) : sms;
+  if (d.latency_workers >= st->workers) d.latency_workers = std::max(1, st->workers / 4);
+  (void)s;
+  *out = st;
+  return 0;
+}
+
+int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch) {
+  cudaError_t e;
+  if ((e = cudaMemcpyAsync(st->dev_dynamic, st->dev_pristine, st->pristine_bytes, cudaMemcpyDeviceToDevice, s)))
+    return -100 - (int)e;
+  if ((e = cudaMemsetAsync(static_cast<char*>(st->dev_dynamic) + st->pristine_bytes, 0,
+                           st->dyn_bytes - st->pristine_bytes, s)))
+    return -100 - (int)e;
+  k_sched_init<<<1, 1, 0, s>>>(st->d, st->roots, st->nroots);
+  const int smem = smem_bytes(st->bs);
+  switch (st->bs) {
+    case 96: k_sched<96><<<st->workers, kThreads, smem, s>>>(map, base, st->d); break;
+    case 64: k_sched<64><<<st->workers, kThreads, smem, s>>>(map, base, st->d); break;
+    case 32: k_sched<32><<<st->workers, kThreads, smem, s>>>(map, base, st->d); break;
+  }
+  *nlaunch += 2;
+  if ((e = cudaGetLastError())) return -100 - (int)e;
+  return 0;
+}
+
+int sched_workers(const SchedState* st) { return st ? st->workers : 0; }
+
+void sched_destroy(SchedState* st) {
+  if (!st) return;
+  cudaFree(st->dev_static);
+  cudaFree(st->dev_dynamic);
+  cudaFree(st->dev_pristine);
+  delete st;
+}
+
+}  // namespace chol

@@ -103,6 +103,7 @@ __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, in
   const int nst = (kend - kbeg) / BK;
   if (c.producer()) {
     if (c.lane == 0) {
+      fence_proxy_async();  // operands may have been written by generic stores (this or other SMs)
       for (int s = 0; s < nst; ++s) {
         const uint32_t q = c.it + s, st = q % kStages, ph = (q / kStages) & 1;
         mbar_wait(&c.empty[st], ph ^ 1);
@@ -118,11 +119,15 @@ __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, in
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
     const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+    // threadIdx.y is 0 (1-D blocks) but unknown to the compiler: used to make the
+    // stage release depend on every shared load of the stage (see below).
+    const uint32_t rt_zero = threadIdx.y;
     for (int s = 0; s < nst; ++s) {
       const uint32_t q = c.it + s, st = q % kStages, ph = (q / kStages) & 1;
       mbar_wait(&c.full[st], ph);
       const uint32_t As = smem_u32(c.pipe) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
       const uint32_t Bs = smem_u32(c.pipe) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
+      uint32_t dep = 0;
 #pragma unroll
       for (int h = 0; h < 2; ++h) {
         // 128B swizzle: 16-byte chunk index ^= (row & 7); rows here are 8-aligned + g.
@@ -132,6 +137,10 @@ __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, in
         for (int mi = 0; mi < C::MI; ++mi) af[mi] = lds128(As + mi * 8 * 128 + chunk);
 #pragma unroll
         for (int ni = 0; ni < C::NI; ++ni) bf[ni] = lds128(Bs + ni * 8 * 128 + chunk);
+#pragma unroll
+        for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(af[mi].x);
+#pragma unroll
+        for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(bf[ni].x);
         // k-permutation: thread t holds k = 8h+2t (x) and 8h+2t+1 (y) for both operands.
 #pragma unroll
         for (int mi = 0; mi < C::MI; ++mi)
@@ -142,8 +151,12 @@ __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, in
 #pragma unroll
           for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].y, bf[ni].y);
       }
+      // Hand the stage back to the producer only once every ld.shared of it has
+      // returned: the arrive is predicated on a value derived from all loaded
+      // registers (lane 0 arrives), so it cannot issue before the loads complete
+      // and a TMA refill can never overwrite data a lane has not read yet.
       __syncwarp();
-      if (c.lane == 0) mbar_arrive(&c.empty[st]);
+      if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty[st]);
     }
   }
   c.it += nst;
@@ -162,14 +175,14 @@ __device__ __forceinline__ void epi_sub_global(const Ctx<BS>& c, const Acc<BS>& 
     for (int ni = 0; ni < C::NI; ++ni) {
       const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
       double2* p = reinterpret_cast<double2*>(Cblk + (int64_t)r * ldc + cc);
-      double2 v = *p;
+      double2 v = __ldcg(p);
       v.x -= acc[mi][ni][0];
       v.y -= acc[mi][ni][1];
       if (!lower_only) {
-        *p = v;
+        __stcg(p, v);
       } else {
-        if (cc <= r) p->x = v.x;
-        if (cc + 1 <= r) p->y = v.y;
+        if (cc <= r) __stcg(&p->x, v.x);
+        if (cc + 1 <= r) __stcg(&p->y, v.y);
       }
     }
 }
@@ -196,7 +209,7 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) {
         const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
-        double2 v = *reinterpret_cast<const double2*>(X + (int64_t)r * ldx + cc);
+        double2 v = __ldcg(reinterpret_cast<const double2*>(X + (int64_t)r * ldx + cc));
         if (has_acc) {
           v.x -= acc[mi][ni][0];
           v.y -= acc[mi][ni][1];
@@ -205,7 +218,7 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc
       }
     for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
       const int r = idx / BS, cc = idx - r * BS;
-      if (cc <= r) c.lbuf[cc * C::kPitch + r] = Ld[(int64_t)r * ldl + cc];
+      if (cc <= r) c.lbuf[cc * C::kPitch + r] = __ldcg(Ld + (int64_t)r * ldl + cc);
     }
   }
   bar_sync(kBarCompute, kComputeThreads);
@@ -239,7 +252,7 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc
 #pragma unroll
   for (int q = 0; q < C::RW; ++q)
 #pragma unroll
-    for (int s = 0; s < C::CPL; ++s) X[(int64_t)(r0 + q) * ldx + s * 32 + lane] = x[q][s];
+    for (int s = 0; s < C::CPL; ++s) __stcg(X + (int64_t)(r0 + q) * ldx + s * 32 + lane, x[q][s]);
   bar_sync(kBarCompute, kComputeThreads);
 }
 
@@ -255,7 +268,7 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
   bar_sync(kBarCompute, kComputeThreads);  // buf aliases the TMA ring
   for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
     const int r = idx / BS, cc = idx - r * BS;
-    if (cc <= r) a[r * C::kPitch + cc] = A[(int64_t)r * lda + cc];
+    if (cc <= r) a[r * C::kPitch + cc] = __ldcg(A + (int64_t)r * lda + cc);
   }
   bar_sync(kBarCompute, kComputeThreads);
   for (int j = 0; j < BS; ++j) {
@@ -280,7 +293,7 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
   }
   for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
     const int r = idx / BS, cc = idx - r * BS;
-    if (cc <= r) A[(int64_t)r * lda + cc] = a[r * C::kPitch + cc];
+    if (cc <= r) __stcg(A + (int64_t)r * lda + cc, a[r * C::kPitch + cc]);
   }
 }
 
@@ -310,7 +323,10 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
     if (cb > 0) gemm_mainloop(c, tile_index(i, k), slab * BS, tile_index(k, k), cb * BS, 0, cb * BS, acc);
     if (!c.producer()) {
       solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
-      fence_proxy_async();  // X[:, cb] (generic stores) is read by TMA in the next block; buf is re-filled by TMA
+      // X[:, cb] (generic stores) is read by TMA in the next block: complete the stores
+      // at L2 (gpu-scope fence), then order them before async-proxy accesses.
+      __threadfence();
+      fence_proxy_async();
     }
     bar_sync(kBarAll, kThreads);
   }
