@@ -1,0 +1,324 @@
+#!/usr/bin/env python
+"""Benchmark of the tiled FP64 Cholesky hot path (BASELINE.json metric:
+"Cholesky FP64 TFLOP/s (n^3/3 / t) at 1/2/4/8 B200; % of FP64 peak").
+
+One step = one factorization A = L L^T of a seeded synthetic SPD matrix through the
+C-ABI (chol_factor_inplace: every Algorithm 1 task -- POTRF, TRSM, SYRK, GEMM -- run by
+the device-side scheduler kernel).  Default workload = BASELINE.json configs[1]:
+n = 19200 as 20 x 20 tiles of nb = 960 on 1 B200.
+
+Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+       [--n 19200] [--nb 960] [--policy cp|dynamic|static] [--executor sched|host]
+Under torchrun (N > 1) each rank factors its own matrix (replicas, see DESIGN.md
+"Multi-GPU"); rank 0 prints ONE JSON line.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import tempfile
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "Cholesky FP64 TFLOP/s (n^3/3 / t)"
+FP64_PEAK_TFLOPS = 37.1  # measured DMMA peak, profiles/r01/fp64_peak_microbench.jsonl
+POLICIES = {"dynamic": 0, "cp": 1, "static": 2}
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=5)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--n", type=int, default=19200)
+    ap.add_argument("--nb", type=int, default=960)
+    ap.add_argument("--policy", choices=list(POLICIES), default="cp")
+    ap.add_argument("--executor", choices=["sched", "host"], default="sched")
+    ap.add_argument("--seed", type=int, default=0)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-bounds", action="store_true")
+    ap.add_argument("--cpu-sample-n", type=int, default=7680)
+    return ap.parse_args()
+
+
+# ----------------------------------------------------------------------------- helpers
+class ClockSampler:
+    """nvidia-smi clocks / throttle reasons sampled every 200 ms during the timed region."""
+
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, device: int):
+        self.device = device
+        self.proc = None
+        self.path = None
+
+    def __enter__(self):
+        fd, self.path = tempfile.mkstemp(suffix=".csv")
+        os.close(fd)
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.device), f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                 "-lms", "200"], stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+        except FileNotFoundError:
+            self.proc = None
+        time.sleep(0.3)
+        return self
+
+    def __exit__(self, *a):
+        if self.proc:
+            self.proc.terminate()
+            self.proc.wait()
+
+    def summary(self):
+        rows = []
+        if self.path and os.path.exists(self.path):
+            for ln in open(self.path):
+                parts = [x.strip() for x in ln.split(",")]
+                if len(parts) >= 9:
+                    rows.append(parts)
+            os.unlink(self.path)
+        if not rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+
+        def num(x):
+            try:
+                return float(x)
+            except ValueError:
+                return None
+
+        sm = [num(r[1]) for r in rows if num(r[1])]
+        mx = [num(r[2]) for r in rows if num(r[2])]
+        power = [num(r[3]) for r in rows if num(r[3])]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[i] for r in rows for i in range(4) if r[5 + i].lower().startswith("active")})
+        loaded = [s for s in sm if s and s > 500] or sm
+        return {"sm_mhz": statistics.median(loaded) if loaded else None, "sm_max_mhz": max(mx) if mx else None,
+                "power_w_max": max(power) if power else None, "samples": len(rows), "reasons": reasons}
+
+
+def dist_setup():
+    ws = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if ws > 1:
+        import torch
+        import torch.distributed as dist
+        torch.cuda.set_device(local)
+        dist.init_process_group("nccl")
+    return ws, rank, local
+
+
+def barrier(ws):
+    if ws > 1:
+        import torch.distributed as dist
+        dist.barrier()
+
+
+def allmax(ws, x: float) -> float:
+    if ws == 1:
+        return x
+    import torch
+    import torch.distributed as dist
+    t = torch.tensor([x], dtype=torch.float64, device="cuda")
+    dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    return float(t.item())
+
+
+# ----------------------------------------------------------------------------- reference arm
+def run_reference(args, ws, rank):
+    """The oracle (oracle/chol_oracle.c, plain C + OpenMP, no BLAS) as it stands, on the
+    host cores, on a bounded sample of the workload (same nb, fewer tiles)."""
+    if rank != 0:
+        return
+    import oracle
+    import spdgen
+    n_s = min(args.n, 3840)
+    A = spdgen.uniform_spd(n_s, args.seed)
+    times = []
+    for it in range(args.warmup + args.steps):
+        t0 = time.perf_counter()
+        L, info = oracle.chol_tiled(A, args.nb)
+        dt = time.perf_counter() - t0
+        assert info == 0
+        if it >= args.warmup:
+            times.append(dt)
+    tot = sum(times)
+    value = n_s ** 3 / 3.0 / (tot / len(times)) / 1e12
+    cores = oracle.num_threads()
+    sample = f"uniform SPD n={n_s} ({n_s // args.nb}x{n_s // args.nb} tiles of nb={args.nb}) per step"
+    line = {
+        "impl": "reference", "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": args.gpus,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * tot / len(times),
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": {"workload": f"FP64 SPD n={args.n} nb={args.nb} (bounded sample: {sample})", "n": args.n,
+                   "nb": args.nb},
+        "cpu_baseline": {"value": value, "unit": "TFLOP/s", "cores": cores, "kind": "oracle", "sample": sample},
+        "e2e": {"value": value, "unit": "TFLOP/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+
+
+# ----------------------------------------------------------------------------- our arm
+def cpu_baseline(args):
+    import oracle
+    import spdgen
+    n_s = min(args.cpu_sample_n, args.n)
+    n_s -= n_s % args.nb
+    A = spdgen.uniform_spd(n_s, args.seed)
+    t0 = time.perf_counter()
+    L, info = oracle.chol_tiled(A, args.nb)
+    dt = time.perf_counter() - t0
+    return {"value": n_s ** 3 / 3.0 / dt / 1e12, "unit": "TFLOP/s", "cores": oracle.num_threads(),
+            "kind": "oracle",
+            "sample": f"one factorization of a uniform SPD n={n_s} ({n_s // args.nb}x{n_s // args.nb} tiles of "
+                      f"nb={args.nb}), {dt:.1f} s"}
+
+
+def calibrate(c, args):
+    """T_lat (task alone on the GPU) and T_thr (per task in a saturating batch), seconds."""
+    n, nb = args.n, args.nb
+    N = n // nb
+    T_lat, T_thr = [], []
+    with c.Plan(3 * nb, nb, executor=c.EXEC_HOST) as p:
+        c.chol_generate(p.h, 1, 0)
+        for t in range(4):
+            c.chol_run_task(p.h, t, 2, 1, 0 if t else 1, 1)
+            T_lat.append(c.chol_run_task(p.h, t, 2, 1, 0 if t else 1, 5) * 1e-3)
+    with c.Plan(n, nb, executor=c.EXEC_HOST) as p:
+        c.chol_generate(p.h, 1, 0)
+        counts = [N, N - 1, N - 1, (N - 1) * (N - 2) // 2]
+        for t in range(4):
+            cnt = max(1, counts[t])
+            c.chol_run_batch(p.h, t, cnt, 1)
+            T_thr.append(c.chol_run_batch(p.h, t, cnt, 2) * 1e-3)
+    return T_lat, T_thr
+
+
+def run_ours(args, ws, rank, local):
+    import torch
+    import paper_conf_ipps_agullobehkmt15_b200 as c
+
+    n, nb = args.n, args.nb
+    flops = n ** 3 / 3.0
+    ex = c.EXEC_SCHEDULER if args.executor == "sched" else c.EXEC_HOST
+    pol = POLICIES[args.policy]
+    plan = c.Plan(n, nb, executor=ex, policy=pol)
+    info_d = c.chol_get_info(plan.h)
+
+    for _ in range(args.warmup):
+        c.chol_generate(plan.h, args.seed, 0)
+        info = c.chol_factor_inplace(plan.h)
+        assert info == 0, info
+    torch.cuda.synchronize()
+
+    times, launches = [], 0
+    with ClockSampler(local) as clk:
+        for _ in range(args.steps):
+            c.chol_generate(plan.h, args.seed, 0)  # fresh input, resident in HBM, untimed
+            barrier(ws)
+            torch.cuda.synchronize()
+            info = c.chol_factor_inplace(plan.h)  # CUDA events on the plan's stream
+            torch.cuda.synchronize()
+            assert info == 0, info
+            times.append(c.chol_last_times(plan.h)[0])
+            launches += c.chol_last_launches(plan.h)
+    clocks = clk.summary()
+    total = allmax(ws, sum(times))
+    t_step = total / args.steps
+    value = ws * flops / t_step / 1e12
+
+    # roofline: the dominant (and only long) kernel is the persistent scheduler kernel
+    achieved = flops / (sum(times) / len(times)) / 1e12
+    traffic = None
+    prof = os.path.join(ROOT, "profiles", "r01", "ncu_summary.json")
+    if os.path.exists(prof):
+        try:
+            traffic = json.load(open(prof)).get("sched_kernel_dram_bytes_per_launch")
+        except Exception:
+            traffic = None
+    roofline = {"bound": "tensor", "achieved": achieved, "peak": FP64_PEAK_TFLOPS, "unit": "TFLOP/s",
+                "frac": achieved / FP64_PEAK_TFLOPS, "traffic": traffic,
+                "kernel": "k_sched (persistent scheduler: all POTRF/TRSM/SYRK/GEMM sub-tasks)",
+                "peak_source": "measured FP64 DMMA microbenchmark (MEASURED_PEAKS.json has no FP64 entry)"}
+
+    line = {
+        "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": ws, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": 1e3 * t_step, "higher_is_better": True,
+        "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": {"workload": f"FP64 SPD n={n} as {n // nb}x{n // nb} tiles of nb={nb} (BASELINE configs[1])",
+                   "n": n, "nb": nb, "block": info_d["block"], "executor": args.executor,
+                   "policy": args.policy, "workers": info_d["workers"],
+                   "parallelism": "1 GPU" if ws == 1 else f"{ws} replicas (one factorization per GPU)",
+                   "input": "uniform family seed %d, regenerated on device before each step (untimed)" % args.seed,
+                   "l2": "inputs 1.47 GB >> 126 MB L2 and rewritten between steps",
+                   "timing": "CUDA events on the plan stream around each factorization, max over ranks"},
+        "pct_fp64_peak": 100.0 * achieved / FP64_PEAK_TFLOPS,
+        "roofline": roofline,
+        "clocks": clocks,
+        "gpu_launches": launches,
+    }
+
+    # end-to-end: the C-ABI with HOST buffers (pinned), copies inside the timed region
+    if not args.no_e2e:
+        A_h = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
+        L_h = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
+        c.chol_generate(plan.h, args.seed, 0)
+        c.chol_gather(plan.h, A_h, n)  # the same matrix, lower triangle (upper zero)
+        e2e_t = []
+        for it in range(3):
+            barrier(ws)
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            info = c.chol_factor(plan.h, A_h, n, L_h, n)
+            dt = time.perf_counter() - t0
+            assert info == 0
+            if it > 0:
+                e2e_t.append(dt)
+        t_e2e = allmax(ws, statistics.mean(e2e_t))
+        tile_bytes = (n // nb) * (n // nb + 1) // 2 * nb * nb * 8
+        line["e2e"] = {"value": ws * flops / t_e2e / 1e12, "unit": "TFLOP/s", "h2d_bytes_per_step": tile_bytes,
+                       "d2h_bytes_per_step": tile_bytes, "ms_per_step": 1e3 * t_e2e,
+                       "layout_ms": 1e3 * c.chol_last_times(plan.h)[1]}
+        del A_h, L_h
+    plan.close()
+
+    if not args.no_bounds and rank == 0:
+        T_lat, T_thr = calibrate(c, args)
+        b = c.chol_bounds(n, nb, 1, T_lat, T_thr)
+        line["bounds"] = {
+            "T_lat_s": dict(zip(c.TYPE_NAMES, T_lat)), "T_thr_s": dict(zip(c.TYPE_NAMES, T_thr)),
+            "seconds": b, "upper_tflops": {k: (flops / v / 1e12 if v and v > 0 else None) for k, v in b.items()},
+            "makespan_over_mixed": t_step / b["mixed"],
+        }
+
+    if rank == 0 and ws == 1 and not args.no_cpu_baseline:
+        line["cpu_baseline"] = cpu_baseline(args)
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+
+
+def main():
+    args = parse()
+    ws, rank, local = dist_setup()
+    if args.impl == "reference":
+        run_reference(args, ws, rank)
+    else:
+        run_ours(args, ws, rank, local)
+    if ws > 1:
+        import torch.distributed as dist
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -148,6 +148,30 @@ int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double
  * (throughput time T_t^thr, reading R9).  Overwrites the store. */
 int chol_run_batch(chol_plan_t p, int type, int count, int reps, double* ms);
 
+/* Number of kernel launches the last chol_factor* issued (the persistent scheduler
+ * issues 2: queue init + the scheduler kernel). */
+int chol_last_launches(chol_plan_t p, int* launches);
+
+/* ---- host-only (no GPU needed) ---- */
+
+/* Task graph of Algorithm 1 for N tiles per side (Fig. 1):
+ * *ntasks = N + N(N-1) + N(N-1)(N-2)/6; *nedges = number of direct data
+ * dependencies (L213-220); edges[2e], edges[2e+1] = (pred, succ) dense task ids
+ * (chol_task_id), at most cap edges written (edges may be NULL). */
+int chol_dag(int64_t N, int64_t* ntasks, int64_t* nedges, int64_t* edges, int64_t cap);
+
+/* Dense id of task (type, i, j, k) in chol_dag / chol_trace numbering. */
+int chol_task_id(int64_t N, int type, int i, int j, int k, int64_t* id);
+
+/* Makespan lower bounds of PAPER.md §III (L334-408, L495-502) for one resource type
+ * (ngpus GPUs), from per-type latency times T_lat[4] (a task alone on an idle GPU)
+ * and throughput times T_thr[4] (per task in a saturating batch), indexed
+ * POTRF, TRSM, SYRK, GEMM, in seconds.  out[0] area = sum_t N_t T_thr_t / M,
+ * out[1] chain = N T_lat_P + (N-1)(T_lat_T + T_lat_S), out[2] mixed = max(area,
+ * chain), out[3] critical path (longest DAG path, T_lat weights; -1 if N > 256),
+ * out[4] GEMM-peak bound (n^3/3) / (M 2 nb^3 / T_thr_G), out[5] max(area, cp). */
+int chol_bounds(int64_t n, int64_t nb, int ngpus, const double* T_lat, const double* T_thr, double* out);
+
 #ifdef __cplusplus
 }
 #endif

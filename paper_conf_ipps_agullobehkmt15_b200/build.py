@@ -8,8 +8,8 @@ import sys
 HERE = os.path.dirname(os.path.abspath(__file__))
 CSRC = os.path.join(HERE, "csrc")
 LIB = os.path.join(HERE, "libchol_b200.so")
-SOURCES = ["api.cu", "kernels.cu", "sched.cu"]
-HEADERS = ["dev_common.cuh", "tile_ops.cuh", "kernels.h", "sched.h", "taskid.h", "sched_dev.cuh"]
+SOURCES = ["api.cu", "kernels.cu", "sched.cu", "dag.cpp"]
+HEADERS = ["dev_common.cuh", "tile_ops.cuh", "kernels.h", "sched.h", "taskid.h", "dag.h"]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 FLAGS = ["-O3", "-std=c++17", "-gencode", "arch=compute_100a,code=sm_100a", "-lineinfo",
          "-Xcompiler", "-fPIC", "-Xcompiler", "-O2", "--expt-relaxed-constexpr"]
@@ -29,7 +29,7 @@ def build(force: bool = False, verbose: bool = False) -> str:
         return LIB
     objs = []
     for s in SOURCES:
-        o = os.path.join(CSRC, s.replace(".cu", ".o"))
+        o = os.path.join(CSRC, os.path.splitext(s)[0] + ".o")
         cmd = [NVCC, *FLAGS, "-c", os.path.join(CSRC, s), "-o", o]
         if verbose:
             cmd.insert(1, "-Xptxas=-v")

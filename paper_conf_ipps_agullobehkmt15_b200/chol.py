@@ -60,6 +60,10 @@ def _load():
                            ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(i32)], i32),
         "chol_run_task": ([P, i32, i32, i32, i32, i32, dp], i32),
         "chol_run_batch": ([P, i32, i32, i32, dp], i32),
+        "chol_last_launches": ([P, ctypes.POINTER(i32)], i32),
+        "chol_dag": ([i64, ctypes.POINTER(i64), ctypes.POINTER(i64), ctypes.POINTER(i64), i64], i32),
+        "chol_task_id": ([i64, i32, i32, i32, i32, ctypes.POINTER(i64)], i32),
+        "chol_bounds": ([i64, i64, i32, dp, dp, dp], i32),
     }
     for name, (args, res) in sig.items():
         f = getattr(L, name)
@@ -71,7 +75,8 @@ def _load():
 _lib = _load()
 EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_destroy", "chol_strerror",
             "chol_generate", "chol_scatter", "chol_gather", "chol_factor_inplace", "chol_last_times",
-            "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch")
+            "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
+            "chol_dag", "chol_task_id", "chol_bounds")
 
 
 def _ptr(x) -> int:
@@ -178,6 +183,39 @@ def chol_run_batch(plan: int, type: int, count: int, reps: int = 1) -> float:
     ms = ctypes.c_double()
     _check(_lib.chol_run_batch(plan, type, count, reps, ctypes.byref(ms)), "chol_run_batch")
     return ms.value
+
+
+def chol_last_launches(plan: int) -> int:
+    n = ctypes.c_int()
+    _check(_lib.chol_last_launches(plan, ctypes.byref(n)), "chol_last_launches")
+    return n.value
+
+
+def chol_dag(N: int):
+    """(ntasks, edges as a list of (pred, succ) dense task ids)."""
+    nt, ne = ctypes.c_int64(), ctypes.c_int64()
+    _check(_lib.chol_dag(N, ctypes.byref(nt), ctypes.byref(ne), None, 0), "chol_dag")
+    buf = (ctypes.c_int64 * max(2 * ne.value, 1))()
+    _check(_lib.chol_dag(N, ctypes.byref(nt), ctypes.byref(ne), buf, ne.value), "chol_dag")
+    return nt.value, [(buf[2 * e], buf[2 * e + 1]) for e in range(ne.value)]
+
+
+def chol_task_id(N: int, type: int, i: int, j: int, k: int) -> int:
+    v = ctypes.c_int64()
+    _check(_lib.chol_task_id(N, type, i, j, k, ctypes.byref(v)), "chol_task_id")
+    return v.value
+
+
+BOUND_NAMES = ("area", "chain", "mixed", "critical_path", "gemm_peak", "max_area_cp")
+
+
+def chol_bounds(n: int, nb: int, ngpus: int, T_lat, T_thr) -> dict:
+    """Makespan lower bounds (seconds) from per-type times [POTRF, TRSM, SYRK, GEMM]."""
+    lat = (ctypes.c_double * 4)(*T_lat)
+    thr = (ctypes.c_double * 4)(*T_thr)
+    out = (ctypes.c_double * 6)()
+    _check(_lib.chol_bounds(n, nb, ngpus, lat, thr, out), "chol_bounds")
+    return dict(zip(BOUND_NAMES, list(out)))
 
 
 class Plan:

@@ -368,6 +368,12 @@ extern "C" int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* 
   return 0;
 }
 
+extern "C" int chol_last_launches(chol_plan_t p, int* launches) {
+  if (!p || !launches) return -4;
+  *launches = p->last_launches;
+  return 0;
+}
+
 extern "C" int chol_last_times(chol_plan_t p, double* factor_s, double* layout_s) {
   if (!p) return -4;
   if (factor_s) *factor_s = p->last_factor_s;

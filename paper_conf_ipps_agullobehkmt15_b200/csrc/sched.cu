@@ -20,6 +20,7 @@
 #include <cstring>
 #include <vector>
 
+#include "dag.h"
 #include "sched.h"
 #include "taskid.h"
 #include "tile_ops.cuh"
@@ -281,49 +282,25 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     }
   }
 
-  // ---- task edges: direct data dependencies from tile read/write sets in program
-  // order (L213-220): each task depends on the last writer of every tile it touches.
-  {
-    std::vector<int> last_writer((size_t)N * (N + 1) / 2, -1);
-    auto touch = [&](int task, int64_t tile, std::vector<int>& preds) {
-      const int w = last_writer[tile];
-      if (w >= 0 && std::find(preds.begin(), preds.end(), w) == preds.end()) preds.push_back(w);
-    };
-    std::vector<int> preds;
-    auto visit = [&](int task, std::initializer_list<int64_t> reads, int64_t write) {
-      preds.clear();
-      for (int64_t t : reads) touch(task, t, preds);
-      touch(task, write, preds);
-      for (int p : preds) B.edge(last_node[p], first_node[task]);
-      last_writer[write] = task;
-    };
-    for (int k = 0; k < N; ++k) {
-      visit((int)id_potrf(N, k), {tile_index(k, k)}, tile_index(k, k));
-      for (int i = k + 1; i < N; ++i) visit((int)id_trsm(N, i, k), {tile_index(k, k), tile_index(i, k)}, tile_index(i, k));
-      for (int j = k + 1; j < N; ++j) {
-        visit((int)id_syrk(N, j, k), {tile_index(j, k), tile_index(j, j)}, tile_index(j, j));
-        for (int i = j + 1; i < N; ++i)
-          visit((int)id_gemm(N, i, j, k), {tile_index(i, k), tile_index(j, k), tile_index(i, j)}, tile_index(i, j));
-      }
-    }
-  }
+  // ---- task edges: direct data dependencies of Algorithm 1 (dag.cpp, L213-220),
+  // mapped onto the nodes (POTRF_k enters at its first inner node, leaves at its last).
+  std::vector<std::pair<int64_t, int64_t>> E;
+  std::vector<int> type_of;
+  build_task_dag(N, E, type_of);
+  for (auto& e : E) B.edge(last_node[e.first], first_node[e.second]);
 
-  // ---- priorities: bottom-level over the node DAG with per-type weights
-  // (latency estimates in microseconds; reading R13), quantised into kBuckets.
+  // ---- priorities: bottom-level of each Algorithm 1 task (HEFT / dmdas, L299-301,
+  // L655-660; reading R13) with latency-estimate weights, quantised into kBuckets;
+  // POTRF's inner nodes inherit the POTRF priority.
   const int nnodes = (int)B.deps.size();
-  // POTRF is 3*nbb inner nodes: each gets a share of the POTRF latency
-  const double w_type[4] = {300.0 / (3.0 * nbb), 300.0, 80.0, 80.0};
-  std::vector<double> bl(nnodes, 0.0);
-  for (int v = nnodes - 1; v >= 0; --v) {  // node creation order is topological
-    double tail = 0.0;
-    for (int s2 : B.succ[v]) tail = std::max(tail, bl[s2]);
-    bl[v] = w_type[B.ptype[v]] + tail;
-  }
+  const double w_type[4] = {300.0, 300.0, 80.0, 80.0};
+  const std::vector<double> bl = bottom_levels(N, w_type);
   const double blmax = *std::max_element(bl.begin(), bl.end()) + 1e-9;
   std::vector<int> node_queue(nnodes, 0);
   for (int v = 0; v < nnodes; ++v) {
     int bucket = 0;
-    if (opts->policy != CHOL_POLICY_DYNAMIC) bucket = std::min(kBuckets - 1, (int)(kBuckets * bl[v] / blmax));
+    if (opts->policy != CHOL_POLICY_DYNAMIC)
+      bucket = std::min(kBuckets - 1, (int)(kBuckets * bl[B.paper[v]] / blmax));
     bool pinned = false;
     if (opts->policy == CHOL_POLICY_STATIC) {
       if (B.ptype[v] == T_POTRF) pinned = true;

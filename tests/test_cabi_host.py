@@ -1,0 +1,72 @@
+"""CPU-only checks of the C-ABI library: it builds, loads without a GPU, exports every
+symbol include/chol.h declares, and its host-side rows of the hot path -- the task
+graph and the bounds (A9) -- agree with the oracle."""
+import ctypes
+import os
+import re
+
+import pytest
+
+from oracle import bounds as obounds
+from oracle import dag as odag
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def chol():
+    from paper_conf_ipps_agullobehkmt15_b200 import build
+    build.build()
+    import paper_conf_ipps_agullobehkmt15_b200 as c
+    return c
+
+
+def declared_symbols():
+    src = open(os.path.join(ROOT, "include", "chol.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(chol_[a-z_]+)\s*\(", src)))
+
+
+def test_header_symbols_exported(chol):
+    lib = ctypes.CDLL(chol.LIB_PATH)
+    syms = declared_symbols()
+    assert len(syms) >= 19
+    for s in syms:
+        assert hasattr(lib, s), s
+    assert set(syms) == set(chol.EXPORTED)
+
+
+def test_strerror(chol):
+    assert chol.chol_strerror(0) == "success"
+    assert "n <= 0" in chol.chol_strerror(-1)
+
+
+def test_no_gpu_plan_fails_loudly(chol):
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("GPU present")
+    with pytest.raises(chol.CholError) as e:
+        chol.chol_plan(1024, 256)
+    assert e.value.status == -3
+
+
+@pytest.mark.parametrize("N", [1, 2, 3, 5, 8, 12])
+def test_dag_matches_oracle(chol, N):
+    nt, E = chol.chol_dag(N)
+    ts, OE = odag.edges(N)
+    assert nt == len(ts)
+    ids = [chol.chol_task_id(N, t.type, t.i, t.j, t.k) for t in ts]
+    assert sorted(ids) == list(range(nt))
+    oracle_edges = {(ids[p], ids[s]) for p, s in OE}
+    assert set(E) == oracle_edges and len(E) == len(OE)
+
+
+def test_bounds_match_oracle(chol):
+    T_lat = [5e-4, 2e-4, 9e-5, 9e-5]
+    T_thr = [1.2e-4, 1.1e-4, 3.6e-5, 5.7e-5]
+    keys = ["POTRF", "TRSM", "SYRK", "GEMM"]
+    for n, nb, M in [(9600, 960, 1), (19200, 960, 1), (46080, 960, 8), (1024, 256, 2)]:
+        got = chol.chol_bounds(n, nb, M, T_lat, T_thr)
+        ref = obounds.all_bounds(n, nb, dict(zip(keys, T_thr)), dict(zip(keys, T_lat)), M)
+        for k in ("area", "chain", "mixed", "critical_path", "gemm_peak"):
+            assert abs(got[k] - ref[k]) <= 1e-12 * max(1.0, abs(ref[k])), (k, got[k], ref[k])
