@@ -98,14 +98,38 @@ __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, i
   return -1;
 }
 
+// One non-inlined function per job type: each gets its own register allocation
+// (inlining all of them into the persistent kernel made ptxas spill the GEMM
+// accumulators to local memory).
+template <int BS>
+__device__ __noinline__ void job_update(Ctx<BS>& c, int i, int j, int k, int bm, int bn) {
+  sub_update(c, i, j, k, bm, bn);
+}
+template <int BS>
+__device__ __noinline__ void job_trsm(Ctx<BS>& c, int i, int k, int slab) {
+  sub_trsm(c, i, k, slab);
+}
+template <int BS>
+__device__ __noinline__ void job_potrf_diag(Ctx<BS>& c, int k, int b, int* info) {
+  sub_potrf_diag(c, k, b, info);
+}
+template <int BS>
+__device__ __noinline__ void job_potrf_panel(Ctx<BS>& c, int k, int b, int r) {
+  sub_potrf_panel(c, k, b, r);
+}
+template <int BS>
+__device__ __noinline__ void job_potrf_update(Ctx<BS>& c, int k, int b, int r, int q) {
+  sub_potrf_update(c, k, b, r, q);
+}
+
 template <int BS>
 __device__ __forceinline__ void run_job(Ctx<BS>& c, const Job& jb, int* info) {
   switch (jb.type) {
-    case J_UPD: sub_update(c, jb.i, jb.j, jb.k, jb.a, jb.b); break;
-    case J_TRSM: sub_trsm(c, jb.i, jb.k, jb.a); break;
-    case J_DIAG: sub_potrf_diag(c, jb.k, jb.a, info); break;
-    case J_PANEL: sub_potrf_panel(c, jb.k, jb.a, jb.b); break;
-    case J_PUPD: sub_potrf_update(c, jb.k, jb.a, jb.b, jb.c); break;
+    case J_UPD: job_update(c, jb.i, jb.j, jb.k, jb.a, jb.b); break;
+    case J_TRSM: job_trsm(c, jb.i, jb.k, jb.a); break;
+    case J_DIAG: job_potrf_diag(c, jb.k, jb.a, info); break;
+    case J_PANEL: job_potrf_panel(c, jb.k, jb.a, jb.b); break;
+    case J_PUPD: job_potrf_update(c, jb.k, jb.a, jb.b, jb.c); break;
   }
 }
 

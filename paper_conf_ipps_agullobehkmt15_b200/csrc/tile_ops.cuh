@@ -7,9 +7,10 @@
 // dims {nb, nb, ntiles}, box {16, BS, 1}, 128-byte swizzle, so any BS-row x 16-column
 // slab of any tile lands in shared memory with one cp.async.bulk.tensor.
 //
-// CTA shape: 8 compute warps (2 x 4 warp grid, warp tile BS/2 x BS/4, FP64 DMMA
-// m8n8k4 with register accumulators) + 1 producer warp that issues TMA into a
-// kStages-deep mbarrier ring.  Sub-task granularity is a BS x BS block (BS = 96 at
+// CTA shape: 8 warps (2 x 4 warp grid, warp tile BS/2 x BS/4, FP64 DMMA m8n8k4 with
+// register accumulators); thread 0 also issues the TMA loads, kStages-1 stages ahead,
+// into a kStages-deep mbarrier ring.  (No dedicated producer warp: 256 threads keep
+// the per-thread register budget at 255 -- a 9th warp caps it at 168.)  Sub-task granularity is a BS x BS block (BS = 96 at
 // nb = 960, so a GEMM task is 100 CTA sub-tasks of 96 x 96 x 960).
 #pragma once
 #include "dev_common.cuh"
@@ -19,8 +20,8 @@ namespace chol {
 
 constexpr int kComputeWarps = 8;
 constexpr int kComputeThreads = kComputeWarps * 32;
-constexpr int kThreads = kComputeThreads + 32;  // + producer warp
-constexpr int kStages = 4;
+constexpr int kThreads = kComputeThreads;
+constexpr int kStages = 5;
 constexpr int BK = 16;  // doubles per TMA box row (128 bytes)
 constexpr int kBarCompute = 1;  // named barrier id: compute warps only
 constexpr int kBarAll = 2;      // named barrier id: all warps
@@ -57,7 +58,7 @@ struct Ctx {
   int warp, lane;
 
   __device__ double* tile(int i, int j) const { return tiles + tile_index(i, j) * (int64_t)nb * nb; }
-  __device__ bool producer() const { return warp == kComputeWarps; }
+  __device__ bool issuer() const { return threadIdx.x == 0; }
 };
 
 template <int BS>
@@ -85,7 +86,7 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
     }
     fence_mbar_init();
   }
-  if (c.producer() && c.lane == 0) tma_prefetch_desc(map);
+  if (c.issuer()) tma_prefetch_desc(map);
   __syncthreads();
   return c;
 }
@@ -97,67 +98,74 @@ using Acc = double[Cfg<BS>::MI][Cfg<BS>::NI][2];
 // (tile-store indices), "NT" form: both operands K-contiguous (row-major tiles).
 // kbeg, kend multiples of BK.  Called by all warps of the CTA.
 template <int BS>
+__device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, int ra, int64_t tb, int rb, int kk) {
+  using C = Cfg<BS>;
+  const uint32_t st = q % kStages, ph = (q / kStages) & 1;
+  mbar_wait(&c.empty[st], ph ^ 1);  // the previous use of this buffer was released by all warps
+  mbar_arrive_expect_tx(&c.full[st], 2 * C::kOpBytes);
+  char* sa = c.pipe + st * 2 * C::kOpBytes;
+  tma_load_3d(sa, c.map, &c.full[st], kk, ra, (int)ta);
+  tma_load_3d(sa + C::kOpBytes, c.map, &c.full[st], kk, rb, (int)tb);
+}
+
+template <int BS>
 __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, int64_t tb, int rb, int kbeg,
                                               int kend, Acc<BS>& acc) {
   using C = Cfg<BS>;
   const int nst = (kend - kbeg) / BK;
-  if (c.producer()) {
-    if (c.lane == 0) {
-      fence_proxy_async();  // operands may have been written by generic stores (this or other SMs)
-      for (int s = 0; s < nst; ++s) {
-        const uint32_t q = c.it + s, st = q % kStages, ph = (q / kStages) & 1;
-        mbar_wait(&c.empty[st], ph ^ 1);
-        mbar_arrive_expect_tx(&c.full[st], 2 * C::kOpBytes);
-        char* sa = c.pipe + st * 2 * C::kOpBytes;
-        tma_load_3d(sa, c.map, &c.full[st], kbeg + s * BK, ra, (int)ta);
-        tma_load_3d(sa + C::kOpBytes, c.map, &c.full[st], kbeg + s * BK, rb, (int)tb);
-      }
+  if (c.issuer()) {
+    fence_proxy_async();  // operands may have been written by generic stores (this or other SMs)
+    const int pre = nst < kStages - 1 ? nst : kStages - 1;
+    for (int s = 0; s < pre; ++s) issue_stage(c, c.it + s, ta, ra, tb, rb, kbeg + s * BK);
+  }
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  // threadIdx.y is 0 (1-D blocks) but unknown to the compiler: used to make the
+  // stage release depend on every shared load of the stage (see below).
+  const uint32_t rt_zero = threadIdx.y;
+  for (int s = 0; s < nst; ++s) {
+    // keep kStages-1 stages in flight: refill the buffer stage s-1 used
+    if (c.issuer() && s + kStages - 1 < nst)
+      issue_stage(c, c.it + s + kStages - 1, ta, ra, tb, rb, kbeg + (s + kStages - 1) * BK);
+    const uint32_t q = c.it + s, st = q % kStages, ph = (q / kStages) & 1;
+    mbar_wait(&c.full[st], ph);
+    const uint32_t As = smem_u32(c.pipe) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
+    const uint32_t Bs = smem_u32(c.pipe) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
+    uint32_t dep = 0;
+#pragma unroll
+    for (int h = 0; h < 2; ++h) {
+      // Thread (g, t) reads logical 16-byte chunk 2t + h of its row (k = 4t + 2h, +1):
+      // with the 128B swizzle (chunk ^= row & 7) the two rows g, g+1 of one 8-lane
+      // phase land on chunks of opposite parity -> conflict-free LDS.128.
+      const int chunk = ((2 * t + h) ^ g) << 4;
+      double2 af[C::MI], bf[C::NI];
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi) af[mi] = lds128(As + mi * 8 * 128 + chunk);
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) bf[ni] = lds128(Bs + ni * 8 * 128 + chunk);
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(af[mi].x);
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(bf[ni].x);
+      // k-permutation: thread t holds k = 4t+2h (x) and 4t+2h+1 (y) for both operands.
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+        for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].x, bf[ni].x);
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+        for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].y, bf[ni].y);
     }
-  } else {
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
-    const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
-    // threadIdx.y is 0 (1-D blocks) but unknown to the compiler: used to make the
-    // stage release depend on every shared load of the stage (see below).
-    const uint32_t rt_zero = threadIdx.y;
-    for (int s = 0; s < nst; ++s) {
-      const uint32_t q = c.it + s, st = q % kStages, ph = (q / kStages) & 1;
-      mbar_wait(&c.full[st], ph);
-      const uint32_t As = smem_u32(c.pipe) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
-      const uint32_t Bs = smem_u32(c.pipe) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
-      uint32_t dep = 0;
-#pragma unroll
-      for (int h = 0; h < 2; ++h) {
-        // 128B swizzle: 16-byte chunk index ^= (row & 7); rows here are 8-aligned + g.
-        const int chunk = ((h * 4 + t) ^ g) << 4;
-        double2 af[C::MI], bf[C::NI];
-#pragma unroll
-        for (int mi = 0; mi < C::MI; ++mi) af[mi] = lds128(As + mi * 8 * 128 + chunk);
-#pragma unroll
-        for (int ni = 0; ni < C::NI; ++ni) bf[ni] = lds128(Bs + ni * 8 * 128 + chunk);
-#pragma unroll
-        for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(af[mi].x);
-#pragma unroll
-        for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(bf[ni].x);
-        // k-permutation: thread t holds k = 8h+2t (x) and 8h+2t+1 (y) for both operands.
-#pragma unroll
-        for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-          for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].x, bf[ni].x);
-#pragma unroll
-        for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-          for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].y, bf[ni].y);
-      }
-      // Hand the stage back to the producer only once every ld.shared of it has
-      // returned: the arrive is predicated on a value derived from all loaded
-      // registers (lane 0 arrives), so it cannot issue before the loads complete
-      // and a TMA refill can never overwrite data a lane has not read yet.
-      __syncwarp();
-      if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty[st]);
-    }
+    // Release the stage only once every ld.shared of it has returned: the arrive is
+    // predicated on a value derived from all loaded registers (lane 0 arrives), so it
+    // cannot issue before the loads complete and a TMA refill can never overwrite
+    // data a lane has not read yet.
+    __syncwarp();
+    if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty[st]);
   }
   c.it += nst;
 }
@@ -187,23 +195,39 @@ __device__ __forceinline__ void epi_sub_global(const Ctx<BS>& c, const Acc<BS>& 
     }
 }
 
+// D(8x8) -= A(8x8 rows ar.., K=8 at column ak) * B(8x8 rows br.., K=8 at column bk)^T
+// on row-major shared-memory operands with pitch P (doubles): two m8n8k4 DMMAs.
+// d = {D[g][2t], D[g][2t+1]} fragment.
+template <int P>
+__device__ __forceinline__ void smem_dmma_sub8(double& d0, double& d1, const double* A, int ar, int ak,
+                                               const double* Bm, int br, int bk, int g, int t) {
+#pragma unroll
+  for (int kk = 0; kk < 8; kk += 4) {
+    const double a = -A[(ar + g) * P + ak + kk + t];
+    const double bv = Bm[(br + g) * P + bk + kk + t];
+    dmma884(d0, d1, a, bv);
+  }
+}
+
 // X <- (X - acc) * Ld^{-T} for one BS x BS block X (ld ldx) against the lower
 // triangular BS x BS diagonal block Ld (ld ldl): the in-block part of TRSM
 // (L200-202), forward substitution x_c = (b_c - sum_{m<c} x_m L[c][m]) / L[c][c]
-// per row, right-looking inside the block.  Rows are independent, so each
-// compute warp owns BS/8 rows in registers (columns split over lanes) and the
-// only communication is a warp shuffle of x_c.  Compute warps only; ends with a
-// compute-warp barrier.  has_acc = false: acc is ignored (treated as zero).
+// per row.  Blocked right-looking over 8-column panels: a panel is solved by
+// substitution (one thread per row), then the trailing columns are updated with
+// FP64 DMMA (X[:, rest] -= X[:, panel] L[rest, panel]^T).  Compute warps only.
+// has_acc = false: acc is ignored (treated as zero).
 template <int BS>
 __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc, bool has_acc, double* X, int ldx,
                                             const double* Ld, int ldl) {
   using C = Cfg<BS>;
-  const int tid = threadIdx.x;
+  constexpr int P = C::kPitch;
+  const int tid = threadIdx.x, g = c.lane >> 2, t = c.lane & 3;
+  double* xb = c.buf;   // X block (aliases the TMA ring)
+  double* lb = c.lbuf;  // L block, lower part; column BS holds 1/L[c][c]
   // buf aliases the TMA ring: every compute warp must be done reading its last stage.
   bar_sync(kBarCompute, kComputeThreads);
-  // 1. buf = X - acc (fragment layout), lbuf = Ld^T (lower part).
   {
-    const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+    const int wm = c.warp >> 2, wn = c.warp & 3;
 #pragma unroll
     for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
@@ -214,86 +238,137 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc
           v.x -= acc[mi][ni][0];
           v.y -= acc[mi][ni][1];
         }
-        *reinterpret_cast<double2*>(c.buf + r * C::kPitch + cc) = v;
+        *reinterpret_cast<double2*>(xb + r * P + cc) = v;
       }
     for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
       const int r = idx / BS, cc = idx - r * BS;
-      if (cc <= r) c.lbuf[cc * C::kPitch + r] = __ldcg(Ld + (int64_t)r * ldl + cc);
+      if (cc <= r) lb[r * P + cc] = __ldcg(Ld + (int64_t)r * ldl + cc);
     }
+    if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
   }
   bar_sync(kBarCompute, kComputeThreads);
-  // 2. per-warp substitution on BS/8 rows held in registers.
-  double x[C::RW][C::CPL];
-  const int r0 = c.warp * C::RW, lane = c.lane;
+#pragma unroll 1
+  for (int c0 = 0; c0 < BS; c0 += 8) {
+    // (a) panel substitution, one thread per row
+    if (tid < BS) {
+      double v[8];
+      double* xr = xb + tid * P + c0;
 #pragma unroll
-  for (int q = 0; q < C::RW; ++q)
-#pragma unroll
-    for (int s = 0; s < C::CPL; ++s) x[q][s] = c.buf[(r0 + q) * C::kPitch + s * 32 + lane];
-#pragma unroll
-  for (int s = 0; s < C::CPL; ++s) {
-    for (int cl = 0; cl < 32; ++cl) {
-      const int ci = s * 32 + cl;
-      const double* lrow = c.lbuf + ci * C::kPitch;  // lrow[c'] = L[c'][ci]
-      const double rd = 1.0 / lrow[ci];
-      double lc[C::CPL];
-#pragma unroll
-      for (int s2 = 0; s2 < C::CPL; ++s2) lc[s2] = (s2 >= s) ? lrow[s2 * 32 + lane] : 0.0;
-#pragma unroll
-      for (int q = 0; q < C::RW; ++q) {
-        const double v = __shfl_sync(0xffffffffu, x[q][s], cl) * rd;
-        if (lane == cl) x[q][s] = v;
-#pragma unroll
-        for (int s2 = s; s2 < C::CPL; ++s2)
-          if (s2 * 32 + lane > ci) x[q][s2] = fma(-v, lc[s2], x[q][s2]);
+      for (int j = 0; j < 8; j += 2) {
+        const double2 q = *reinterpret_cast<const double2*>(xr + j);
+        v[j] = q.x;
+        v[j + 1] = q.y;
       }
+#pragma unroll
+      for (int j = 0; j < 8; ++j) {
+        v[j] *= lb[(c0 + j) * P + BS];
+#pragma unroll
+        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], lb[(c0 + j2) * P + c0 + j], v[j2]);
+      }
+#pragma unroll
+      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(xr + j) = make_double2(v[j], v[j + 1]);
     }
+    bar_sync(kBarCompute, kComputeThreads);
+    // (b) trailing update X[:, c0+8:] -= X[:, c0:c0+8] L[c0+8:, c0:c0+8]^T
+    const int nN = (BS - c0 - 8) / 8;
+    if (nN == 0) break;
+    for (int blk = c.warp; blk < (BS / 8) * nN; blk += kComputeWarps) {
+      const int mb = blk / nN, nk = blk - mb * nN;
+      const int r = mb * 8, q = c0 + 8 + nk * 8;
+      double2 d = *reinterpret_cast<const double2*>(xb + (r + g) * P + q + 2 * t);
+      smem_dmma_sub8<P>(d.x, d.y, xb, r, c0, lb, q, c0, g, t);
+      *reinterpret_cast<double2*>(xb + (r + g) * P + q + 2 * t) = d;
+    }
+    bar_sync(kBarCompute, kComputeThreads);
   }
-  // 3. write the solved rows back (coalesced).
-#pragma unroll
-  for (int q = 0; q < C::RW; ++q)
-#pragma unroll
-    for (int s = 0; s < C::CPL; ++s) __stcg(X + (int64_t)(r0 + q) * ldx + s * 32 + lane, x[q][s]);
+  // write the solved block back (coalesced rows)
+  for (int idx = tid; idx < BS * (BS / 2); idx += kComputeThreads) {
+    const int r = idx / (BS / 2), cc = 2 * (idx - r * (BS / 2));
+    __stcg(reinterpret_cast<double2*>(X + (int64_t)r * ldx + cc), *reinterpret_cast<const double2*>(xb + r * P + cc));
+  }
   bar_sync(kBarCompute, kComputeThreads);
 }
 
-// Unblocked Cholesky of the BS x BS diagonal block A (ld lda), lower, in shared
-// memory (POTRF, L196-199).  Right-looking column algorithm; on a pivot !(d > 0)
-// records info = col0 + c + 1 with atomicMin (LAPACK convention, reading R6).
-// Compute warps only.
+// Cholesky of the BS x BS diagonal block A (ld lda), lower, in shared memory
+// (POTRF, L196-199), blocked right-looking over 8-column panels:
+//   (a) one warp factors the 8x8 diagonal block (column algorithm of SURVEY §8c),
+//   (b) the rows below solve against it (one thread per row),
+//   (c) the trailing lower triangle is updated with FP64 DMMA.
+// A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
+// reading R6).  Compute warps only.
 template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   using C = Cfg<BS>;
-  const int tid = threadIdx.x;
+  constexpr int P = C::kPitch;
+  const int tid = threadIdx.x, lane = c.lane, g = lane >> 2, t = lane & 3;
   double* a = c.buf;
   bar_sync(kBarCompute, kComputeThreads);  // buf aliases the TMA ring
   for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
     const int r = idx / BS, cc = idx - r * BS;
-    if (cc <= r) a[r * C::kPitch + cc] = __ldcg(A + (int64_t)r * lda + cc);
+    if (cc <= r) a[r * P + cc] = __ldcg(A + (int64_t)r * lda + cc);
   }
   bar_sync(kBarCompute, kComputeThreads);
-  for (int j = 0; j < BS; ++j) {
-    const double d = a[j * C::kPitch + j];
-    const double ljj = sqrt(d);
-    if (tid == 0 && !(d > 0.0)) atomicMin(info, col0 + j + 1);
-    if (tid < BS - 1 - j) {
-      const int r = j + 1 + tid;
-      a[r * C::kPitch + j] = a[r * C::kPitch + j] / ljj;
+#pragma unroll 1
+  for (int c0 = 0; c0 < BS; c0 += 8) {
+    // (a) 8x8 diagonal block, warp 0, lane r < 8 owns row c0 + r
+    if (c.warp == 0) {
+#pragma unroll
+      for (int j = 0; j < 8; ++j) {
+        const double d = a[(c0 + j) * P + c0 + j];
+        const double ljj = sqrt(d);
+        if (lane == 0 && !(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
+        __syncwarp();
+        if (lane > j && lane < 8) a[(c0 + lane) * P + c0 + j] = a[(c0 + lane) * P + c0 + j] / ljj;
+        if (lane == j) {
+          a[(c0 + j) * P + c0 + j] = ljj;
+          a[(c0 + j) * P + BS] = 1.0 / ljj;
+        }
+        __syncwarp();
+        if (lane > j && lane < 8) {
+          const double lrj = a[(c0 + lane) * P + c0 + j];
+          for (int q = j + 1; q <= lane; ++q)
+            a[(c0 + lane) * P + c0 + q] = fma(-lrj, a[(c0 + q) * P + c0 + j], a[(c0 + lane) * P + c0 + q]);
+        }
+        __syncwarp();
+      }
     }
     bar_sync(kBarCompute, kComputeThreads);
-    if (tid == 0) a[j * C::kPitch + j] = ljj;
-    const int m = BS - 1 - j;
-    for (int idx = tid; idx < m * m; idx += kComputeThreads) {
-      const int rr = idx / m, cc = idx - rr * m;
-      if (cc <= rr) {
-        const int r = j + 1 + rr, col = j + 1 + cc;
-        a[r * C::kPitch + col] = fma(-a[r * C::kPitch + j], a[col * C::kPitch + j], a[r * C::kPitch + col]);
+    const int rows = BS - c0 - 8;
+    if (rows == 0) break;
+    // (b) panel rows below the diagonal block
+    if (tid < rows) {
+      double v[8];
+      double* ar = a + (c0 + 8 + tid) * P + c0;
+#pragma unroll
+      for (int j = 0; j < 8; ++j) v[j] = ar[j];
+#pragma unroll
+      for (int j = 0; j < 8; ++j) {
+        v[j] *= a[(c0 + j) * P + BS];
+#pragma unroll
+        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], a[(c0 + j2) * P + c0 + j], v[j2]);
       }
+#pragma unroll
+      for (int j = 0; j < 8; ++j) ar[j] = v[j];
+    }
+    bar_sync(kBarCompute, kComputeThreads);
+    // (c) trailing lower update: A[r][q] -= L[r, panel] L[q, panel]^T, 8x8 blocks nk <= mb
+    const int nr = rows / 8;
+    for (int blk = c.warp; blk < nr * (nr + 1) / 2; blk += kComputeWarps) {
+      int mb = 0, rem = blk;
+      while (rem > mb) {
+        rem -= mb + 1;
+        ++mb;
+      }
+      const int r = c0 + 8 + mb * 8, q = c0 + 8 + rem * 8;
+      double2 d = *reinterpret_cast<const double2*>(a + (r + g) * P + q + 2 * t);
+      smem_dmma_sub8<P>(d.x, d.y, a, r, c0, a, q, c0, g, t);
+      *reinterpret_cast<double2*>(a + (r + g) * P + q + 2 * t) = d;
     }
     bar_sync(kBarCompute, kComputeThreads);
   }
   for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
     const int r = idx / BS, cc = idx - r * BS;
-    if (cc <= r) __stcg(A + (int64_t)r * lda + cc, a[r * C::kPitch + cc]);
+    if (cc <= r) __stcg(A + (int64_t)r * lda + cc, a[r * P + cc]);
   }
 }
 
@@ -307,8 +382,7 @@ template <int BS>
 __device__ __forceinline__ void sub_update(Ctx<BS>& c, int i, int j, int k, int bm, int bn) {
   Acc<BS> acc;
   gemm_mainloop(c, tile_index(i, k), bm * BS, tile_index(j, k), bn * BS, 0, c.nb, acc);
-  if (!c.producer())
-    epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
+  epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
 }
 
 // TRSM_i_k sub-task = row slab `slab` of A_ik:  X <- X L_kk^{-T}  (L200-202),
@@ -321,13 +395,11 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
   for (int cb = 0; cb < nbb; ++cb) {
     Acc<BS> acc;
     if (cb > 0) gemm_mainloop(c, tile_index(i, k), slab * BS, tile_index(k, k), cb * BS, 0, cb * BS, acc);
-    if (!c.producer()) {
-      solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
-      // X[:, cb] (generic stores) is read by TMA in the next block: complete the stores
-      // at L2 (gpu-scope fence), then order them before async-proxy accesses.
-      __threadfence();
-      fence_proxy_async();
-    }
+    solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+    // X[:, cb] (generic stores) is read by TMA in the next block: complete the stores
+    // at L2 (gpu-scope fence), then order them before async-proxy accesses.
+    __threadfence();
+    fence_proxy_async();
     bar_sync(kBarAll, kThreads);
   }
 }
@@ -336,19 +408,15 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
 //   potf2 of block (b, b)
 template <int BS>
 __device__ __forceinline__ void sub_potrf_diag(Ctx<BS>& c, int k, int b, int* info) {
-  if (!c.producer()) {
-    double* A = c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS;
-    potf2_block(c, A, c.nb, k * c.nb + b * BS, info);
-  }
+  double* A = c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS;
+  potf2_block(c, A, c.nb, k * c.nb + b * BS, info);
 }
 //   block (r, b), r > b:  X <- X L_bb^{-T}
 template <int BS>
 __device__ __forceinline__ void sub_potrf_panel(Ctx<BS>& c, int k, int b, int r) {
-  if (!c.producer()) {
-    double* T = c.tile(k, k);
-    Acc<BS> acc;
-    solve_block(c, acc, false, T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
-  }
+  double* T = c.tile(k, k);
+  Acc<BS> acc;
+  solve_block(c, acc, false, T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
 }
 //   block (r, q), b < q <= r:  A[r, q] -= L[r, b] L[q, b]^T   (K = BS)
 template <int BS>
@@ -356,7 +424,7 @@ __device__ __forceinline__ void sub_potrf_update(Ctx<BS>& c, int k, int b, int r
   Acc<BS> acc;
   const int64_t t = tile_index(k, k);
   gemm_mainloop(c, t, r * BS, t, q * BS, b * BS, (b + 1) * BS, acc);
-  if (!c.producer()) epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);
+  epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);
 }
 
 }  // namespace chol
