@@ -35,7 +35,8 @@ struct Cfg {
   static constexpr int kPipeBytes = kStages * 2 * kOpBytes;
   static constexpr int kPitch = BS + 2;            // doubles; keeps double2 alignment
   static constexpr int kBufBytes = BS * kPitch * 8;
-  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + 2 * kStages * 8 + 1024;
+  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + (2 * kStages + 2) * 8 + 1024;
+  static_assert(kBufBytes >= BS * BS * 8, "lbuf holds a TMA-prefetched BS x BS C block");
   static constexpr int RW = BS / kComputeWarps;    // rows per warp in the solves
   static constexpr int CPL = BS / 32;              // columns per lane in the solves
   static_assert(BS % 32 == 0 && WM % 8 == 0 && WN % 8 == 0, "tile shape");
@@ -54,7 +55,9 @@ struct Ctx {
   double* lbuf;    // BS x kPitch (transposed L block)
   uint64_t* full;  // kStages
   uint64_t* empty; // kStages
+  uint64_t* cbar;  // C-block prefetch (TMA -> lbuf)
   uint32_t it;     // stages consumed so far
+  uint32_t cphase; // parity of the next cbar completion
   int warp, lane;
 
   __device__ double* tile(int i, int j) const { return tiles + tile_index(i, j) * (int64_t)nb * nb; }
@@ -76,7 +79,9 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
   c.lbuf = reinterpret_cast<double*>(base + C::kPipeBytes);
   c.full = reinterpret_cast<uint64_t*>(base + C::kPipeBytes + C::kBufBytes);
   c.empty = c.full + kStages;
+  c.cbar = c.empty + kStages;
   c.it = 0;
+  c.cphase = 0;
   c.warp = threadIdx.x >> 5;
   c.lane = threadIdx.x & 31;
   if (threadIdx.x == 0) {
@@ -84,6 +89,7 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
       mbar_init(&c.full[s], 1);
       mbar_init(&c.empty[s], kComputeWarps);
     }
+    mbar_init(c.cbar, 1);
     fence_mbar_init();
   }
   if (c.issuer()) tma_prefetch_desc(map);
@@ -97,6 +103,25 @@ using Acc = double[Cfg<BS>::MI][Cfg<BS>::NI][2];
 // acc = A[ra:ra+BS, kbeg:kend] * B[rb:rb+BS, kbeg:kend]^T with A = tile ta, B = tile tb
 // (tile-store indices), "NT" form: both operands K-contiguous (row-major tiles).
 // kbeg, kend multiples of BK.  Called by all warps of the CTA.
+// Prefetch the BS x BS block (rows r0.., cols c0..) of store tile `tile` into lbuf with
+// TMA (BS/16 boxes of BS rows x 128 B, 128B-swizzled), completing on cbar.  Issued by
+// thread 0 right after the mainloop prologue so the epilogue's C read overlaps the
+// mainloop.
+struct CPrefetch {
+  int64_t tile;
+  int r0, c0;
+};
+
+template <int BS>
+__device__ __forceinline__ void prefetch_c(Ctx<BS>& c, int64_t tile, int r0, int c0) {
+  if (!c.issuer()) return;
+  fence_proxy_async();
+  mbar_arrive_expect_tx(c.cbar, BS * BS * 8);
+  char* dst = reinterpret_cast<char*>(c.lbuf);
+#pragma unroll 1
+  for (int b = 0; b < BS / 16; ++b) tma_load_3d(dst + b * BS * 128, c.map, c.cbar, c0 + 16 * b, r0, (int)tile);
+}
+
 template <int BS>
 __device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, int ra, int64_t tb, int rb, int kk) {
   using C = Cfg<BS>;
@@ -110,13 +135,14 @@ __device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, 
 
 template <int BS>
 __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, int64_t tb, int rb, int kbeg,
-                                              int kend, Acc<BS>& acc) {
+                                              int kend, Acc<BS>& acc, const CPrefetch* cpre = nullptr) {
   using C = Cfg<BS>;
   const int nst = (kend - kbeg) / BK;
   if (c.issuer()) {
     fence_proxy_async();  // operands may have been written by generic stores (this or other SMs)
     const int pre = nst < kStages - 1 ? nst : kStages - 1;
     for (int s = 0; s < pre; ++s) issue_stage(c, c.it + s, ta, ra, tb, rb, kbeg + s * BK);
+    if (cpre) prefetch_c(c, cpre->tile, cpre->r0, cpre->c0);
   }
 #pragma unroll
   for (int mi = 0; mi < C::MI; ++mi)
@@ -170,22 +196,31 @@ __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, in
   c.it += nst;
 }
 
-// C[0:BS, 0:BS] -= acc for the BS x BS block at Cblk (leading dimension ldc).
+// Prefetch the BS x BS block (rows r0.., cols c0..) of store tile `tile` into lbuf with
+// TMA (BS/16 boxes of BS rows x 128 B, 128B-swizzled), completing on cbar.  Issued by
+// thread 0 at the start of a job so the C read of the epilogue overlaps the mainloop.
+// C[0:BS, 0:BS] -= acc for the BS x BS block at Cblk (leading dimension ldc); the old
+// C values come from the lbuf prefetch (prefetch_c), results go to global memory.
 // lower_only: diagonal block of a diagonal tile -- only r >= c is written (SYRK, L207-208).
 template <int BS>
-__device__ __forceinline__ void epi_sub_global(const Ctx<BS>& c, const Acc<BS>& acc, double* Cblk, int ldc,
+__device__ __forceinline__ void epi_sub_global(Ctx<BS>& c, const Acc<BS>& acc, double* Cblk, int ldc,
                                                bool lower_only) {
   using C = Cfg<BS>;
   const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  mbar_wait(c.cbar, c.cphase);
+  c.cphase ^= 1;
+  const uint32_t cs = smem_u32(c.lbuf);
 #pragma unroll
   for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
     for (int ni = 0; ni < C::NI; ++ni) {
       const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
-      double2* p = reinterpret_cast<double2*>(Cblk + (int64_t)r * ldc + cc);
-      double2 v = __ldcg(p);
+      // box cc/16, row r, logical 16-byte chunk (cc%16)/2, 128B swizzle
+      const uint32_t addr = cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4);
+      double2 v = lds128(addr);
       v.x -= acc[mi][ni][0];
       v.y -= acc[mi][ni][1];
+      double2* p = reinterpret_cast<double2*>(Cblk + (int64_t)r * ldc + cc);
       if (!lower_only) {
         __stcg(p, v);
       } else {
@@ -381,7 +416,8 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
 template <int BS>
 __device__ __forceinline__ void sub_update(Ctx<BS>& c, int i, int j, int k, int bm, int bn) {
   Acc<BS> acc;
-  gemm_mainloop(c, tile_index(i, k), bm * BS, tile_index(j, k), bn * BS, 0, c.nb, acc);
+  const CPrefetch cp{tile_index(i, j), bm * BS, bn * BS};
+  gemm_mainloop(c, tile_index(i, k), bm * BS, tile_index(j, k), bn * BS, 0, c.nb, acc, &cp);
   epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
 }
 
@@ -423,7 +459,8 @@ template <int BS>
 __device__ __forceinline__ void sub_potrf_update(Ctx<BS>& c, int k, int b, int r, int q) {
   Acc<BS> acc;
   const int64_t t = tile_index(k, k);
-  gemm_mainloop(c, t, r * BS, t, q * BS, b * BS, (b + 1) * BS, acc);
+  const CPrefetch cp{t, r * BS, q * BS};
+  gemm_mainloop(c, t, r * BS, t, q * BS, b * BS, (b + 1) * BS, acc, &cp);
   epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);
 }
 
