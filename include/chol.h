@@ -68,7 +68,8 @@ typedef struct {
   int trsm_pin_distance; /* STATIC only: TRSM_i_k with i-k <= d are pinned (0 = N, all) */
   int latency_workers;   /* STATIC only: CTAs reserved for pinned tasks (0 = 8) */
   int grid_p, grid_q;    /* 2D block-cyclic process grid (0,0 = 1 x ngpus) */
-  int trace;             /* 1 = record per-task t0/t1 (needed by chol_trace) */
+  int trace;             /* 1 = record per-task t0/t1 (needed by chol_trace);
+                            2 = also per-job (CTA sub-task) records (chol_job_trace) */
   int executor;          /* CHOL_EXEC_* */
   int workers;           /* persistent CTAs (0 = one per SM) */
 } chol_opts_t;
@@ -107,6 +108,14 @@ int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* L, int64_t 
  * cap = 0 to query), sets *nrecs to the number of tasks and *makespan_s to
  * max t1 - min t0 in seconds. */
 int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int64_t* nrecs, double* makespan_s);
+
+/* Per-job (CTA sub-task) trace of the last factorization by the persistent
+ * scheduler (requires opts.trace = 2): per job j, out[4j] = t0_ns, out[4j+1] =
+ * t1_ns (as chol_trace), out[4j+2] = worker << 32 | SM id, out[4j+3] = job type
+ * << 32 | dense task id (job types: 0 SYRK/GEMM block, 1 TRSM row slab, 2 POTRF
+ * diagonal block, 3 POTRF panel block, 4 POTRF update block).  At most cap jobs;
+ * *njobs = number of jobs.  -7 if not available. */
+int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t* njobs);
 
 int chol_destroy(chol_plan_t p);
 const char* chol_strerror(int status);

@@ -64,6 +64,7 @@ def _load():
         "chol_dag": ([i64, ctypes.POINTER(i64), ctypes.POINTER(i64), ctypes.POINTER(i64), i64], i32),
         "chol_task_id": ([i64, i32, i32, i32, i32, ctypes.POINTER(i64)], i32),
         "chol_bounds": ([i64, i64, i32, dp, dp, dp], i32),
+        "chol_job_trace": ([P, ctypes.POINTER(ctypes.c_uint64), i64, ctypes.POINTER(i64)], i32),
     }
     for name, (args, res) in sig.items():
         f = getattr(L, name)
@@ -76,7 +77,7 @@ _lib = _load()
 EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_destroy", "chol_strerror",
             "chol_generate", "chol_scatter", "chol_gather", "chol_factor_inplace", "chol_last_times",
             "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
-            "chol_dag", "chol_task_id", "chol_bounds")
+            "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace")
 
 
 def _ptr(x) -> int:
@@ -134,6 +135,17 @@ def chol_trace(plan: int):
     out = [{"type": r.type, "gpu": r.gpu, "worker": r.worker, "i": r.i, "j": r.j, "k": r.k,
             "t0_ns": r.t0_ns, "t1_ns": r.t1_ns} for r in recs[:n.value]]
     return out, ms.value
+
+
+def chol_job_trace(plan: int):
+    """numpy array (njobs, 4): t0_ns, t1_ns, worker << 32 | smid, type << 32 | task id."""
+    import numpy as np
+    n = ctypes.c_int64(0)
+    _check(_lib.chol_job_trace(plan, None, 0, ctypes.byref(n)), "chol_job_trace")
+    out = np.zeros((max(n.value, 1), 4), dtype=np.uint64)
+    _check(_lib.chol_job_trace(plan, out.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)), n.value,
+                               ctypes.byref(n)), "chol_job_trace")
+    return out[:n.value]
 
 
 def chol_destroy(plan: int) -> None:

@@ -118,7 +118,7 @@ extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t*
   if (o) opts = *o;
   if (opts.policy < 0 || opts.policy > 2 || opts.executor < 0 || opts.executor > 1 || opts.trsm_pin_distance < 0 ||
       opts.latency_workers < 0 || opts.workers < 0 || opts.grid_p < 0 || opts.grid_q < 0 || opts.trace < 0 ||
-      opts.trace > 1)
+      opts.trace > 2)
     return -6;
   int ndev = 0;
   if (cudaGetDeviceCount(&ndev) != cudaSuccess) ndev = 0;
@@ -423,6 +423,13 @@ extern "C" int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int
   if (nrecs) *nrecs = w;
   if (makespan_s) *makespan_s = (hi > lo) ? (hi - lo) * 1e-9 : 0.0;
   return 0;
+}
+
+extern "C" int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t* njobs) {
+  if (!p) return -4;
+  if (!p->sched || p->opts.trace != 2 || !p->factored) return -7;
+  cudaSetDevice(p->device);
+  return sched_job_trace(p->sched, out, cap, njobs);
 }
 
 // ------------------------------------------------------------------ calibration / single tasks

@@ -53,6 +53,7 @@ struct DevSched {
   int* q_tail;             // kQueues * kQStride
   int* done_nodes;
   int* finished;
+  uint64_t* job_trace;     // trace == 2: per job {t0, t1, worker << 32 | smid}
   int total_nodes;
   int latency_workers;     // STATIC: CTAs [0, latency_workers) serve the pinned queues only
   int policy;
@@ -172,6 +173,11 @@ __global__ void __launch_bounds__(kThreads, 1) k_sched(const __grid_constant__ C
       const int node = d.job_node[job];
       if (sp.tr_t0) {
         const uint64_t t_end = globaltimer_ns() - *sp.tr_base;
+        if (d.job_trace) {
+          d.job_trace[3 * (size_t)job] = s_t0;
+          d.job_trace[3 * (size_t)job + 1] = t_end;
+          d.job_trace[3 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
+        }
         const int pt = d.node_paper[node];
         atomicMin(reinterpret_cast<unsigned long long*>(sp.tr_t0 + pt), (unsigned long long)s_t0);
         atomicMax(reinterpret_cast<unsigned long long*>(sp.tr_t1 + pt),
@@ -209,6 +215,9 @@ struct SchedState {
   void* dev_pristine = nullptr; // initial node_deps / node_left
   size_t pristine_bytes = 0;
   int* roots = nullptr;
+  uint64_t* job_trace = nullptr;           // device, 3 per job (trace == 2)
+  std::vector<int16_t> h_job_type;         // host copies for chol_job_trace
+  std::vector<int> h_job_paper;
 };
 
 namespace {
@@ -349,6 +358,12 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
 
   st->nnodes = nnodes;
   st->njobs = (int)B.jobs.size();
+  st->h_job_type.resize(st->njobs);
+  st->h_job_paper.resize(st->njobs);
+  for (int j = 0; j < st->njobs; ++j) {
+    st->h_job_type[j] = B.jobs[j].type;
+    st->h_job_paper[j] = B.paper[B.job_node[j]];
+  }
   st->nroots = (int)roots.size();
 
   // ---- device layout: static (read-only) part
@@ -426,6 +441,14 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   d.done_nodes = reinterpret_cast<int*>(D + d_done);
   d.finished = reinterpret_cast<int*>(D + d_fin);
   d.total_nodes = nnodes;
+  if (opts->trace == 2) {
+    if ((e = cudaMalloc(&st->job_trace, (size_t)st->njobs * 3 * sizeof(uint64_t)))) {
+      cudaGetLastError();
+      sched_destroy(st);
+      return -9;
+    }
+  }
+  d.job_trace = st->job_trace;
   d.policy = opts->policy;
   d.latency_workers = opts->policy == CHOL_POLICY_STATIC ? (opts->latency_workers > 0 ? opts->latency_workers : 8) : 0;
 
@@ -473,11 +496,28 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
 
 int sched_workers(const SchedState* st) { return st ? st->workers : 0; }
 
+int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* njobs) {
+  if (njobs) *njobs = st->njobs;
+  if (!st->job_trace) return -7;
+  if (!out || cap <= 0) return 0;
+  std::vector<uint64_t> h((size_t)st->njobs * 3);
+  cudaError_t e = cudaMemcpy(h.data(), st->job_trace, h.size() * 8, cudaMemcpyDeviceToHost);
+  if (e) return -100 - (int)e;
+  for (int64_t j = 0; j < st->njobs && j < cap; ++j) {
+    out[4 * j] = h[3 * j];
+    out[4 * j + 1] = h[3 * j + 1];
+    out[4 * j + 2] = h[3 * j + 2];
+    out[4 * j + 3] = ((uint64_t)(uint16_t)st->h_job_type[j] << 32) | (uint32_t)st->h_job_paper[j];
+  }
+  return 0;
+}
+
 void sched_destroy(SchedState* st) {
   if (!st) return;
   cudaFree(st->dev_static);
   cudaFree(st->dev_dynamic);
   cudaFree(st->dev_pristine);
+  cudaFree(st->job_trace);
   delete st;
 }
 

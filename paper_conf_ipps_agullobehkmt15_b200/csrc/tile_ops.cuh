@@ -92,7 +92,7 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
     mbar_init(c.cbar, 1);
     fence_mbar_init();
   }
-  if (c.issuer()) tma_prefetch_desc(map);
+  if (c.issuer() && map) tma_prefetch_desc(map);
   __syncthreads();
   return c;
 }
@@ -230,67 +230,146 @@ __device__ __forceinline__ void epi_sub_global(Ctx<BS>& c, const Acc<BS>& acc, d
     }
 }
 
-// D(8x8) -= A(8x8 rows ar.., K=8 at column ak) * B(8x8 rows br.., K=8 at column bk)^T
-// on row-major shared-memory operands with pitch P (doubles): two m8n8k4 DMMAs.
-// d = {D[g][2t], D[g][2t+1]} fragment.
-template <int P>
-__device__ __forceinline__ void smem_dmma_sub8(double& d0, double& d1, const double* A, int ar, int ak,
-                                               const double* Bm, int br, int bk, int g, int t) {
+// dst[r*P + c] = src[r*ld + c] for a BS x BS block: 16-byte chunks, every load of
+// the thread issued before the first shared store (latency paid once).
+template <int BS>
+__device__ __forceinline__ void load_block(double* dst, const double* src, int64_t ld) {
+  constexpr int P = Cfg<BS>::kPitch, CH = BS / 2, NPT = BS * CH / kComputeThreads;
+  // loads in flight per thread (register budget)
+  constexpr int BATCH = NPT % 6 == 0 ? 6 : (NPT % 4 == 0 ? 4 : (NPT % 2 == 0 ? 2 : 1));
+  static_assert((BS * CH) % kComputeThreads == 0 && NPT % BATCH == 0, "block chunks per thread");
 #pragma unroll
-  for (int kk = 0; kk < 8; kk += 4) {
-    const double a = -A[(ar + g) * P + ak + kk + t];
-    const double bv = Bm[(br + g) * P + bk + kk + t];
-    dmma884(d0, d1, a, bv);
+  for (int i0 = 0; i0 < NPT; i0 += BATCH) {
+    double2 v[BATCH];
+#pragma unroll
+    for (int i = 0; i < BATCH; ++i) {
+      const int idx = threadIdx.x + (i0 + i) * kComputeThreads, r = idx / CH, c2 = idx - r * CH;
+      v[i] = __ldcg(reinterpret_cast<const double2*>(src + r * ld + 2 * c2));
+    }
+#pragma unroll
+    for (int i = 0; i < BATCH; ++i) {
+      const int idx = threadIdx.x + (i0 + i) * kComputeThreads, r = idx / CH, c2 = idx - r * CH;
+      *reinterpret_cast<double2*>(dst + r * P + 2 * c2) = v[i];
+    }
+  }
+}
+
+// Panel buffers for the register-resident in-block algorithms: two BS x 8 panels
+// (double-buffered) at the end of lbuf's padding-free tail.  lbuf layout:
+//   [0, BS*kPitch)  L block (solve_block) -- pitch kPitch, column BS holds 1/L[c][c]
+// The panels live in buf (which aliases the TMA ring; the ring is idle here).
+constexpr int kPanelPitch = 10;  // doubles per panel row (8 + 2 pad: fewer bank conflicts)
+
+// Load the BS x BS block at G (ld ldg) into x[][][] in the accumulator fragment
+// layout (thread owns rows wm*WM + mi*8 + g, cols wn*WN + ni*8 + 2t, +1).
+template <int BS>
+__device__ __forceinline__ void frag_load(const Ctx<BS>& c, Acc<BS>& x, const double* G, int64_t ldg) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const double2 v = __ldcg(reinterpret_cast<const double2*>(G + (int64_t)(wm * C::WM + mi * 8 + g) * ldg +
+                                                                wn * C::WN + ni * 8 + 2 * t));
+      x[mi][ni][0] = v.x;
+      x[mi][ni][1] = v.y;
+    }
+}
+
+template <int BS>
+__device__ __forceinline__ void frag_store(const Ctx<BS>& c, const Acc<BS>& x, double* G, int64_t ldg,
+                                           bool lower_blocks_only) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int rb = wm * C::MI + mi, cb = wn * C::NI + ni;
+      if (lower_blocks_only && cb > rb) continue;
+      __stcg(reinterpret_cast<double2*>(G + (int64_t)(rb * 8 + g) * ldg + cb * 8 + 2 * t),
+             make_double2(x[mi][ni][0], x[mi][ni][1]));
+    }
+}
+
+// Owner warps (those holding 8-column block p) copy that column block of x to the panel.
+template <int BS>
+__device__ __forceinline__ void frag_to_panel(const Ctx<BS>& c, const Acc<BS>& x, int p, double* pan) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  if (wn != p / C::NI) return;
+  const int ni = p % C::NI;
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi) {
+    const int r = wm * C::WM + mi * 8 + g;
+#pragma unroll
+    for (int q = 0; q < C::NI; ++q)
+      if (q == ni) *reinterpret_cast<double2*>(pan + r * kPanelPitch + 2 * t) = make_double2(x[mi][q][0], x[mi][q][1]);
+  }
+}
+template <int BS>
+__device__ __forceinline__ void panel_to_frag(const Ctx<BS>& c, Acc<BS>& x, int p, const double* pan) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  if (wn != p / C::NI) return;
+  const int ni = p % C::NI;
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi) {
+    const int r = wm * C::WM + mi * 8 + g;
+    const double2 v = *reinterpret_cast<const double2*>(pan + r * kPanelPitch + 2 * t);
+#pragma unroll
+    for (int q = 0; q < C::NI; ++q)
+      if (q == ni) {
+        x[mi][q][0] = v.x;
+        x[mi][q][1] = v.y;
+      }
   }
 }
 
 // X <- (X - acc) * Ld^{-T} for one BS x BS block X (ld ldx) against the lower
 // triangular BS x BS diagonal block Ld (ld ldl): the in-block part of TRSM
 // (L200-202), forward substitution x_c = (b_c - sum_{m<c} x_m L[c][m]) / L[c][c]
-// per row.  Blocked right-looking over 8-column panels: a panel is solved by
-// substitution (one thread per row), then the trailing columns are updated with
-// FP64 DMMA (X[:, rest] -= X[:, panel] L[rest, panel]^T).  Compute warps only.
-// has_acc = false: acc is ignored (treated as zero).
+// per row.  Register-resident, blocked right-looking over 8-column panels: X stays
+// in the accumulator fragments; for each panel the owner warps copy it to a shared
+// panel buffer, one thread per row solves it against the 8x8 diagonal block of L,
+// and every warp updates its trailing column blocks with FP64 DMMA
+// (X[:, later] -= X[:, panel] L[later, panel]^T).  has_acc = false: X alone.
 template <int BS>
 __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc, bool has_acc, double* X, int ldx,
                                             const double* Ld, int ldl) {
   using C = Cfg<BS>;
   constexpr int P = C::kPitch;
-  const int tid = threadIdx.x, g = c.lane >> 2, t = c.lane & 3;
-  double* xb = c.buf;   // X block (aliases the TMA ring)
-  double* lb = c.lbuf;  // L block, lower part; column BS holds 1/L[c][c]
-  // buf aliases the TMA ring: every compute warp must be done reading its last stage.
-  bar_sync(kBarCompute, kComputeThreads);
-  {
-    const int wm = c.warp >> 2, wn = c.warp & 3;
+  const int tid = threadIdx.x, wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  double* lb = c.lbuf;  // L block; column BS holds 1/L[c][c]
+  double* pans = c.buf; // 2 panels of BS x kPanelPitch (the TMA ring is idle here)
+  Acc<BS> x;
+  frag_load(c, x, X, ldx);
+  if (has_acc) {
 #pragma unroll
     for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) {
-        const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
-        double2 v = __ldcg(reinterpret_cast<const double2*>(X + (int64_t)r * ldx + cc));
-        if (has_acc) {
-          v.x -= acc[mi][ni][0];
-          v.y -= acc[mi][ni][1];
-        }
-        *reinterpret_cast<double2*>(xb + r * P + cc) = v;
+        x[mi][ni][0] -= acc[mi][ni][0];
+        x[mi][ni][1] -= acc[mi][ni][1];
       }
-    for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
-      const int r = idx / BS, cc = idx - r * BS;
-      if (cc <= r) lb[r * P + cc] = __ldcg(Ld + (int64_t)r * ldl + cc);
-    }
-    if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
   }
+  // buf/lbuf reuse: every warp must be done with the TMA ring and the previous lbuf use.
   bar_sync(kBarCompute, kComputeThreads);
+  load_block<BS>(lb, Ld, ldl);
+  if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
 #pragma unroll 1
-  for (int c0 = 0; c0 < BS; c0 += 8) {
-    // (a) panel substitution, one thread per row
-    if (tid < BS) {
+  for (int p = 0; p < BS / 8; ++p) {
+    const int c0 = 8 * p;
+    double* pan = pans + (p & 1) * BS * kPanelPitch;
+    frag_to_panel(c, x, p, pan);
+    bar_sync(kBarCompute, kComputeThreads);  // (also publishes lb on p == 0)
+    if (tid < BS) {  // substitution of row tid against L[c0:c0+8, c0:c0+8]
       double v[8];
-      double* xr = xb + tid * P + c0;
+      double* pr = pan + tid * kPanelPitch;
 #pragma unroll
       for (int j = 0; j < 8; j += 2) {
-        const double2 q = *reinterpret_cast<const double2*>(xr + j);
+        const double2 q = *reinterpret_cast<const double2*>(pr + j);
         v[j] = q.x;
         v[j + 1] = q.y;
       }
@@ -301,110 +380,128 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc
         for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], lb[(c0 + j2) * P + c0 + j], v[j2]);
       }
 #pragma unroll
-      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(xr + j) = make_double2(v[j], v[j + 1]);
+      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(pr + j) = make_double2(v[j], v[j + 1]);
     }
     bar_sync(kBarCompute, kComputeThreads);
-    // (b) trailing update X[:, c0+8:] -= X[:, c0:c0+8] L[c0+8:, c0:c0+8]^T
-    const int nN = (BS - c0 - 8) / 8;
-    if (nN == 0) break;
-    for (int blk = c.warp; blk < (BS / 8) * nN; blk += kComputeWarps) {
-      const int mb = blk / nN, nk = blk - mb * nN;
-      const int r = mb * 8, q = c0 + 8 + nk * 8;
-      double2 d = *reinterpret_cast<const double2*>(xb + (r + g) * P + q + 2 * t);
-      smem_dmma_sub8<P>(d.x, d.y, xb, r, c0, lb, q, c0, g, t);
-      *reinterpret_cast<double2*>(xb + (r + g) * P + q + 2 * t) = d;
+    panel_to_frag(c, x, p, pan);
+    // trailing update of this warp's column blocks cb > p
+    double a[C::MI][2];
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) {
+      const double* pr = pan + (wm * C::WM + mi * 8 + g) * kPanelPitch;
+      a[mi][0] = -pr[t];
+      a[mi][1] = -pr[t + 4];
     }
-    bar_sync(kBarCompute, kComputeThreads);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int cb = wn * C::NI + ni;
+      if (cb <= p) continue;
+      const double* lr = lb + (cb * 8 + g) * P + c0;
+      const double b0 = lr[t], b1 = lr[t + 4];
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi) {
+        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][0], b0);
+        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][1], b1);
+      }
+    }
   }
-  // write the solved block back (coalesced rows)
-  for (int idx = tid; idx < BS * (BS / 2); idx += kComputeThreads) {
-    const int r = idx / (BS / 2), cc = 2 * (idx - r * (BS / 2));
-    __stcg(reinterpret_cast<double2*>(X + (int64_t)r * ldx + cc), *reinterpret_cast<const double2*>(xb + r * P + cc));
-  }
-  bar_sync(kBarCompute, kComputeThreads);
+  frag_store(c, x, X, ldx, false);
+  bar_sync(kBarCompute, kComputeThreads);  // buf / lbuf free for the next user
 }
 
-// Cholesky of the BS x BS diagonal block A (ld lda), lower, in shared memory
-// (POTRF, L196-199), blocked right-looking over 8-column panels:
-//   (a) one warp factors the 8x8 diagonal block (column algorithm of SURVEY §8c),
-//   (b) the rows below solve against it (one thread per row),
-//   (c) the trailing lower triangle is updated with FP64 DMMA.
-// A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
-// reading R6).  Compute warps only.
+// Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
+// L196-199).  Register-resident like solve_block: for each 8-column panel, the owner
+// warps copy it to shared memory, warp 0 factors its 8x8 diagonal block in registers
+// (column algorithm of SURVEY §8c, lanes = rows, shuffles), one thread per row
+// solves the rows below, and every warp applies the rank-8 update to its lower
+// blocks with FP64 DMMA.  A pivot !(d > 0) records info = col0 + c + 1 with
+// atomicMin (LAPACK convention, reading R6).  The strictly upper blocks are never
+// stored; the upper halves of diagonal 8x8 blocks are scratch (never read).
 template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   using C = Cfg<BS>;
-  constexpr int P = C::kPitch;
-  const int tid = threadIdx.x, lane = c.lane, g = lane >> 2, t = lane & 3;
-  double* a = c.buf;
-  bar_sync(kBarCompute, kComputeThreads);  // buf aliases the TMA ring
-  for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
-    const int r = idx / BS, cc = idx - r * BS;
-    if (cc <= r) a[r * P + cc] = __ldcg(A + (int64_t)r * lda + cc);
-  }
-  bar_sync(kBarCompute, kComputeThreads);
+  const int tid = threadIdx.x, lane = c.lane, wm = c.warp >> 2, wn = c.warp & 3, g = lane >> 2, t = lane & 3;
+  double* pans = c.buf;
+  double* rdiag = c.lbuf;  // 1/L[c][c] of the current panel (8 doubles)
+  Acc<BS> x;
+  frag_load(c, x, A, lda);
+  bar_sync(kBarCompute, kComputeThreads);  // buf / lbuf reuse
 #pragma unroll 1
-  for (int c0 = 0; c0 < BS; c0 += 8) {
-    // (a) 8x8 diagonal block, warp 0, lane r < 8 owns row c0 + r
-    if (c.warp == 0) {
-#pragma unroll
-      for (int j = 0; j < 8; ++j) {
-        const double d = a[(c0 + j) * P + c0 + j];
-        const double ljj = sqrt(d);
-        if (lane == 0 && !(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
-        __syncwarp();
-        if (lane > j && lane < 8) a[(c0 + lane) * P + c0 + j] = a[(c0 + lane) * P + c0 + j] / ljj;
-        if (lane == j) {
-          a[(c0 + j) * P + c0 + j] = ljj;
-          a[(c0 + j) * P + BS] = 1.0 / ljj;
-        }
-        __syncwarp();
-        if (lane > j && lane < 8) {
-          const double lrj = a[(c0 + lane) * P + c0 + j];
-          for (int q = j + 1; q <= lane; ++q)
-            a[(c0 + lane) * P + c0 + q] = fma(-lrj, a[(c0 + q) * P + c0 + j], a[(c0 + lane) * P + c0 + q]);
-        }
-        __syncwarp();
-      }
-    }
+  for (int p = 0; p < BS / 8; ++p) {
+    const int c0 = 8 * p;
+    double* pan = pans + (p & 1) * BS * kPanelPitch;
+    frag_to_panel(c, x, p, pan);
     bar_sync(kBarCompute, kComputeThreads);
-    const int rows = BS - c0 - 8;
-    if (rows == 0) break;
-    // (b) panel rows below the diagonal block
-    if (tid < rows) {
+    if (c.warp == 0) {  // 8x8 diagonal block in registers: lane r < 8 holds row c0 + r
       double v[8];
-      double* ar = a + (c0 + 8 + tid) * P + c0;
+      double* pr = pan + (c0 + (lane & 7)) * kPanelPitch;
 #pragma unroll
-      for (int j = 0; j < 8; ++j) v[j] = ar[j];
+      for (int j = 0; j < 8; ++j) v[j] = pr[j];
 #pragma unroll
       for (int j = 0; j < 8; ++j) {
-        v[j] *= a[(c0 + j) * P + BS];
+        const double d = __shfl_sync(0xffffffffu, v[j], j);
+        if (lane == 0 && !(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
+        const double ljj = sqrt(d);
+        const double rl = 1.0 / ljj;
+        if (lane == j) v[j] = ljj;
+        if (lane > j) v[j] *= rl;
+        if (lane == 0) rdiag[j] = rl;
 #pragma unroll
-        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], a[(c0 + j2) * P + c0 + j], v[j2]);
+        for (int q = j + 1; q < 8; ++q) {
+          const double lqj = __shfl_sync(0xffffffffu, v[j], q);
+          if (lane >= q) v[q] = fma(-v[j], lqj, v[q]);
+        }
       }
+      if (lane < 8)
 #pragma unroll
-      for (int j = 0; j < 8; ++j) ar[j] = v[j];
+        for (int j = 0; j < 8; ++j) pr[j] = v[j];
     }
     bar_sync(kBarCompute, kComputeThreads);
-    // (c) trailing lower update: A[r][q] -= L[r, panel] L[q, panel]^T, 8x8 blocks nk <= mb
-    const int nr = rows / 8;
-    for (int blk = c.warp; blk < nr * (nr + 1) / 2; blk += kComputeWarps) {
-      int mb = 0, rem = blk;
-      while (rem > mb) {
-        rem -= mb + 1;
-        ++mb;
+    const int r = c0 + 8 + tid;
+    if (r < BS) {  // rows below the diagonal block: L[r, panel] = A[r, panel] L_dd^{-T}
+      double v[8];
+      double* pr = pan + r * kPanelPitch;
+#pragma unroll
+      for (int j = 0; j < 8; j += 2) {
+        const double2 q = *reinterpret_cast<const double2*>(pr + j);
+        v[j] = q.x;
+        v[j + 1] = q.y;
       }
-      const int r = c0 + 8 + mb * 8, q = c0 + 8 + rem * 8;
-      double2 d = *reinterpret_cast<const double2*>(a + (r + g) * P + q + 2 * t);
-      smem_dmma_sub8<P>(d.x, d.y, a, r, c0, a, q, c0, g, t);
-      *reinterpret_cast<double2*>(a + (r + g) * P + q + 2 * t) = d;
+#pragma unroll
+      for (int j = 0; j < 8; ++j) {
+        v[j] *= rdiag[j];
+#pragma unroll
+        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], pan[(c0 + j2) * kPanelPitch + j], v[j2]);
+      }
+#pragma unroll
+      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(pr + j) = make_double2(v[j], v[j + 1]);
     }
     bar_sync(kBarCompute, kComputeThreads);
+    panel_to_frag(c, x, p, pan);
+    // rank-8 update of this warp's lower blocks (rb >= cb > p)
+    double a[C::MI][2];
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) {
+      const double* pr = pan + (wm * C::WM + mi * 8 + g) * kPanelPitch;
+      a[mi][0] = -pr[t];
+      a[mi][1] = -pr[t + 4];
+    }
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int cb = wn * C::NI + ni;
+      if (cb <= p) continue;
+      const double* lr = pan + (cb * 8 + g) * kPanelPitch;
+      const double b0 = lr[t], b1 = lr[t + 4];
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi) {
+        if (wm * C::MI + mi < cb) continue;
+        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][0], b0);
+        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][1], b1);
+      }
+    }
   }
-  for (int idx = tid; idx < BS * BS; idx += kComputeThreads) {
-    const int r = idx / BS, cc = idx - r * BS;
-    if (cc <= r) __stcg(A + (int64_t)r * lda + cc, a[r * P + cc]);
-  }
+  frag_store(c, x, A, lda, true);
+  bar_sync(kBarCompute, kComputeThreads);
 }
 
 // ------------------------------------------------------------------ sub-tasks
