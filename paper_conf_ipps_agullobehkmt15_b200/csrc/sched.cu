@@ -99,103 +99,238 @@ __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, i
   return -1;
 }
 
-// One non-inlined function per job type: each gets its own register allocation
-// (inlining all of them into the persistent kernel made ptxas spill the GEMM
-// accumulators to local memory).
-template <int BS>
-__device__ __noinline__ void job_update(Ctx<BS>& c, int i, int j, int k, int bm, int bn) {
-  sub_update(c, i, j, k, bm, bn);
+// ------------------------------------------------------------------ warp-specialised worker
+// CTA = 12 warps: warps 0-7 compute (setmaxnreg 232), warp 8 = TMA producer,
+// warp 9 = scheduler, warps 10-11 idle (control warpgroup, setmaxnreg 40).
+// The scheduler pops the next job while the current one computes and does the
+// completion bookkeeping off the compute warps; the producer walks the same job
+// sequence through a 2-deep shared-memory job ring and issues every TMA load,
+// running ahead into the next job as soon as ring stages free up.
+constexpr int kWsThreads = 384;
+constexpr int kProdWarp = 8, kSchedWarp = 9;
+constexpr int kRegsCompute = 232, kRegsControl = 40;
+
+__device__ __forceinline__ void write_desc(int4* slot, int job, const Job& jb, int skip) {
+  slot[0] = make_int4(job, (int)jb.type | (skip << 8), jb.i, jb.j);
+  slot[1] = make_int4(jb.k, jb.a, jb.b, jb.c);
 }
+
+// ---- producer (one lane): issue the stages of a job, in the order the compute warps consume them
 template <int BS>
-__device__ __noinline__ void job_trsm(Ctx<BS>& c, int i, int k, int slab) {
-  sub_trsm(c, i, k, slab);
-}
-template <int BS>
-__device__ __noinline__ void job_potrf_diag(Ctx<BS>& c, int k, int b, int* info) {
-  sub_potrf_diag(c, k, b, info);
-}
-template <int BS>
-__device__ __noinline__ void job_potrf_panel(Ctx<BS>& c, int k, int b, int r) {
-  sub_potrf_panel(c, k, b, r);
-}
-template <int BS>
-__device__ __noinline__ void job_potrf_update(Ctx<BS>& c, int k, int b, int r, int q) {
-  sub_potrf_update(c, k, b, r, q);
+__device__ __forceinline__ void produce_range(Ctx<BS>& c, uint32_t& pit, int nst, int64_t ta, int ra, int64_t tb,
+                                              int rb, int kbeg, int from, int to) {
+  for (int s = from; s < to && s < nst; ++s) issue_stage(c, pit + s, ta, ra, tb, rb, kbeg + s * BK);
 }
 
 template <int BS>
-__device__ __forceinline__ void run_job(Ctx<BS>& c, const Job& jb, int* info) {
-  switch (jb.type) {
-    case J_UPD: job_update(c, jb.i, jb.j, jb.k, jb.a, jb.b); break;
-    case J_TRSM: job_trsm(c, jb.i, jb.k, jb.a); break;
-    case J_DIAG: job_potrf_diag(c, jb.k, jb.a, info); break;
-    case J_PANEL: job_potrf_panel(c, jb.k, jb.a, jb.b); break;
-    case J_PUPD: job_potrf_update(c, jb.k, jb.a, jb.b, jb.c); break;
+__device__ void producer_loop(Ctx<BS>& c) {
+  uint32_t q = 0, pit = 0, tcount = 0;
+  while (true) {
+    const int e = q & 1;
+    mbar_wait(&c.jfull[e], (q >> 1) & 1);
+    const int4 d0 = c.jdesc[e * 3], d1 = c.jdesc[e * 3 + 1];
+    const int job = d0.x, type = d0.y & 0xff, skip = d0.y >> 8;
+    if (job < 0) break;
+    fence_proxy_async();  // operands written by generic stores (this or other SMs)
+    if (!skip) {
+      if (type == J_UPD || type == J_PUPD) {
+        int64_t ta, tb, tcb;
+        int ra, rb, kb, nst, cr, cc;
+        if (type == J_UPD) {  // GEMM/SYRK block (i, j, k, bm, bn)
+          ta = tile_index(d0.z, d1.x); ra = d1.y * BS;
+          tb = tile_index(d0.w, d1.x); rb = d1.z * BS;
+          kb = 0; nst = c.nb / BK;
+          tcb = tile_index(d0.z, d0.w); cr = d1.y * BS; cc = d1.z * BS;
+        } else {              // POTRF update block (k, b, r, q)
+          ta = tb = tcb = tile_index(d1.x, d1.x);
+          ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
+          cr = ra; cc = rb;
+        }
+        // stages first (they only need ring space), then the C prefetch into lbuf once
+        // the previous job has released lbuf, then the rest
+        produce_range(c, pit, nst, ta, ra, tb, rb, kb, 0, kStages);
+        if (q > 0) mbar_wait(c.lfree, (q - 1) & 1);
+        prefetch_c_issue(c, tcb, cr, cc);
+        produce_range(c, pit, nst, ta, ra, tb, rb, kb, kStages, nst);
+        pit += nst;
+      } else if (type == J_TRSM) {  // row slab (i, k, slab): mainloop cb reads X[:, :cb] (solved)
+        const int nbb = c.nb / BS;
+        for (int cb = 1; cb < nbb; ++cb) {
+          mbar_wait(c.tstep, tcount & 1);
+          ++tcount;
+          fence_proxy_async();
+          const int nst = cb * BS / BK;
+          produce_range(c, pit, nst, tile_index(d0.z, d1.x), d1.y * BS, tile_index(d1.x, d1.x), cb * BS, 0, 0, nst);
+          pit += nst;
+        }
+      }
+    }
+    ++q;
+  }
+}
+
+// ---- compute warps: run the job's consumer side
+template <int BS>
+__device__ __forceinline__ void compute_job(Ctx<BS>& c, int type, const int4& d0, const int4& d1, int* info) {
+  Acc<BS> acc;
+  if (type == J_UPD) {
+    const int i = d0.z, j = d0.w, k = d1.x, bm = d1.y, bn = d1.z;
+    gemm_consume(c, c.nb / BK, acc);
+    epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
+    (void)k;
+  } else if (type == J_PUPD) {
+    const int k = d1.x, r = d1.z, q = d1.w;
+    gemm_consume(c, BS / BK, acc);
+    epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);
+  } else if (type == J_TRSM) {
+    const int i = d0.z, k = d1.x, slab = d1.y, nbb = c.nb / BS;
+    double* X = c.tile(i, k) + (int64_t)slab * BS * c.nb;
+    const double* L = c.tile(k, k);
+    for (int cb = 0; cb < nbb; ++cb) {
+      if (cb > 0) gemm_consume(c, cb * BS / BK, acc);
+      solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+      if (cb + 1 < nbb) {
+        // X[:, cb] is read by the producer's TMA for the next column block
+        __threadfence();
+        fence_proxy_async();
+        __syncwarp();
+        if (c.lane == 0) mbar_arrive(c.tstep);
+      }
+    }
+  } else if (type == J_DIAG) {
+    sub_potrf_diag(c, d1.x, d1.y, info);
+  } else if (type == J_PANEL) {
+    sub_potrf_panel(c, d1.x, d1.y, d1.z);
   }
 }
 
 template <int BS>
-__global__ void __launch_bounds__(kThreads, 1) k_sched(const __grid_constant__ CUtensorMap map, StepParams sp,
-                                                       DevSched d) {
-  __shared__ int s_job, s_skip;
-  __shared__ uint64_t s_t0;
+__device__ void compute_loop(Ctx<BS>& c, int* info) {
+  uint32_t q = 0;
+  while (true) {
+    const int e = q & 1;
+    mbar_wait(&c.jfull[e], (q >> 1) & 1);
+    const int4 d0 = c.jdesc[e * 3], d1 = c.jdesc[e * 3 + 1];
+    if (d0.x < 0) break;
+    if (c.warp == 0 && c.lane == 0) {
+      const unsigned long long t0 = globaltimer_ns();
+      c.jdesc[e * 3 + 2] = make_int4((int)(t0 & 0xffffffffull), (int)(t0 >> 32), 0, 0);
+    }
+    const int type = d0.y & 0xff, skip = d0.y >> 8;
+    if (!skip) compute_job(c, type, d0, d1, info);
+    __syncwarp();
+    if (c.lane == 0) {
+      mbar_arrive(c.lfree);  // lbuf (C block / L block / rdiag) no longer needed
+      if (c.warp == 0) {     // end time of the job as seen by warp 0
+        const unsigned long long t1 = globaltimer_ns();
+        c.jdesc[e * 3 + 2].z = (int)(t1 & 0xffffffffull);
+        c.jdesc[e * 3 + 2].w = (int)(t1 >> 32);
+      }
+      mbar_arrive(&c.jdone[e]);  // the job's global stores precede this release
+    }
+    ++q;
+  }
+}
+
+// ---- scheduler warp
+__device__ __forceinline__ void complete_job(const DevSched& d, const StepParams& sp, int job, uint64_t t0_abs,
+                                             uint64_t t1_abs) {
+  __threadfence();  // the compute warps' stores (acquired through jdone) before the counters
+  const int node = d.job_node[job];
+  if (sp.tr_t0) {
+    const uint64_t base = *sp.tr_base;
+    const uint64_t t0 = t0_abs - base, t_end = t1_abs - base;
+    const int pt = d.node_paper[node];
+    atomicMin(reinterpret_cast<unsigned long long*>(sp.tr_t0 + pt), (unsigned long long)t0);
+    atomicMax(reinterpret_cast<unsigned long long*>(sp.tr_t1 + pt), (unsigned long long)((t_end << 16) | smid()));
+    if (d.job_trace) {
+      d.job_trace[3 * (size_t)job] = t0;
+      d.job_trace[3 * (size_t)job + 1] = t_end;
+      d.job_trace[3 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
+    }
+  }
+  if (atomicSub(&d.node_left[node], 1) == 1) {
+    __threadfence();
+    for (int e = d.succ_off[node]; e < d.succ_off[node + 1]; ++e) {
+      const int s = d.succ[e];
+      if (atomicSub(&d.node_deps[s], 1) == 1) push_node(d, s);
+    }
+    if (atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
+      __threadfence();
+      atomicExch(d.finished, 1);
+    }
+  }
+}
+
+template <int BS>
+__device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& sp, bool latency_worker) {
+  const int lane = c.lane;
+  uint32_t q_issue = 0, q_done = 0;
+  int pending[2] = {-1, -1};
+  unsigned backoff = 32;
+  while (true) {
+    // 1. retire finished jobs in order
+    while (q_done < q_issue) {
+      const int e = q_done & 1;
+      if (!mbar_try_wait(smem_u32(&c.jdone[e]), (q_done >> 1) & 1)) break;
+      if (lane == 0) {
+        const int4 tt = c.jdesc[e * 3 + 2];
+        const uint64_t t0 = (uint64_t)(uint32_t)tt.x | ((uint64_t)(uint32_t)tt.y << 32);
+        const uint64_t t1 = (uint64_t)(uint32_t)tt.z | ((uint64_t)(uint32_t)tt.w << 32);
+        complete_job(d, sp, pending[e], t0, t1);
+      }
+      __syncwarp();
+      ++q_done;
+    }
+    // 2. keep the 2-deep job ring full
+    if (q_issue - q_done < 2) {
+      const int job = try_pop(d, latency_worker, lane);
+      if (job >= 0) {
+        const int e = q_issue & 1;
+        if (lane == 0) {
+          __threadfence();  // acquire: the job's inputs were published before it was enqueued
+          const Job jb = d.jobs[job];
+          write_desc(&c.jdesc[e * 3], job, jb, ld_volatile(sp.info) != INT_MAX);
+          mbar_arrive(&c.jfull[e]);
+        }
+        __syncwarp();
+        pending[e] = job;
+        ++q_issue;
+        backoff = 32;
+        continue;
+      }
+    }
+    // 3. done?
+    if (q_done == q_issue && ld_volatile(d.finished)) {
+      if (lane == 0) {
+        const int e = q_issue & 1;
+        c.jdesc[e * 3] = make_int4(-1, 0, 0, 0);
+        mbar_arrive(&c.jfull[e]);
+      }
+      __syncwarp();
+      break;
+    }
+    __nanosleep(backoff);
+    backoff = backoff < 512 ? backoff * 2 : 512;
+  }
+}
+
+template <int BS>
+__global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__ CUtensorMap map, StepParams sp,
+                                                         DevSched d) {
   auto c = make_ctx<BS>(&map, sp.tiles, sp.nb, sp.N);
   const bool latency_worker = d.policy == 2 && (int)blockIdx.x < d.latency_workers;
-  const int tid = threadIdx.x;
-  while (true) {
-    if (c.warp == 0) {
-      int job = -1;
-      unsigned backoff = 32;
-      while (true) {
-        job = try_pop(d, latency_worker, c.lane);
-        if (job >= 0) break;
-        if (ld_volatile(d.finished)) break;
-        __nanosleep(backoff);
-        backoff = backoff < 1024 ? backoff * 2 : 1024;
-      }
-      if (c.lane == 0) {
-        __threadfence();  // acquire: the job's inputs were published before it was enqueued
-        s_job = job;
-        s_skip = ld_volatile(sp.info) != INT_MAX;
-        s_t0 = sp.tr_base ? globaltimer_ns() - *sp.tr_base : 0;
-      }
+  if (c.warp >= kComputeWarps) {
+    asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(kRegsControl));
+    if (c.warp == kProdWarp) {
+      if (c.lane == 0) producer_loop(c);
+    } else if (c.warp == kSchedWarp) {
+      scheduler_loop(c, d, sp, latency_worker);
     }
-    __syncthreads();
-    const int job = s_job;
-    if (job < 0) break;
-    const Job jb = d.jobs[job];
-    if (!s_skip) run_job(c, jb, sp.info);
-    __threadfence();      // this job's global writes are complete at L2 ...
-    fence_proxy_async();  // ... and ordered before later async-proxy (TMA) accesses
-    __syncthreads();
-    if (tid == 0) {
-      __threadfence();  // release this job's global writes
-      const int node = d.job_node[job];
-      if (sp.tr_t0) {
-        const uint64_t t_end = globaltimer_ns() - *sp.tr_base;
-        if (d.job_trace) {
-          d.job_trace[3 * (size_t)job] = s_t0;
-          d.job_trace[3 * (size_t)job + 1] = t_end;
-          d.job_trace[3 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
-        }
-        const int pt = d.node_paper[node];
-        atomicMin(reinterpret_cast<unsigned long long*>(sp.tr_t0 + pt), (unsigned long long)s_t0);
-        atomicMax(reinterpret_cast<unsigned long long*>(sp.tr_t1 + pt),
-                  (unsigned long long)((t_end << 16) | smid()));
-      }
-      if (atomicSub(&d.node_left[node], 1) == 1) {
-        __threadfence();
-        for (int e = d.succ_off[node]; e < d.succ_off[node + 1]; ++e) {
-          const int s = d.succ[e];
-          if (atomicSub(&d.node_deps[s], 1) == 1) push_node(d, s);
-        }
-        if (atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
-          __threadfence();
-          atomicExch(d.finished, 1);
-        }
-      }
-    }
+    return;
   }
+  asm volatile("setmaxnreg.inc.sync.aligned.u32 %0;\n" ::"n"(kRegsCompute));
+  compute_loop(c, sp.info);
 }
 
 __global__ void k_sched_init(DevSched d, const int* roots, int nroots) {
@@ -458,11 +593,11 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   cudaError_t ea = cudaSuccess;
   switch (bs) {
     case 96: ea = cudaFuncSetAttribute(k_sched<96>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<96>, kThreads, smem); break;
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<96>, kWsThreads, smem); break;
     case 64: ea = cudaFuncSetAttribute(k_sched<64>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<64>, kThreads, smem); break;
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<64>, kWsThreads, smem); break;
     case 32: ea = cudaFuncSetAttribute(k_sched<32>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<32>, kThreads, smem); break;
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<32>, kWsThreads, smem); break;
   }
   if (ea || per_sm < 1) {
     sched_destroy(st);
@@ -485,9 +620,9 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
   k_sched_init<<<1, 1, 0, s>>>(st->d, st->roots, st->nroots);
   const int smem = smem_bytes(st->bs);
   switch (st->bs) {
-    case 96: k_sched<96><<<st->workers, kThreads, smem, s>>>(map, base, st->d); break;
-    case 64: k_sched<64><<<st->workers, kThreads, smem, s>>>(map, base, st->d); break;
-    case 32: k_sched<32><<<st->workers, kThreads, smem, s>>>(map, base, st->d); break;
+    case 96: k_sched<96><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;
+    case 64: k_sched<64><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;
+    case 32: k_sched<32><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;
   }
   *nlaunch += 2;
   if ((e = cudaGetLastError())) return -100 - (int)e;

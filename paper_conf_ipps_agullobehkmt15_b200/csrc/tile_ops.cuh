@@ -35,7 +35,9 @@ struct Cfg {
   static constexpr int kPipeBytes = kStages * 2 * kOpBytes;
   static constexpr int kPitch = BS + 2;            // doubles; keeps double2 alignment
   static constexpr int kBufBytes = BS * kPitch * 8;
-  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + (2 * kStages + 2) * 8 + 1024;
+  static constexpr int kPanBytes = 2 * BS * 10 * 8;  // two BS x 8 panels (pitch 10)
+  static constexpr int kBarBytes = 256;               // mbarriers + job ring descriptors
+  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kPanBytes + kBarBytes + 1024;
   static_assert(kBufBytes >= BS * BS * 8, "lbuf holds a TMA-prefetched BS x BS C block");
   static constexpr int RW = BS / kComputeWarps;    // rows per warp in the solves
   static constexpr int CPL = BS / 32;              // columns per lane in the solves
@@ -56,6 +58,13 @@ struct Ctx {
   uint64_t* full;  // kStages
   uint64_t* empty; // kStages
   uint64_t* cbar;  // C-block prefetch (TMA -> lbuf)
+  // warp-specialised persistent kernel only (sched.cu):
+  uint64_t* jfull; // [2] job descriptor ready (scheduler -> producer, compute)
+  uint64_t* jdone; // [2] job finished (compute -> scheduler)
+  uint64_t* lfree; // lbuf released by the current job (compute -> producer)
+  uint64_t* tstep; // TRSM column block solved and stored (compute -> producer)
+  int4* jdesc;     // [2] x 3 int4 job descriptors
+  double* pans;    // two BS x 8 panels for the in-block solves
   uint32_t it;     // stages consumed so far
   uint32_t cphase; // parity of the next cbar completion
   int warp, lane;
@@ -77,9 +86,16 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
   c.pipe = base;
   c.buf = reinterpret_cast<double*>(base);
   c.lbuf = reinterpret_cast<double*>(base + C::kPipeBytes);
-  c.full = reinterpret_cast<uint64_t*>(base + C::kPipeBytes + C::kBufBytes);
+  c.pans = reinterpret_cast<double*>(base + C::kPipeBytes + C::kBufBytes);
+  char* bars = base + C::kPipeBytes + C::kBufBytes + C::kPanBytes;  // kBarBytes
+  c.full = reinterpret_cast<uint64_t*>(bars);
   c.empty = c.full + kStages;
   c.cbar = c.empty + kStages;
+  c.jfull = c.cbar + 1;
+  c.jdone = c.jfull + 2;
+  c.lfree = c.jdone + 2;
+  c.tstep = c.lfree + 1;  // 2*kStages + 7 = 17 barriers = 136 bytes
+  c.jdesc = reinterpret_cast<int4*>(bars + 160);  // 2 x 3 int4
   c.it = 0;
   c.cphase = 0;
   c.warp = threadIdx.x >> 5;
@@ -90,6 +106,12 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
       mbar_init(&c.empty[s], kComputeWarps);
     }
     mbar_init(c.cbar, 1);
+    for (int e = 0; e < 2; ++e) {
+      mbar_init(&c.jfull[e], 1);
+      mbar_init(&c.jdone[e], kComputeWarps);
+    }
+    mbar_init(c.lfree, kComputeWarps);
+    mbar_init(c.tstep, kComputeWarps);
     fence_mbar_init();
   }
   if (c.issuer() && map) tma_prefetch_desc(map);
@@ -113,13 +135,17 @@ struct CPrefetch {
 };
 
 template <int BS>
-__device__ __forceinline__ void prefetch_c(Ctx<BS>& c, int64_t tile, int r0, int c0) {
-  if (!c.issuer()) return;
+__device__ __forceinline__ void prefetch_c_issue(Ctx<BS>& c, int64_t tile, int r0, int c0) {
   fence_proxy_async();
   mbar_arrive_expect_tx(c.cbar, BS * BS * 8);
   char* dst = reinterpret_cast<char*>(c.lbuf);
 #pragma unroll 1
   for (int b = 0; b < BS / 16; ++b) tma_load_3d(dst + b * BS * 128, c.map, c.cbar, c0 + 16 * b, r0, (int)tile);
+}
+
+template <int BS>
+__device__ __forceinline__ void prefetch_c(Ctx<BS>& c, int64_t tile, int r0, int c0) {
+  if (c.issuer()) prefetch_c_issue(c, tile, r0, c0);
 }
 
 template <int BS>
@@ -133,10 +159,70 @@ __device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, 
   tma_load_3d(sa + C::kOpBytes, c.map, &c.full[st], kk, rb, (int)tb);
 }
 
+// Consume one TMA stage: wait for it, DMMA it into acc, release it to the producer.
+template <int BS>
+__device__ __forceinline__ void consume_stage(Ctx<BS>& c, uint32_t q, Acc<BS>& acc, uint32_t rt_zero) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  const uint32_t st = q % kStages, ph = (q / kStages) & 1;
+  mbar_wait(&c.full[st], ph);
+  const uint32_t As = smem_u32(c.pipe) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
+  const uint32_t Bs = smem_u32(c.pipe) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
+  uint32_t dep = 0;
+#pragma unroll
+  for (int h = 0; h < 2; ++h) {
+    // Thread (g, t) reads logical 16-byte chunk 2t + h of its row (k = 4t + 2h, +1):
+    // with the 128B swizzle (chunk ^= row & 7) the two rows g, g+1 of one 8-lane
+    // phase land on chunks of opposite parity -> conflict-free LDS.128.
+    const int chunk = ((2 * t + h) ^ g) << 4;
+    double2 af[C::MI], bf[C::NI];
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) af[mi] = lds128(As + mi * 8 * 128 + chunk);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) bf[ni] = lds128(Bs + ni * 8 * 128 + chunk);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(af[mi].x);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(bf[ni].x);
+    // k-permutation: thread t holds k = 4t+2h (x) and 4t+2h+1 (y) for both operands.
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].x, bf[ni].x);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].y, bf[ni].y);
+  }
+  // Release the stage only once every ld.shared of it has returned: the arrive is
+  // predicated on a value derived from all loaded registers (lane 0 arrives), so it
+  // cannot issue before the loads complete and a TMA refill can never overwrite
+  // data a lane has not read yet.
+  __syncwarp();
+  if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty[st]);
+}
+
+template <int BS>
+__device__ __forceinline__ void zero_acc(Acc<BS>& acc) {
+#pragma unroll
+  for (int mi = 0; mi < Cfg<BS>::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < Cfg<BS>::NI; ++ni) acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
+}
+
+// Consumer side only (warp-specialised kernel: a separate producer issues the stages).
+template <int BS>
+__device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) {
+  zero_acc<BS>(acc);
+  const uint32_t rt_zero = threadIdx.y;  // 0, unknown to the compiler (see consume_stage)
+  for (int s = 0; s < nst; ++s) consume_stage(c, c.it + s, acc, rt_zero);
+  c.it += nst;
+}
+
+// Issue + consume (all-compute CTA, thread 0 issues kStages-1 stages ahead).
 template <int BS>
 __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, int64_t tb, int rb, int kbeg,
                                               int kend, Acc<BS>& acc, const CPrefetch* cpre = nullptr) {
-  using C = Cfg<BS>;
   const int nst = (kend - kbeg) / BK;
   if (c.issuer()) {
     fence_proxy_async();  // operands may have been written by generic stores (this or other SMs)
@@ -144,61 +230,17 @@ __device__ __forceinline__ void gemm_mainloop(Ctx<BS>& c, int64_t ta, int ra, in
     for (int s = 0; s < pre; ++s) issue_stage(c, c.it + s, ta, ra, tb, rb, kbeg + s * BK);
     if (cpre) prefetch_c(c, cpre->tile, cpre->r0, cpre->c0);
   }
-#pragma unroll
-  for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
-  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
-  // threadIdx.y is 0 (1-D blocks) but unknown to the compiler: used to make the
-  // stage release depend on every shared load of the stage (see below).
+  zero_acc<BS>(acc);
   const uint32_t rt_zero = threadIdx.y;
   for (int s = 0; s < nst; ++s) {
     // keep kStages-1 stages in flight: refill the buffer stage s-1 used
     if (c.issuer() && s + kStages - 1 < nst)
       issue_stage(c, c.it + s + kStages - 1, ta, ra, tb, rb, kbeg + (s + kStages - 1) * BK);
-    const uint32_t q = c.it + s, st = q % kStages, ph = (q / kStages) & 1;
-    mbar_wait(&c.full[st], ph);
-    const uint32_t As = smem_u32(c.pipe) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
-    const uint32_t Bs = smem_u32(c.pipe) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
-    uint32_t dep = 0;
-#pragma unroll
-    for (int h = 0; h < 2; ++h) {
-      // Thread (g, t) reads logical 16-byte chunk 2t + h of its row (k = 4t + 2h, +1):
-      // with the 128B swizzle (chunk ^= row & 7) the two rows g, g+1 of one 8-lane
-      // phase land on chunks of opposite parity -> conflict-free LDS.128.
-      const int chunk = ((2 * t + h) ^ g) << 4;
-      double2 af[C::MI], bf[C::NI];
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) af[mi] = lds128(As + mi * 8 * 128 + chunk);
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) bf[ni] = lds128(Bs + ni * 8 * 128 + chunk);
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(af[mi].x);
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(bf[ni].x);
-      // k-permutation: thread t holds k = 4t+2h (x) and 4t+2h+1 (y) for both operands.
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-        for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].x, bf[ni].x);
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-        for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], af[mi].y, bf[ni].y);
-    }
-    // Release the stage only once every ld.shared of it has returned: the arrive is
-    // predicated on a value derived from all loaded registers (lane 0 arrives), so it
-    // cannot issue before the loads complete and a TMA refill can never overwrite
-    // data a lane has not read yet.
-    __syncwarp();
-    if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty[st]);
+    consume_stage(c, c.it + s, acc, rt_zero);
   }
   c.it += nst;
 }
 
-// Prefetch the BS x BS block (rows r0.., cols c0..) of store tile `tile` into lbuf with
-// TMA (BS/16 boxes of BS rows x 128 B, 128B-swizzled), completing on cbar.  Issued by
-// thread 0 at the start of a job so the C read of the epilogue overlaps the mainloop.
 // C[0:BS, 0:BS] -= acc for the BS x BS block at Cblk (leading dimension ldc); the old
 // C values come from the lbuf prefetch (prefetch_c), results go to global memory.
 // lower_only: diagonal block of a diagonal tile -- only r >= c is written (SYRK, L207-208).
@@ -334,24 +376,27 @@ __device__ __forceinline__ void panel_to_frag(const Ctx<BS>& c, Acc<BS>& x, int 
 // in the accumulator fragments; for each panel the owner warps copy it to a shared
 // panel buffer, one thread per row solves it against the 8x8 diagonal block of L,
 // and every warp updates its trailing column blocks with FP64 DMMA
-// (X[:, later] -= X[:, panel] L[later, panel]^T).  has_acc = false: X alone.
+// (X[:, later] -= X[:, panel] L[later, panel]^T).  On entry x holds acc (has_acc) or
+// scratch; it is overwritten with the solved block.
 template <int BS>
-__device__ __forceinline__ void solve_block(const Ctx<BS>& c, const Acc<BS>& acc, bool has_acc, double* X, int ldx,
+__device__ __forceinline__ void solve_block(const Ctx<BS>& c, Acc<BS>& x, bool has_acc, double* X, int ldx,
                                             const double* Ld, int ldl) {
   using C = Cfg<BS>;
   constexpr int P = C::kPitch;
   const int tid = threadIdx.x, wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
   double* lb = c.lbuf;  // L block; column BS holds 1/L[c][c]
-  double* pans = c.buf; // 2 panels of BS x kPanelPitch (the TMA ring is idle here)
-  Acc<BS> x;
-  frag_load(c, x, X, ldx);
-  if (has_acc) {
+  double* pans = c.pans; // 2 panels of BS x kPanelPitch
+  // x := X - acc in place (acc is consumed; one 72-register array live)
+  {
+    const int wm0 = wm * C::WM, wn0 = wn * C::WN;
 #pragma unroll
     for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) {
-        x[mi][ni][0] -= acc[mi][ni][0];
-        x[mi][ni][1] -= acc[mi][ni][1];
+        const double2 v = __ldcg(reinterpret_cast<const double2*>(X + (int64_t)(wm0 + mi * 8 + g) * ldx + wn0 +
+                                                                  ni * 8 + 2 * t));
+        x[mi][ni][0] = has_acc ? v.x - x[mi][ni][0] : v.x;
+        x[mi][ni][1] = has_acc ? v.y - x[mi][ni][1] : v.y;
       }
   }
   // buf/lbuf reuse: every warp must be done with the TMA ring and the previous lbuf use.
@@ -421,7 +466,7 @@ template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   using C = Cfg<BS>;
   const int tid = threadIdx.x, lane = c.lane, wm = c.warp >> 2, wn = c.warp & 3, g = lane >> 2, t = lane & 3;
-  double* pans = c.buf;
+  double* pans = c.pans;
   double* rdiag = c.lbuf;  // 1/L[c][c] of the current panel (8 doubles)
   Acc<BS> x;
   frag_load(c, x, A, lda);
