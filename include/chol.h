@@ -110,10 +110,12 @@ int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* L, int64_t 
 int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int64_t* nrecs, double* makespan_s);
 
 /* Per-job (CTA sub-task) trace of the last factorization by the persistent
- * scheduler (requires opts.trace = 2): per job j, out[4j] = t0_ns, out[4j+1] =
- * t1_ns (as chol_trace), out[4j+2] = worker << 32 | SM id, out[4j+3] = job type
+ * scheduler (requires opts.trace = 2): per job j, out[5j] = t0_ns, out[5j+1] =
+ * t1_ns (as chol_trace), out[5j+2] = worker << 32 | SM id, out[5j+4] = time the
+ * job was enqueued (its node became ready), out[5j+3] = job type
  * << 32 | dense task id (job types: 0 SYRK/GEMM block, 1 TRSM row slab, 2 POTRF
- * diagonal block, 3 POTRF panel block, 4 POTRF update block).  At most cap jobs;
+ * diagonal block, 3 POTRF panel block, 4 POTRF update block, 5 TRSM block solve,
+ * 6 TRSM block update).  At most cap jobs;
  * *njobs = number of jobs.  -7 if not available. */
 int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t* njobs);
 

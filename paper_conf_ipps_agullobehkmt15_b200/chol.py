@@ -138,11 +138,11 @@ def chol_trace(plan: int):
 
 
 def chol_job_trace(plan: int):
-    """numpy array (njobs, 4): t0_ns, t1_ns, worker << 32 | smid, type << 32 | task id."""
+    """numpy array (njobs, 5): t0_ns, t1_ns, worker << 32 | smid, type << 32 | task id, t_enqueue_ns."""
     import numpy as np
     n = ctypes.c_int64(0)
     _check(_lib.chol_job_trace(plan, None, 0, ctypes.byref(n)), "chol_job_trace")
-    out = np.zeros((max(n.value, 1), 4), dtype=np.uint64)
+    out = np.zeros((max(n.value, 1), 5), dtype=np.uint64)
     _check(_lib.chol_job_trace(plan, out.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)), n.value,
                                ctypes.byref(n)), "chol_job_trace")
     return out[:n.value]

@@ -429,7 +429,7 @@ extern "C" int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t
   if (!p) return -4;
   if (!p->sched || p->opts.trace != 2 || !p->factored) return -7;
   cudaSetDevice(p->device);
-  return sched_job_trace(p->sched, out, cap, njobs);
+  return sched_job_trace(p->sched, out, cap, njobs);  // 5 u64 per job
 }
 
 // ------------------------------------------------------------------ calibration / single tasks

@@ -17,6 +17,7 @@
 // (the paper's TRSM-distance rule, L1019-1025).
 #include <algorithm>
 #include <climits>
+#include <cstdlib>
 #include <cstring>
 #include <vector>
 
@@ -27,11 +28,15 @@
 
 namespace chol {
 
-constexpr int kBuckets = 16;           // priority buckets per queue class
-constexpr int kQueues = 2 * kBuckets;  // [0, 16) normal, [16, 32) pinned
+constexpr int kBuckets = 64;           // priority buckets per queue class
+constexpr int kQueues = 2 * kBuckets;  // [0, 64) normal, [64, 128) pinned
 constexpr int kQStride = 32;           // ints between queue heads (separate 128B lines)
 
-enum JobType : int16_t { J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4 };
+// Job types: J_UPD GEMM/SYRK block (K = nb); J_TRSM row slab (left-looking, unused by the
+// default plan); POTRF inner: J_DIAG potf2 of block (b,b), J_PANEL solve of block (r,b),
+// J_PUPD K=BS update of block (r,q); TRSM right-looking: J_TS solve of block (s,c) of
+// A_ik against L_kk[c,c], J_TU K=BS update A_ik[s,c'] -= A_ik[s,c] L_kk[c',c]^T.
+enum JobType : int16_t { J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6 };
 struct Job {
   int16_t type, i, j, k, a, b, c, pad;
 };
@@ -47,13 +52,15 @@ struct DevSched {
   const int* succ;
   const int* node_paper;   // paper-level task id (taskid.h) for the trace
   const int* node_queue;   // queue index
-  int* q_items;            // job id + 1 (0 = not yet written)
+  int* q_items;            // node id + 1 (0 = not yet written)
+  int* node_next;          // next job index to hand out within a node
   const int* q_base;       // start of each queue in q_items
   int* q_head;             // kQueues * kQStride
   int* q_tail;             // kQueues * kQStride
   int* done_nodes;
   int* finished;
-  uint64_t* job_trace;     // trace == 2: per job {t0, t1, worker << 32 | smid}
+  uint64_t* job_trace;     // trace == 2: per job {t0, t1, worker << 32 | smid, t_enqueue}
+  const uint64_t* tr_base; // globaltimer at factorization start (trace only)
   int total_nodes;
   int latency_workers;     // STATIC: CTAs [0, latency_workers) serve the pinned queues only
   int policy;
@@ -62,39 +69,50 @@ struct DevSched {
 // ------------------------------------------------------------------ device queue ops
 __device__ __forceinline__ int ld_volatile(const int* p) { return *reinterpret_cast<const volatile int*>(p); }
 
+// A ready node is enqueued ONCE (one queue item per node); workers then claim its jobs
+// one by one with an atomicAdd on the node's job counter (never fails while jobs
+// remain -- a CAS-per-job queue serialised dispatch at one job per L2 round trip).
 __device__ __forceinline__ void push_node(const DevSched& d, int node) {
-  const int q = d.node_queue[node], cnt = d.node_job_count[node], jb = d.node_job_begin[node];
-  const int slot = atomicAdd(&d.q_tail[q * kQStride], cnt);
-  int* items = d.q_items + d.q_base[q] + slot;
-  for (int c = 0; c < cnt; ++c) items[c] = jb + c + 1;
-  __threadfence();
+  const int q = d.node_queue[node];
+  if (d.job_trace) {
+    const uint64_t tq = globaltimer_ns() - *d.tr_base;
+    const int cnt = d.node_job_count[node], jb = d.node_job_begin[node];
+    for (int c = 0; c < cnt; ++c) d.job_trace[4 * (size_t)(jb + c) + 3] = tq;
+  }
+  const int slot = atomicAdd(&d.q_tail[q * kQStride], 1);
+  __threadfence();  // node counters / inputs before the item that publishes the node
+  atomicExch(&d.q_items[d.q_base[q] + slot], node + 1);
 }
 
-// Warp 0 pops one job (lane l inspects queue order[l]); returns job id or -1 if none.
+// One warp pops one job: lanes inspect 32 queues at a time, highest priority first
+// (two passes over the kBuckets buckets of the worker's class); the head node of the
+// best non-empty queue hands out its next job; an exhausted head node is retired by
+// advancing the queue head.  Returns -1 if nothing is ready.
 __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, int lane) {
-  // queue inspected by this lane: highest priority = lowest lane
-  int q;
-  if (d.policy == 2 && latency_worker)
-    q = lane < kBuckets ? kBuckets + (kBuckets - 1 - lane) : -1;  // pinned only
-  else
-    q = lane < kBuckets ? (kBuckets - 1 - lane) : -1;             // normal only
-  for (int attempt = 0; attempt < 8; ++attempt) {
-    int h = 0;
-    bool avail = false;
-    if (q >= 0) {
-      h = ld_volatile(&d.q_head[q * kQStride]);
+  const int cls = (d.policy == 2 && latency_worker) ? kBuckets : 0;  // pinned queues or normal ones
+  for (int pass = 0; pass < kBuckets / 32; ++pass) {
+    const int q = cls + (kBuckets - 1 - (pass * 32 + lane));
+    for (int attempt = 0; attempt < 16; ++attempt) {
+      const int h = ld_volatile(&d.q_head[q * kQStride]);
       const int t = ld_volatile(&d.q_tail[q * kQStride]);
-      avail = h < t && ld_volatile(&d.q_items[d.q_base[q] + h]) != 0;
+      const int item = h < t ? ld_volatile(&d.q_items[d.q_base[q] + h]) : 0;
+      const unsigned m = __ballot_sync(0xffffffffu, item != 0);
+      if (!m) break;
+      const int src = __ffs(m) - 1;
+      int job = -1;
+      if (lane == src) {
+        const int node = item - 1;
+        const int j = atomicAdd(&d.node_next[node], 1);
+        if (j < d.node_job_count[node]) {
+          job = d.node_job_begin[node] + j;
+        } else {
+          atomicCAS(&d.q_head[q * kQStride], h, h + 1);  // node exhausted: retire it
+          job = -2;
+        }
+      }
+      job = __shfl_sync(0xffffffffu, job, src);
+      if (job >= 0) return job;
     }
-    const unsigned m = __ballot_sync(0xffffffffu, avail);
-    if (!m) return -1;
-    const int src = __ffs(m) - 1;
-    int job = -1;
-    if (lane == src) {
-      if (atomicCAS(&d.q_head[q * kQStride], h, h + 1) == h) job = ld_volatile(&d.q_items[d.q_base[q] + h]) - 1;
-    }
-    job = __shfl_sync(0xffffffffu, job, src);
-    if (job >= 0) return job;
   }
   return -1;
 }
@@ -122,9 +140,15 @@ __device__ __forceinline__ void produce_range(Ctx<BS>& c, uint32_t& pit, int nst
   for (int s = from; s < to && s < nst; ++s) issue_stage(c, pit + s, ta, ra, tb, rb, kbeg + s * BK);
 }
 
+// Jobs whose TMA loads the producer has finished issuing (shared memory, read by the
+// scheduler warp): the scheduler claims job q+1 only once job q is fully issued, so a
+// freshly enqueued critical job waits behind at most the tail of a running job.
+__device__ __forceinline__ int* prod_issued_ptr(int4* jdesc) { return reinterpret_cast<int*>(jdesc + 6); }
+
 template <int BS>
 __device__ void producer_loop(Ctx<BS>& c) {
   uint32_t q = 0, pit = 0, tcount = 0;
+  volatile int* issued = prod_issued_ptr(c.jdesc);
   while (true) {
     const int e = q & 1;
     mbar_wait(&c.jfull[e], (q >> 1) & 1);
@@ -133,7 +157,7 @@ __device__ void producer_loop(Ctx<BS>& c) {
     if (job < 0) break;
     fence_proxy_async();  // operands written by generic stores (this or other SMs)
     if (!skip) {
-      if (type == J_UPD || type == J_PUPD) {
+      if (type == J_UPD || type == J_PUPD || type == J_TU) {
         int64_t ta, tb, tcb;
         int ra, rb, kb, nst, cr, cc;
         if (type == J_UPD) {  // GEMM/SYRK block (i, j, k, bm, bn)
@@ -141,8 +165,13 @@ __device__ void producer_loop(Ctx<BS>& c) {
           tb = tile_index(d0.w, d1.x); rb = d1.z * BS;
           kb = 0; nst = c.nb / BK;
           tcb = tile_index(d0.z, d0.w); cr = d1.y * BS; cc = d1.z * BS;
-        } else {              // POTRF update block (k, b, r, q)
+        } else if (type == J_PUPD) {  // POTRF update block (k, b, r, q)
           ta = tb = tcb = tile_index(d1.x, d1.x);
+          ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
+          cr = ra; cc = rb;
+        } else {  // TRSM update (i, k, c, s, c'): A_ik[s, c'] -= A_ik[s, c] L_kk[c', c]^T
+          ta = tcb = tile_index(d0.z, d1.x);
+          tb = tile_index(d1.x, d1.x);
           ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
           cr = ra; cc = rb;
         }
@@ -166,6 +195,7 @@ __device__ void producer_loop(Ctx<BS>& c) {
       }
     }
     ++q;
+    *issued = (int)q;
   }
 }
 
@@ -197,6 +227,14 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, int type, const int4& d0
         if (c.lane == 0) mbar_arrive(c.tstep);
       }
     }
+  } else if (type == J_TU) {
+    const int i = d0.z, k = d1.x, sl = d1.z, c2 = d1.w;
+    gemm_consume(c, BS / BK, acc);
+    epi_sub_global(c, acc, c.tile(i, k) + (int64_t)sl * BS * c.nb + c2 * BS, c.nb, false);
+  } else if (type == J_TS) {
+    const int i = d0.z, k = d1.x, cb = d1.y, sl = d1.z;
+    solve_block(c, acc, false, c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
+                c.tile(k, k) + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
   } else if (type == J_DIAG) {
     sub_potrf_diag(c, d1.x, d1.y, info);
   } else if (type == J_PANEL) {
@@ -244,9 +282,9 @@ __device__ __forceinline__ void complete_job(const DevSched& d, const StepParams
     atomicMin(reinterpret_cast<unsigned long long*>(sp.tr_t0 + pt), (unsigned long long)t0);
     atomicMax(reinterpret_cast<unsigned long long*>(sp.tr_t1 + pt), (unsigned long long)((t_end << 16) | smid()));
     if (d.job_trace) {
-      d.job_trace[3 * (size_t)job] = t0;
-      d.job_trace[3 * (size_t)job + 1] = t_end;
-      d.job_trace[3 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
+      d.job_trace[4 * (size_t)job] = t0;
+      d.job_trace[4 * (size_t)job + 1] = t_end;
+      d.job_trace[4 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
     }
   }
   if (atomicSub(&d.node_left[node], 1) == 1) {
@@ -282,8 +320,9 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
       __syncwarp();
       ++q_done;
     }
-    // 2. keep the 2-deep job ring full
-    if (q_issue - q_done < 2) {
+    // 2. claim the next job once the ring has room and the producer is done with the
+    //    running job's loads (late claim keeps critical-path hops short)
+    if (q_issue - q_done < 2 && (q_issue == q_done || ld_volatile(prod_issued_ptr(c.jdesc)) >= (int)q_issue)) {
       const int job = try_pop(d, latency_worker, lane);
       if (job >= 0) {
         const int e = q_issue & 1;
@@ -399,6 +438,10 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   const int nbb = (int)(nb / bs);
   Builder B{N, nbb, opts->policy, opts->trsm_pin_distance > 0 ? opts->trsm_pin_distance : (int)N};
 
+  // TRSM decomposition: row-slab jobs (default) or right-looking block nodes
+  // (CHOL_TRSM_BLOCKS=1, development switch; measured 2.5% slower at n=19200).
+  const char* ev = getenv("CHOL_TRSM_BLOCKS");
+  const bool trsm_slab = !(ev && ev[0] == '1');
   // ---- nodes and jobs, Algorithm 1 order
   std::vector<int> first_node(n_tasks(N)), last_node(n_tasks(N));
   for (int k = 0; k < N; ++k) {
@@ -426,11 +469,36 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     }
     last_node[pid] = prev;
     for (int i = k + 1; i < N; ++i) {
+      if (trsm_slab) {  // one left-looking row-slab job per BS rows
+        const int tid = (int)id_trsm(N, i, k);
+        const int n = B.add_node(tid, T_TRSM, i, k);
+        for (int sl = 0; sl < nbb; ++sl)
+          B.add_job(n, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
+        first_node[tid] = last_node[tid] = n;
+        continue;
+      }
+      // TRSM_i_k, right-looking over the BS-column blocks c of A_ik (rows independent):
+      //   TS(c): A_ik[:, c] <- A_ik[:, c] L_kk[c,c]^{-T}        (nbb row-block jobs)
+      //   TU(c): A_ik[:, c'] -= A_ik[:, c] L_kk[c',c]^T, c' > c  (nbb x (nbb-1-c) jobs, K = BS)
       const int tid = (int)id_trsm(N, i, k);
-      const int n = B.add_node(tid, T_TRSM, i, k);
-      for (int sl = 0; sl < nbb; ++sl)
-        B.add_job(n, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
-      first_node[tid] = last_node[tid] = n;
+      int prev_t = -1;
+      for (int cb = 0; cb < nbb; ++cb) {
+        const int ts = B.add_node(tid, T_TRSM, i, k);
+        for (int sl = 0; sl < nbb; ++sl)
+          B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+        if (prev_t >= 0) B.edge(prev_t, ts);
+        if (cb == 0) first_node[tid] = ts;
+        prev_t = ts;
+        if (cb + 1 < nbb) {
+          const int tu = B.add_node(tid, T_TRSM, i, k);
+          for (int sl = 0; sl < nbb; ++sl)
+            for (int c2 = cb + 1; c2 < nbb; ++c2)
+              B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
+          B.edge(ts, tu);
+          prev_t = tu;
+        }
+      }
+      last_node[tid] = prev_t;
     }
     for (int j = k + 1; j < N; ++j) {
       const int sid = (int)id_syrk(N, j, k);
@@ -479,7 +547,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
 
   // ---- queue capacities
   std::vector<int> qcap(kQueues, 0), qbase(kQueues, 0);
-  for (int v = 0; v < nnodes; ++v) qcap[node_queue[v]] += B.jcnt[v];
+  for (int v = 0; v < nnodes; ++v) qcap[node_queue[v]] += 1;
   for (int q = 1; q < kQueues; ++q) qbase[q] = qbase[q - 1] + qcap[q - 1];
 
   std::vector<int> succ_off(nnodes + 1, 0), succ;
@@ -532,7 +600,8 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   const size_t d_deps = doff; doff = align(doff + nnodes * 4);
   const size_t d_left = doff; doff = align(doff + nnodes * 4);
   const size_t pristine = doff;  // [0, pristine) is restored from the pristine copy
-  const size_t d_items = doff; doff = align(doff + (size_t)st->njobs * 4);
+  const size_t d_items = doff; doff = align(doff + (size_t)nnodes * 4);
+  const size_t d_next = doff; doff = align(doff + (size_t)nnodes * 4);
   const size_t d_head = doff; doff = align(doff + kQueues * kQStride * 4);
   const size_t d_tail = doff; doff = align(doff + kQueues * kQStride * 4);
   const size_t d_done = doff; doff = align(doff + 4);
@@ -571,13 +640,14 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   d.node_deps = reinterpret_cast<int*>(D + d_deps);
   d.node_left = reinterpret_cast<int*>(D + d_left);
   d.q_items = reinterpret_cast<int*>(D + d_items);
+  d.node_next = reinterpret_cast<int*>(D + d_next);
   d.q_head = reinterpret_cast<int*>(D + d_head);
   d.q_tail = reinterpret_cast<int*>(D + d_tail);
   d.done_nodes = reinterpret_cast<int*>(D + d_done);
   d.finished = reinterpret_cast<int*>(D + d_fin);
   d.total_nodes = nnodes;
   if (opts->trace == 2) {
-    if ((e = cudaMalloc(&st->job_trace, (size_t)st->njobs * 3 * sizeof(uint64_t)))) {
+    if ((e = cudaMalloc(&st->job_trace, (size_t)st->njobs * 4 * sizeof(uint64_t)))) {
       cudaGetLastError();
       sched_destroy(st);
       return -9;
@@ -617,6 +687,9 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
   if ((e = cudaMemsetAsync(static_cast<char*>(st->dev_dynamic) + st->pristine_bytes, 0,
                            st->dyn_bytes - st->pristine_bytes, s)))
     return -100 - (int)e;
+  st->d.tr_base = base.tr_base;
+  if (!base.tr_base) st->d.job_trace = nullptr;  // job trace needs the time base
+  else st->d.job_trace = st->job_trace;
   k_sched_init<<<1, 1, 0, s>>>(st->d, st->roots, st->nroots);
   const int smem = smem_bytes(st->bs);
   switch (st->bs) {
@@ -635,14 +708,15 @@ int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* n
   if (njobs) *njobs = st->njobs;
   if (!st->job_trace) return -7;
   if (!out || cap <= 0) return 0;
-  std::vector<uint64_t> h((size_t)st->njobs * 3);
+  std::vector<uint64_t> h((size_t)st->njobs * 4);
   cudaError_t e = cudaMemcpy(h.data(), st->job_trace, h.size() * 8, cudaMemcpyDeviceToHost);
   if (e) return -100 - (int)e;
   for (int64_t j = 0; j < st->njobs && j < cap; ++j) {
-    out[4 * j] = h[3 * j];
-    out[4 * j + 1] = h[3 * j + 1];
-    out[4 * j + 2] = h[3 * j + 2];
-    out[4 * j + 3] = ((uint64_t)(uint16_t)st->h_job_type[j] << 32) | (uint32_t)st->h_job_paper[j];
+    out[5 * j] = h[4 * j];
+    out[5 * j + 1] = h[4 * j + 1];
+    out[5 * j + 2] = h[4 * j + 2];
+    out[5 * j + 3] = ((uint64_t)(uint16_t)st->h_job_type[j] << 32) | (uint32_t)st->h_job_paper[j];
+    out[5 * j + 4] = h[4 * j + 3];
   }
   return 0;
 }

@@ -95,7 +95,8 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
   c.jdone = c.jfull + 2;
   c.lfree = c.jdone + 2;
   c.tstep = c.lfree + 1;  // 2*kStages + 7 = 17 barriers = 136 bytes
-  c.jdesc = reinterpret_cast<int4*>(bars + 160);  // 2 x 3 int4
+  c.jdesc = reinterpret_cast<int4*>(bars + 160);  // 2 x 3 int4 + producer progress word
+  if (threadIdx.x == 0) *reinterpret_cast<int*>(c.jdesc + 6) = 0;
   c.it = 0;
   c.cphase = 0;
   c.warp = threadIdx.x >> 5;

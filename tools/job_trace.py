@@ -7,7 +7,7 @@ import paper_conf_ipps_agullobehkmt15_b200 as c
 n = int(sys.argv[1]) if len(sys.argv) > 1 else 19200
 pol = int(sys.argv[2]) if len(sys.argv) > 2 else 1
 nb = 960
-JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD"]
+JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU"]
 with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=pol, trace=2) as p:
     for rep in range(2):
         c.chol_generate(p.h, 0, 0)
@@ -22,7 +22,7 @@ span = t1.max() - t0.min()
 busy = (t1 - t0).sum()
 out = {"n": n, "policy": pol, "factor_ms": t_f * 1e3, "span_ms": span / 1e6, "jobs": len(jt), "workers": int(W),
        "utilisation": busy / (W * span)}
-for k in range(5):
+for k in range(7):
     m = typ == k
     if m.any():
         d = (t1[m] - t0[m]) / 1e3
@@ -47,4 +47,29 @@ for i in range(20):
     ov = np.clip(np.minimum(t1, hi) - np.maximum(t0, lo), 0, None).sum()
     util.append(round(float(ov / (W * (hi - lo))), 2))
 out["util_timeline"] = util
+tq = jt[:, 4].astype(np.int64)
+wait = (t0 - tq) / 1e3
+for k in range(7):
+    m = typ == k
+    if m.any():
+        out[JT[k]]["wait_p50_us"] = round(float(np.median(wait[m])), 1)
+        out[JT[k]]["wait_p90_us"] = round(float(np.percentile(wait[m], 90)), 1)
+# queued (ready, not started) jobs over time, sampled at 20 points
+samples = np.linspace(t0.min(), t1.max(), 20)
+out["queued_timeline"] = [int(((tq <= s) & (t0 > s)).sum()) for s in samples]
+out["running_timeline"] = [int(((t0 <= s) & (t1 > s)).sum()) for s in samples]
 print(json.dumps(out))
+# long gaps: what job type preceded / followed, and when (fraction of span)
+rows = []
+for w in range(W):
+    m = np.where(worker == w)[0]
+    o = m[np.argsort(t0[m])]
+    for a, b in zip(o[:-1], o[1:]):
+        g = (t0[b] - t1[a]) / 1e3
+        if g > 20:
+            rows.append((g, JT[typ[a]], JT[typ[b]], round(float((t1[a] - t0.min()) / span), 3), round(float((t0[b] - tq[b]) / 1e3), 1)))
+rows.sort(reverse=True)
+from collections import Counter
+print(json.dumps({"long_gaps": len(rows), "total_long_gap_ms_per_worker": round(sum(r[0] for r in rows) / W / 1e3, 2),
+                  "by_prev_next": Counter((r[1], r[2]) for r in rows).most_common(8),
+                  "examples(gap_us,prev,next,when,next_wait_us)": rows[:12]}))
