@@ -65,8 +65,9 @@ enum {
 /* Options; a zero-initialised struct means "defaults". */
 typedef struct {
   int policy;            /* CHOL_POLICY_* (default DYNAMIC) */
-  int trsm_pin_distance; /* STATIC only: TRSM_i_k with i-k <= d are pinned (0 = N, all) */
-  int latency_workers;   /* STATIC only: CTAs reserved for pinned tasks (0 = 8) */
+  int trsm_pin_distance; /* STATIC only: TRSM_i_k with i-k <= d are pinned (0 = default 1:
+                            the TRSMs on the POTRF-TRSM-SYRK chain) */
+  int latency_workers;   /* STATIC only: CTAs reserved for pinned tasks (0 = default 16) */
   int grid_p, grid_q;    /* 2D block-cyclic process grid (0,0 = 1 x ngpus) */
   int trace;             /* 1 = record per-task t0/t1 (needed by chol_trace);
                             2 = also per-job (CTA sub-task) records (chol_job_trace) */

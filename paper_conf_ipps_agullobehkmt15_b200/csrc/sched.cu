@@ -436,7 +436,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   st->bs = bs;
   st->opts = *opts;
   const int nbb = (int)(nb / bs);
-  Builder B{N, nbb, opts->policy, opts->trsm_pin_distance > 0 ? opts->trsm_pin_distance : (int)N};
+  Builder B{N, nbb, opts->policy, opts->trsm_pin_distance > 0 ? opts->trsm_pin_distance : 1};
 
   // TRSM decomposition: row-slab jobs (default) or right-looking block nodes
   // (CHOL_TRSM_BLOCKS=1, development switch; measured 2.5% slower at n=19200).
@@ -655,7 +655,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   }
   d.job_trace = st->job_trace;
   d.policy = opts->policy;
-  d.latency_workers = opts->policy == CHOL_POLICY_STATIC ? (opts->latency_workers > 0 ? opts->latency_workers : 8) : 0;
+  d.latency_workers = opts->policy == CHOL_POLICY_STATIC ? (opts->latency_workers > 0 ? opts->latency_workers : 16) : 0;
 
   // ---- workers: one CTA per SM (all co-resident)
   int per_sm = 0;
