@@ -51,7 +51,7 @@ def test_trace_respects_dag(n, nb, policy):
     t0 = jt[:, 0].astype(np.int64)
     t1 = jt[:, 1].astype(np.int64)
     w = (jt[:, 2] >> np.uint64(32)).astype(np.int64)
-    assert np.all(t1 >= t0) and np.all(t0 > 0) | (t0 == 0)
+    assert np.all(t1 >= t0)
     for worker in np.unique(w):
         m = np.where(w == worker)[0]
         o = m[np.argsort(t0[m])]
