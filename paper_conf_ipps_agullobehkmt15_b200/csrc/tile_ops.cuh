@@ -487,8 +487,11 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
       for (int j = 0; j < 8; ++j) {
         const double d = __shfl_sync(0xffffffffu, v[j], j);
         if (lane == 0 && !(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
-        const double ljj = sqrt(d);
-        const double rl = 1.0 / ljj;
+        // one rsqrt on the column's dependency chain instead of sqrt followed by a
+        // division: L[j][j] = d * d^{-1/2}, scale = d^{-1/2} (exact for the perfect
+        // squares of the integer family; within an ulp otherwise)
+        const double rl = rsqrt(d);
+        const double ljj = d * rl;
         if (lane == j) v[j] = ljj;
         if (lane > j) v[j] *= rl;
         if (lane == 0) rdiag[j] = rl;

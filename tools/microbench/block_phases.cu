@@ -6,22 +6,24 @@ __device__ long long g_ph[64];
 __device__ long long g_last;
 namespace chol {
 template <int BS>
-__device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, const Acc<BS>& acc, bool has_acc, double* X, int ldx,
+__device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, Acc<BS>& x, bool has_acc, double* X, int ldx,
                                             const double* Ld, int ldl) {
   using C = Cfg<BS>;
   constexpr int P = C::kPitch;
   const int tid = threadIdx.x, wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
   double* lb = c.lbuf;  // L block; column BS holds 1/L[c][c]
-  double* pans = c.buf; // 2 panels of BS x kPanelPitch (the TMA ring is idle here)
-  Acc<BS> x;
-  frag_load(c, x, X, ldx);
-  if (has_acc) {
+  double* pans = c.pans; // 2 panels of BS x kPanelPitch
+  // x := X - acc in place (acc is consumed; one 72-register array live)
+  {
+    const int wm0 = wm * C::WM, wn0 = wn * C::WN;
 #pragma unroll
     for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) {
-        x[mi][ni][0] -= acc[mi][ni][0];
-        x[mi][ni][1] -= acc[mi][ni][1];
+        const double2 v = __ldcg(reinterpret_cast<const double2*>(X + (int64_t)(wm0 + mi * 8 + g) * ldx + wn0 +
+                                                                  ni * 8 + 2 * t));
+        x[mi][ni][0] = has_acc ? v.x - x[mi][ni][0] : v.x;
+        x[mi][ni][1] = has_acc ? v.y - x[mi][ni][1] : v.y;
       }
   }
   // buf/lbuf reuse: every warp must be done with the TMA ring and the previous lbuf use.
@@ -95,7 +97,7 @@ template <int BS>
 __device__ __forceinline__ void potf2_block_T(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   using C = Cfg<BS>;
   const int tid = threadIdx.x, lane = c.lane, wm = c.warp >> 2, wn = c.warp & 3, g = lane >> 2, t = lane & 3;
-  double* pans = c.buf;
+  double* pans = c.pans;
   double* rdiag = c.lbuf;  // 1/L[c][c] of the current panel (8 doubles)
   Acc<BS> x;
   frag_load(c, x, A, lda);
@@ -117,8 +119,11 @@ __device__ __forceinline__ void potf2_block_T(const Ctx<BS>& c, double* A, int l
       for (int j = 0; j < 8; ++j) {
         const double d = __shfl_sync(0xffffffffu, v[j], j);
         if (lane == 0 && !(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
-        const double ljj = sqrt(d);
-        const double rl = 1.0 / ljj;
+        // one rsqrt on the column's dependency chain instead of sqrt followed by a
+        // division: L[j][j] = d * d^{-1/2}, scale = d^{-1/2} (exact for the perfect
+        // squares of the integer family; within an ulp otherwise)
+        const double rl = rsqrt(d);
+        const double ljj = d * rl;
         if (lane == j) v[j] = ljj;
         if (lane > j) v[j] *= rl;
         if (lane == 0) rdiag[j] = rl;
