@@ -160,6 +160,33 @@ int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double
  * (throughput time T_t^thr, reading R9).  Overwrites the store. */
 int chol_run_batch(chol_plan_t p, int type, int count, int reps, double* ms);
 
+/* ---- multi-GPU: one process (or logical rank) per GPU, 2D block-cyclic owner-computes ----
+ * (tile (i,j) lives on rank (i mod p)*q + (j mod q) of the p x q grid,
+ * opts->grid_p x opts->grid_q, default 1 x nranks; every task runs on the owner of the tile
+ * it overwrites).  A rank stores the tiles it owns plus a cache of the remote panel tiles
+ * (L_kk, L_ik) its tasks read; each such tile is pulled once over NVLink by device jobs of
+ * the persistent scheduler as soon as its owner publishes it (no host in the loop).
+ *
+ * chol_plan_dist: plan rank `rank` of `nranks` on the CURRENT device (call cudaSetDevice /
+ *   torch.cuda.set_device first).  opts->executor must be CHOL_EXEC_SCHEDULER.
+ * chol_dist_export: the rank's connection blob (CUDA IPC handles of its tile store and
+ *   publish flags; *len bytes, call with blob = NULL to query the size).
+ * chol_dist_connect: blobs = the nranks blobs concatenated in rank order, `stride` bytes
+ *   apart (the caller exchanges them, e.g. torch.distributed.all_gather_object).  Blobs
+ *   from the same process are used as plain device pointers (logical ranks sharing a
+ *   GPU, each with opts->workers CTAs).  Must precede any factorization.
+ * chol_generate / chol_scatter / chol_factor* / chol_gather then act on the owned tiles;
+ *   *info is this rank's (the global info is the minimum non-zero over ranks).  All
+ *   ranks must run the same sequence of factorizations.
+ * chol_factor_async / chol_wait: launch / complete a factorization (logical ranks in
+ *   one process must all be launched before any wait). */
+int chol_plan_dist(int64_t n, int64_t nb, int nranks, int rank, const chol_opts_t* opts, chol_plan_t* out);
+int chol_dist_export(chol_plan_t p, void* blob, int64_t cap, int64_t* len);
+int chol_dist_connect(chol_plan_t p, const void* blobs, int64_t stride);
+int chol_get_dist(chol_plan_t p, int* rank, int* nranks, int* grid_p, int* grid_q, int64_t* nowned, int64_t* nslots);
+int chol_factor_async(chol_plan_t p);
+int chol_wait(chol_plan_t p, int* info);
+
 /* Number of kernel launches the last chol_factor* issued (the persistent scheduler
  * issues 2: queue init + the scheduler kernel). */
 int chol_last_launches(chol_plan_t p, int* launches);
@@ -171,6 +198,13 @@ int chol_last_launches(chol_plan_t p, int* launches);
  * dependencies (L213-220); edges[2e], edges[2e+1] = (pred, succ) dense task ids
  * (chol_task_id), at most cap edges written (edges may be NULL). */
 int chol_dag(int64_t N, int64_t* ntasks, int64_t* nedges, int64_t* edges, int64_t cap);
+
+/* Multi-GPU layout of rank `rank` on the p x q grid (host only): *nowned tiles owned,
+ * *ncached remote panel tiles received; slot_map[t] (t = i(i+1)/2 + j, at most cap
+ * entries, may be NULL) = local slot of tile t (owned: [0, nowned) in tile order; cached:
+ * [nowned, nowned + ncached) in order of first use), -1 if absent. */
+int chol_dist_layout(int64_t n, int64_t nb, int p, int q, int rank, int* nowned, int* ncached, int32_t* slot_map,
+                     int64_t cap);
 
 /* Dense id of task (type, i, j, k) in chol_dag / chol_trace numbering. */
 int chol_task_id(int64_t N, int type, int i, int j, int k, int64_t* id);

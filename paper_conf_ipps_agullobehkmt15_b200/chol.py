@@ -65,6 +65,15 @@ def _load():
         "chol_task_id": ([i64, i32, i32, i32, i32, ctypes.POINTER(i64)], i32),
         "chol_bounds": ([i64, i64, i32, dp, dp, dp], i32),
         "chol_job_trace": ([P, ctypes.POINTER(ctypes.c_uint64), i64, ctypes.POINTER(i64)], i32),
+        "chol_plan_dist": ([i64, i64, i32, i32, ctypes.POINTER(chol_opts_t), ctypes.POINTER(P)], i32),
+        "chol_dist_export": ([P, vp, i64, ctypes.POINTER(i64)], i32),
+        "chol_dist_connect": ([P, vp, i64], i32),
+        "chol_get_dist": ([P, ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(i32),
+                           ctypes.POINTER(i64), ctypes.POINTER(i64)], i32),
+        "chol_factor_async": ([P], i32),
+        "chol_wait": ([P, ctypes.POINTER(i32)], i32),
+        "chol_dist_layout": ([i64, i64, i32, i32, i32, ctypes.POINTER(i32), ctypes.POINTER(i32),
+                              ctypes.POINTER(ctypes.c_int32), i64], i32),
     }
     for name, (args, res) in sig.items():
         f = getattr(L, name)
@@ -77,7 +86,8 @@ _lib = _load()
 EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_destroy", "chol_strerror",
             "chol_generate", "chol_scatter", "chol_gather", "chol_factor_inplace", "chol_last_times",
             "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
-            "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace")
+            "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
+            "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout")
 
 
 def _ptr(x) -> int:
@@ -228,6 +238,87 @@ def chol_bounds(n: int, nb: int, ngpus: int, T_lat, T_thr) -> dict:
     out = (ctypes.c_double * 6)()
     _check(_lib.chol_bounds(n, nb, ngpus, lat, thr, out), "chol_bounds")
     return dict(zip(BOUND_NAMES, list(out)))
+
+
+def chol_plan_dist(n: int, nb: int, nranks: int, rank: int, **opts) -> int:
+    o = chol_opts_t(**opts)
+    h = ctypes.c_void_p()
+    _check(_lib.chol_plan_dist(n, nb, nranks, rank, ctypes.byref(o), ctypes.byref(h)), "chol_plan_dist")
+    return h.value
+
+
+def chol_dist_export(plan: int) -> bytes:
+    ln = ctypes.c_int64()
+    _check(_lib.chol_dist_export(plan, None, 0, ctypes.byref(ln)), "chol_dist_export")
+    buf = ctypes.create_string_buffer(ln.value)
+    _check(_lib.chol_dist_export(plan, buf, ln.value, ctypes.byref(ln)), "chol_dist_export")
+    return buf.raw
+
+
+def chol_dist_connect(plan: int, blobs: list) -> None:
+    stride = len(blobs[0])
+    assert all(len(b) == stride for b in blobs)
+    joined = ctypes.create_string_buffer(b"".join(blobs), stride * len(blobs))
+    _check(_lib.chol_dist_connect(plan, joined, stride), "chol_dist_connect")
+
+
+def chol_get_dist(plan: int) -> dict:
+    r, nr, gp, gq = ctypes.c_int(), ctypes.c_int(), ctypes.c_int(), ctypes.c_int()
+    no, ns = ctypes.c_int64(), ctypes.c_int64()
+    _check(_lib.chol_get_dist(plan, ctypes.byref(r), ctypes.byref(nr), ctypes.byref(gp), ctypes.byref(gq),
+                              ctypes.byref(no), ctypes.byref(ns)), "chol_get_dist")
+    return {"rank": r.value, "nranks": nr.value, "grid_p": gp.value, "grid_q": gq.value, "nowned": no.value,
+            "nslots": ns.value}
+
+
+def chol_factor_async(plan: int) -> None:
+    _check(_lib.chol_factor_async(plan), "chol_factor_async")
+
+
+def chol_wait(plan: int) -> int:
+    info = ctypes.c_int(0)
+    _check(_lib.chol_wait(plan, ctypes.byref(info)), "chol_wait")
+    return info.value
+
+
+def chol_dist_layout(n: int, nb: int, p: int, q: int, rank: int):
+    """(nowned, ncached, slot_map list) of a rank of the p x q grid (host only)."""
+    no, nc = ctypes.c_int(), ctypes.c_int()
+    N = n // nb
+    sm = (ctypes.c_int32 * max(N * (N + 1) // 2, 1))()
+    _check(_lib.chol_dist_layout(n, nb, p, q, rank, ctypes.byref(no), ctypes.byref(nc), sm, N * (N + 1) // 2),
+           "chol_dist_layout")
+    return no.value, nc.value, list(sm[:N * (N + 1) // 2])
+
+
+class DistPlan:
+    """One rank of a multi-GPU factorization.  `allgather(bytes) -> list[bytes]` exchanges
+    the connection blobs (e.g. torch.distributed.all_gather_object); for logical ranks in
+    one process build all plans first and connect them with connect_local()."""
+
+    def __init__(self, n: int, nb: int, nranks: int, rank: int, allgather=None, **opts):
+        self.n, self.nb, self.nranks, self.rank = n, nb, nranks, rank
+        opts.setdefault("executor", EXEC_SCHEDULER)
+        self.h = chol_plan_dist(n, nb, nranks, rank, **opts)
+        if allgather is not None:
+            chol_dist_connect(self.h, allgather(chol_dist_export(self.h)))
+
+    @staticmethod
+    def connect_local(plans: list) -> None:
+        blobs = [chol_dist_export(p.h) for p in plans]
+        for p in plans:
+            chol_dist_connect(p.h, blobs)
+
+    def close(self):
+        if self.h:
+            chol_destroy(self.h)
+            self.h = 0
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
 
 
 class Plan:

@@ -10,7 +10,10 @@
 #include <thread>
 #include <vector>
 
+#include <unistd.h>
+
 #include "../../include/chol.h"
+#include "dag.h"
 #include "kernels.h"
 #include "sched.h"
 #include "taskid.h"
@@ -33,6 +36,21 @@ struct chol_plan_s {
   bool factored = false;
   int last_launches = 0;
   SchedState* sched = nullptr;  // persistent-scheduler state (sched.cu)
+  // ---- multi-GPU (chol_plan_dist): this rank's share of the 2D block-cyclic layout
+  bool dist = false, connected = false;
+  int rank = 0, nranks = 1, p = 1, q = 1;
+  int64_t nslots = 0, nowned = 0;
+  std::vector<int> h_slot_map, h_owned_tile;  // tile -> local slot; owned slot -> tile
+  int* d_slot_map = nullptr;
+  int* d_owner_slot = nullptr;
+  int* d_owned_tile = nullptr;
+  int* d_diag_slots = nullptr;  // owned diagonal tiles' slots
+  int ndiag = 0;
+  int* d_flags = nullptr;       // per tile: epoch in which this rank published it
+  double** d_peer_slots = nullptr;
+  int** d_peer_flags = nullptr;
+  std::vector<void*> ipc_opened;
+  unsigned epoch = 0;
 };
 
 #define CUDA_TRY(x)                                   \
@@ -95,6 +113,14 @@ extern "C" int chol_destroy(chol_plan_t p) {
   if (p->sched) sched_destroy(p->sched);
   cudaSetDevice(p->device);
   if (p->stream) cudaStreamSynchronize(p->stream);
+  for (void* ptr : p->ipc_opened) cudaIpcCloseMemHandle(ptr);
+  cudaFree(p->d_slot_map);
+  cudaFree(p->d_owner_slot);
+  cudaFree(p->d_owned_tile);
+  cudaFree(p->d_diag_slots);
+  cudaFree(p->d_flags);
+  cudaFree(p->d_peer_slots);
+  cudaFree(p->d_peer_flags);
   cudaFree(p->tiles);
   cudaFree(p->d_info);
   cudaFree(p->d_base);
@@ -178,6 +204,182 @@ extern "C" int chol_plan(int64_t n, int64_t nb, int ngpus, chol_plan_t* out) {
   return chol_plan_ex(n, nb, ngpus, nullptr, out);
 }
 
+// ------------------------------------------------------------------ multi-GPU plan
+// One process (or one logical rank) per GPU; 2D block-cyclic owner-computes.
+extern "C" int chol_plan_dist(int64_t n, int64_t nb, int nranks, int rank, const chol_opts_t* o, chol_plan_t* out) {
+  if (!out) return -4;
+  *out = nullptr;
+  if (n <= 0) return -1;
+  if (nb <= 0 || n % nb != 0 || nb % 32 != 0) return -2;
+  if (nranks < 1 || rank < 0 || rank >= nranks) return -3;
+  chol_opts_t opts{};
+  if (o) opts = *o;
+  if (opts.policy < 0 || opts.policy > 2 || opts.executor != CHOL_EXEC_SCHEDULER || opts.trsm_pin_distance < 0 ||
+      opts.latency_workers < 0 || opts.workers < 0 || opts.grid_p < 0 || opts.grid_q < 0 || opts.trace < 0 ||
+      opts.trace > 2)
+    return -6;
+  if (opts.grid_p == 0 && opts.grid_q == 0) {
+    opts.grid_p = 1;
+    opts.grid_q = nranks;
+  }
+  if (opts.grid_p * opts.grid_q != nranks) return -3;
+  int ndev = 0;
+  if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev < 1) {
+    cudaGetLastError();
+    return -3;
+  }
+  auto* p = new (std::nothrow) chol_plan_s();
+  if (!p) return -9;
+  auto fail = [&](int s) {
+    chol_destroy(p);
+    return s;
+  };
+  p->n = n;
+  p->nb = nb;
+  p->N = n / nb;
+  p->ntasks = n_tasks(p->N);
+  p->bs = pick_block(nb);
+  p->opts = opts;
+  p->dist = true;
+  p->rank = rank;
+  p->nranks = nranks;
+  p->p = opts.grid_p;
+  p->q = opts.grid_q;
+  cudaError_t e;
+  if ((e = cudaGetDevice(&p->device))) return fail(-100 - (int)e);
+  cudaDeviceGetAttribute(&p->sms, cudaDevAttrMultiProcessorCount, p->device);
+  int nowned = 0, ncached = 0;
+  dist_layout(p->N, p->p, p->q, rank, p->h_slot_map, &nowned, &ncached);
+  p->nowned = nowned;
+  p->nslots = nowned + ncached;
+  p->ntiles = std::max<int64_t>(p->nslots, 1);
+  p->h_owned_tile.assign(nowned, 0);
+  std::vector<int> diag;
+  for (int64_t t = 0; t < (int64_t)p->h_slot_map.size(); ++t)
+    if (p->h_slot_map[t] >= 0 && p->h_slot_map[t] < nowned) p->h_owned_tile[p->h_slot_map[t]] = (int)t;
+  for (int64_t k = 0; k < p->N; ++k)
+    if (tile_owner_h(k, k, p->p, p->q) == rank) diag.push_back(p->h_slot_map[tile_index(k, k)]);
+  p->ndiag = (int)diag.size();
+  std::vector<int> oslot;
+  owner_slots(p->N, p->p, p->q, oslot);
+  const size_t tiles_n = p->h_slot_map.size();
+  e = cudaMalloc(&p->tiles, (size_t)p->ntiles * nb * nb * sizeof(double));
+  if (e == cudaErrorMemoryAllocation) {
+    cudaGetLastError();
+    return fail(-9);
+  }
+  if (e) return fail(-100 - (int)e);
+  if ((e = cudaMalloc(&p->d_slot_map, tiles_n * 4)) || (e = cudaMalloc(&p->d_owner_slot, tiles_n * 4)) ||
+      (e = cudaMalloc(&p->d_owned_tile, std::max<size_t>(nowned, 1) * 4)) ||
+      (e = cudaMalloc(&p->d_diag_slots, std::max<size_t>(diag.size(), 1) * 4)) ||
+      (e = cudaMalloc(&p->d_flags, tiles_n * 4)) || (e = cudaMalloc(&p->d_peer_slots, nranks * sizeof(double*))) ||
+      (e = cudaMalloc(&p->d_peer_flags, nranks * sizeof(int*))))
+    return fail(-100 - (int)e);
+  cudaMemcpy(p->d_slot_map, p->h_slot_map.data(), tiles_n * 4, cudaMemcpyHostToDevice);
+  cudaMemcpy(p->d_owner_slot, oslot.data(), tiles_n * 4, cudaMemcpyHostToDevice);
+  if (nowned) cudaMemcpy(p->d_owned_tile, p->h_owned_tile.data(), nowned * 4, cudaMemcpyHostToDevice);
+  if (!diag.empty()) cudaMemcpy(p->d_diag_slots, diag.data(), diag.size() * 4, cudaMemcpyHostToDevice);
+  cudaMemset(p->d_flags, 0, tiles_n * 4);
+  if ((e = cudaStreamCreateWithFlags(&p->stream, cudaStreamNonBlocking))) return fail(-100 - (int)e);
+  if ((e = cudaMalloc(&p->d_info, sizeof(int)))) return fail(-100 - (int)e);
+  if ((e = cudaMalloc(&p->d_base, sizeof(uint64_t)))) return fail(-100 - (int)e);
+  if (opts.trace) {
+    if ((e = cudaMalloc(&p->d_t0, p->ntasks * sizeof(uint64_t)))) return fail(-100 - (int)e);
+    if ((e = cudaMalloc(&p->d_t1, p->ntasks * sizeof(uint64_t)))) return fail(-100 - (int)e);
+  }
+  for (cudaEvent_t* ev : {&p->ev0, &p->ev1, &p->ev2, &p->ev3})
+    if ((e = cudaEventCreate(ev))) return fail(-100 - (int)e);
+  int st = 0;
+  if ((st = encode_tile_map(p))) return fail(st);
+  if ((e = prepare_kernels(p->bs))) return fail(-100 - (int)e);
+  DistInfo di{p->p, p->q, rank, nranks, p->h_slot_map.data()};
+  if ((st = sched_create(&p->sched, p->N, p->nb, p->bs, p->sms, &p->opts, p->stream, &di))) return fail(st);
+  *out = p;
+  return 0;
+}
+
+namespace {
+struct ExportBlob {  // what a rank tells the others (chol_dist_export / chol_dist_connect)
+  uint32_t magic, version;
+  int32_t pid, device, rank, nranks;
+  uint64_t slots_ptr, flags_ptr;
+  cudaIpcMemHandle_t slots_h, flags_h;
+};
+constexpr uint32_t kBlobMagic = 0x43484f4cu;  // "CHOL"
+}  // namespace
+
+extern "C" int chol_dist_export(chol_plan_t p, void* blob, int64_t cap, int64_t* len) {
+  if (!p || !p->dist) return -4;
+  if (len) *len = (int64_t)sizeof(ExportBlob);
+  if (!blob) return 0;
+  if (cap < (int64_t)sizeof(ExportBlob)) return -4;
+  cudaSetDevice(p->device);
+  ExportBlob b{};
+  b.magic = kBlobMagic;
+  b.version = 1;
+  b.pid = (int32_t)getpid();
+  b.device = p->device;
+  b.rank = p->rank;
+  b.nranks = p->nranks;
+  b.slots_ptr = (uint64_t)(uintptr_t)p->tiles;
+  b.flags_ptr = (uint64_t)(uintptr_t)p->d_flags;
+  CUDA_TRY(cudaIpcGetMemHandle(&b.slots_h, p->tiles));
+  CUDA_TRY(cudaIpcGetMemHandle(&b.flags_h, p->d_flags));
+  memcpy(blob, &b, sizeof(b));
+  return 0;
+}
+
+extern "C" int chol_dist_connect(chol_plan_t p, const void* blobs, int64_t stride) {
+  if (!p || !p->dist || !blobs || stride < (int64_t)sizeof(ExportBlob)) return -4;
+  if (p->connected) return 0;
+  cudaSetDevice(p->device);
+  std::vector<double*> slots(p->nranks);
+  std::vector<int*> flags(p->nranks);
+  const int me = (int)getpid();
+  for (int r = 0; r < p->nranks; ++r) {
+    ExportBlob b;
+    memcpy(&b, static_cast<const char*>(blobs) + r * stride, sizeof(b));
+    if (b.magic != kBlobMagic || b.rank != r || b.nranks != p->nranks) return -6;
+    if (r == p->rank) {
+      slots[r] = p->tiles;
+      flags[r] = p->d_flags;
+    } else if (b.pid == me) {  // logical ranks in one process: plain device pointers
+      if (b.device != p->device) {
+        cudaError_t e = cudaDeviceEnablePeerAccess(b.device, 0);
+        if (e != cudaSuccess && e != cudaErrorPeerAccessAlreadyEnabled) return -100 - (int)e;
+        cudaGetLastError();
+      }
+      slots[r] = reinterpret_cast<double*>(b.slots_ptr);
+      flags[r] = reinterpret_cast<int*>(b.flags_ptr);
+    } else {  // another process: map its allocations (NVLink peer memory)
+      void *ps = nullptr, *pf = nullptr;
+      CUDA_TRY(cudaIpcOpenMemHandle(&ps, b.slots_h, cudaIpcMemLazyEnablePeerAccess));
+      p->ipc_opened.push_back(ps);
+      CUDA_TRY(cudaIpcOpenMemHandle(&pf, b.flags_h, cudaIpcMemLazyEnablePeerAccess));
+      p->ipc_opened.push_back(pf);
+      slots[r] = static_cast<double*>(ps);
+      flags[r] = static_cast<int*>(pf);
+    }
+  }
+  CUDA_TRY(cudaMemcpy(p->d_peer_slots, slots.data(), p->nranks * sizeof(double*), cudaMemcpyHostToDevice));
+  CUDA_TRY(cudaMemcpy(p->d_peer_flags, flags.data(), p->nranks * sizeof(int*), cudaMemcpyHostToDevice));
+  sched_set_dist(p->sched, p->d_slot_map, p->d_owner_slot, p->d_peer_slots, p->d_peer_flags, p->d_flags);
+  p->connected = true;
+  return 0;
+}
+
+extern "C" int chol_get_dist(chol_plan_t p, int* rank, int* nranks, int* grid_p, int* grid_q, int64_t* nowned,
+                             int64_t* nslots) {
+  if (!p) return -4;
+  if (rank) *rank = p->rank;
+  if (nranks) *nranks = p->nranks;
+  if (grid_p) *grid_p = p->p;
+  if (grid_q) *grid_q = p->q;
+  if (nowned) *nowned = p->dist ? p->nowned : p->ntiles;
+  if (nslots) *nslots = p->dist ? p->nslots : p->ntiles;
+  return 0;
+}
+
 extern "C" int chol_get_stream(chol_plan_t p, void** stream) {
   if (!p || !stream) return -4;
   *stream = (void*)p->stream;
@@ -206,11 +408,19 @@ static bool is_device_ptr(const void* ptr) {
   return a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged;
 }
 
+static int64_t store_slot(const chol_plan_s* p, int64_t i, int64_t j) {
+  return p->dist ? p->h_slot_map[tile_index(i, j)] : tile_index(i, j);
+}
+static bool owns(const chol_plan_s* p, int64_t i, int64_t j) {
+  return !p->dist || tile_owner_h(i, j, p->p, p->q) == p->rank;
+}
+
 static int scatter_impl(chol_plan_s* p, const double* A, int64_t lda) {
   const int64_t nb = p->nb;
   for (int64_t i = 0; i < p->N; ++i)
     for (int64_t j = 0; j <= i; ++j) {
-      double* dst = p->tiles + tile_index((int)i, (int)j) * nb * nb;
+      if (!owns(p, i, j)) continue;
+      double* dst = p->tiles + store_slot(p, i, j) * nb * nb;
       const double* src = A + i * nb * lda + j * nb;
       CUDA_TRY(cudaMemcpy2DAsync(dst, nb * 8, src, lda * 8, nb * 8, nb, cudaMemcpyDefault, p->stream));
     }
@@ -233,20 +443,27 @@ static void host_zero_upper_tiles(double* L, int64_t ldl, int64_t n, int64_t nb)
   (void)N;
 }
 
+// Multi-GPU plans write only the tiles this rank owns; rank 0 also zeroes the strictly
+// upper tiles (a caller gathering every rank into one buffer gets the full L).
 static int gather_impl(chol_plan_s* p, double* L, int64_t ldl) {
   const int64_t nb = p->nb, n = p->n;
-  CUDA_TRY(launch_zero_upper_diag(p->tiles, (int)nb, (int)p->N, p->stream));
+  if (p->dist)
+    CUDA_TRY(launch_zero_upper_diag(p->tiles, (int)nb, (int)p->N, p->stream, p->d_diag_slots, p->ndiag));
+  else
+    CUDA_TRY(launch_zero_upper_diag(p->tiles, (int)nb, (int)p->N, p->stream));
   const bool dev = is_device_ptr(L);
+  const bool zero_upper = !p->dist || p->rank == 0;
   for (int64_t i = 0; i < p->N; ++i) {
     for (int64_t j = 0; j <= i; ++j) {
-      const double* src = p->tiles + tile_index((int)i, (int)j) * nb * nb;
+      if (!owns(p, i, j)) continue;
+      const double* src = p->tiles + store_slot(p, i, j) * nb * nb;
       double* dst = L + i * nb * ldl + j * nb;
       CUDA_TRY(cudaMemcpy2DAsync(dst, ldl * 8, src, nb * 8, nb * 8, nb, cudaMemcpyDefault, p->stream));
     }
-    if (dev && (i + 1) * nb < n)
+    if (zero_upper && dev && (i + 1) * nb < n)
       CUDA_TRY(cudaMemset2DAsync(L + i * nb * ldl + (i + 1) * nb, ldl * 8, 0, (n - (i + 1) * nb) * 8, nb, p->stream));
   }
-  if (!dev) host_zero_upper_tiles(L, ldl, n, nb);
+  if (zero_upper && !dev) host_zero_upper_tiles(L, ldl, n, nb);
   return 0;
 }
 
@@ -274,7 +491,8 @@ extern "C" int chol_generate(chol_plan_t p, uint64_t seed, int family) {
   if (!p) return -4;
   if (family < 0 || family > 1) return -6;
   cudaSetDevice(p->device);
-  CUDA_TRY(launch_generate(p->tiles, p->n, (int)p->nb, (int)p->N, seed, family, p->stream));
+  CUDA_TRY(launch_generate(p->tiles, p->n, (int)p->nb, (int)p->N, seed, family, p->stream,
+                           p->dist ? p->d_owned_tile : nullptr, p->nowned));
   CUDA_TRY(cudaStreamSynchronize(p->stream));
   return 0;
 }
@@ -321,10 +539,12 @@ static int factor_launch(chol_plan_s* p) {
   int nl = 0;
   CUDA_TRY(cudaEventRecord(p->ev0, p->stream));
   int st = 0;
+  if (p->dist && !p->connected) return -8;
+  ++p->epoch;
   if (p->opts.executor == CHOL_EXEC_HOST)
     st = run_host_sequenced(p, &nl);
   else
-    st = sched_run(p->sched, p->map, base_params(p), p->stream, &nl);
+    st = sched_run(p->sched, p->map, base_params(p), p->stream, &nl, p->epoch);
   if (st) return st;
   CUDA_TRY(cudaEventRecord(p->ev1, p->stream));
   p->last_launches = nl;
@@ -341,6 +561,18 @@ static int finish_info(chol_plan_s* p, int* info) {
   p->factored = true;
   if (info) *info = (h == INT_MAX) ? 0 : h;
   return 0;
+}
+
+extern "C" int chol_factor_async(chol_plan_t p) {
+  if (!p) return -4;
+  cudaSetDevice(p->device);
+  return factor_launch(p);
+}
+
+extern "C" int chol_wait(chol_plan_t p, int* info) {
+  if (!p) return -4;
+  cudaSetDevice(p->device);
+  return finish_info(p, info);
 }
 
 extern "C" int chol_factor_inplace(chol_plan_t p, int* info) {
@@ -393,6 +625,7 @@ extern "C" int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int
   uint64_t lo = UINT64_MAX, hi = 0;
   int64_t w = 0;
   auto emit = [&](int type, int i, int j, int k, int64_t id) {
+    if (p->dist && t0[id] == UINT64_MAX) return;  // task ran on another rank
     const uint64_t a = t0[id], b = t1[id] >> 16;
     if (t0[id] != UINT64_MAX) {
       lo = std::min(lo, a);
@@ -401,7 +634,7 @@ extern "C" int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int
     if (recs && w < cap) {
       chol_task_rec_t& r = recs[w];
       r.type = (uint8_t)type;
-      r.gpu = 0;
+      r.gpu = (uint8_t)p->rank;
       r.worker = (uint16_t)(t1[id] & 0xffff);
       r.i = i;
       r.j = j;
@@ -435,6 +668,7 @@ extern "C" int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t
 // ------------------------------------------------------------------ calibration / single tasks
 extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double* ms) {
   if (!p) return -4;
+  if (p->dist) return -8;
   const int N = (int)p->N;
   if (type < 0 || type > 3 || reps < 1 || k < 0 || k >= N) return -6;
   if (type == T_TRSM && !(i > k && i < N)) return -6;
@@ -471,6 +705,7 @@ extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int r
 
 extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, double* ms) {
   if (!p) return -4;
+  if (p->dist) return -8;
   const int N = (int)p->N;
   if (type < 0 || type > 3 || reps < 1 || count < 1) return -6;
   // instances at step k = 0: POTRF on diagonal tiles 0..count-1, TRSM (i, 0),

@@ -80,9 +80,62 @@ std::vector<double> bottom_levels(int64_t N, const double w[4]) {
   return bl;
 }
 
+// Multi-GPU layout (2D block-cyclic owner-computes): the tiles this
+// rank owns get slots 0..nowned-1 in tile-index order; the remote tiles its tasks read
+// (final panel tiles L_kk, L_ik) get cache slots in order of first use.
+void dist_layout(int64_t N, int p, int q, int rank, std::vector<int>& slot_map, int* nowned, int* ncached) {
+  const int64_t ntiles = N * (N + 1) / 2;
+  slot_map.assign(ntiles, -1);
+  int s = 0;
+  for (int64_t i = 0; i < N; ++i)
+    for (int64_t j = 0; j <= i; ++j)
+      if (tile_owner_h(i, j, p, q) == rank) slot_map[tile_index(i, j)] = s++;
+  *nowned = s;
+  auto need = [&](int64_t i, int64_t j) {
+    const int64_t t = tile_index(i, j);
+    if (slot_map[t] < 0) slot_map[t] = s++;
+  };
+  for (int64_t k = 0; k < N; ++k) {
+    for (int64_t i = k + 1; i < N; ++i)
+      if (tile_owner_h(i, k, p, q) == rank) need(k, k);  // TRSM_i_k reads L_kk
+    for (int64_t j = k + 1; j < N; ++j) {
+      if (tile_owner_h(j, j, p, q) == rank) need(j, k);  // SYRK_j_k reads L_jk
+      for (int64_t i = j + 1; i < N; ++i)
+        if (tile_owner_h(i, j, p, q) == rank) {  // GEMM_i_j_k reads L_ik, L_jk
+          need(i, k);
+          need(j, k);
+        }
+    }
+  }
+  *ncached = s - *nowned;
+}
+
+// slot of every tile in its owner's store
+void owner_slots(int64_t N, int p, int q, std::vector<int>& out) {
+  out.assign(N * (N + 1) / 2, -1);
+  std::vector<int> cnt(p * q, 0);
+  for (int64_t i = 0; i < N; ++i)
+    for (int64_t j = 0; j <= i; ++j) out[tile_index(i, j)] = cnt[tile_owner_h(i, j, p, q)]++;
+}
+
 }  // namespace chol
 
 using namespace chol;
+
+extern "C" int chol_dist_layout(int64_t n, int64_t nb, int p, int q, int rank, int* nowned, int* ncached,
+                                int32_t* slot_map, int64_t cap) {
+  if (n <= 0) return -1;
+  if (nb <= 0 || n % nb) return -2;
+  if (p < 1 || q < 1 || rank < 0 || rank >= p * q) return -3;
+  std::vector<int> sm;
+  int no = 0, nc = 0;
+  dist_layout(n / nb, p, q, rank, sm, &no, &nc);
+  if (nowned) *nowned = no;
+  if (ncached) *ncached = nc;
+  if (slot_map)
+    for (int64_t t = 0; t < (int64_t)sm.size() && t < cap; ++t) slot_map[t] = sm[t];
+  return 0;
+}
 
 extern "C" int chol_dag(int64_t N, int64_t* ntasks, int64_t* nedges, int64_t* edges, int64_t cap) {
   if (N <= 0) return -1;

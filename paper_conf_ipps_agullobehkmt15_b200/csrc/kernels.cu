@@ -119,9 +119,10 @@ __global__ void k_stamp(uint64_t* base) { *base = globaltimer_ns(); }
 __global__ void k_init_info(int* info) { *info = INT_MAX; }
 
 // zero the strictly upper triangle of every diagonal tile
-__global__ void k_zero_upper_diag(double* tiles, int nb, int N) {
+// slots: store slots of the diagonal tiles to clean (null: tile k at tile_index(k, k))
+__global__ void k_zero_upper_diag(double* tiles, int nb, int N, const int* slots) {
   const int k = blockIdx.y;
-  double* T = tiles + tile_index(k, k) * (int64_t)nb * nb;
+  double* T = tiles + (slots ? (int64_t)slots[k] : tile_index(k, k)) * (int64_t)nb * nb;
   for (int64_t idx = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; idx < (int64_t)nb * nb;
        idx += (int64_t)gridDim.x * blockDim.x) {
     const int r = (int)(idx / nb), c = (int)(idx % nb);
@@ -154,14 +155,17 @@ __device__ __forceinline__ int64_t l0_band(uint64_t seed, int64_t n, int64_t x, 
   return top < 2 ? -1 : (top < 4 ? 1 : 0);
 }
 
-__global__ void k_generate(double* tiles, int64_t n, int nb, int N, uint64_t seed, int family, int64_t t_off) {
-  const int64_t t = t_off + blockIdx.y;  // tile index in the store
+// slot_tile: tile index held by each generated store slot (null: slot == tile index)
+__global__ void k_generate(double* tiles, int64_t n, int nb, int N, uint64_t seed, int family, int64_t t_off,
+                           const int* slot_tile) {
+  const int64_t slot = t_off + blockIdx.y;
+  const int64_t t = slot_tile ? (int64_t)slot_tile[slot] : slot;  // tile index
   // decode t -> (ti, tj), ti >= tj
   int ti = (int)((sqrt(8.0 * (double)t + 1.0) - 1.0) / 2.0);
   while ((int64_t)ti * (ti + 1) / 2 > t) --ti;
   while ((int64_t)(ti + 1) * (ti + 2) / 2 <= t) ++ti;
   const int tj = (int)(t - (int64_t)ti * (ti + 1) / 2);
-  double* T = tiles + t * (int64_t)nb * nb;
+  double* T = tiles + slot * (int64_t)nb * nb;
   for (int64_t idx = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; idx < (int64_t)nb * nb;
        idx += (int64_t)gridDim.x * blockDim.x) {
     const int64_t r = idx / nb, c = idx % nb;
@@ -283,15 +287,17 @@ cudaError_t launch_init_info(int* info, cudaStream_t s) {
   k_init_info<<<1, 1, 0, s>>>(info);
   return cudaGetLastError();
 }
-cudaError_t launch_zero_upper_diag(double* tiles, int nb, int N, cudaStream_t s) {
-  k_zero_upper_diag<<<dim3(64, N), 256, 0, s>>>(tiles, nb, N);
+cudaError_t launch_zero_upper_diag(double* tiles, int nb, int N, cudaStream_t s, const int* slots, int count) {
+  if (count == 0) return cudaSuccess;
+  k_zero_upper_diag<<<dim3(64, slots ? count : N), 256, 0, s>>>(tiles, nb, N, slots);
   return cudaGetLastError();
 }
-cudaError_t launch_generate(double* tiles, int64_t n, int nb, int N, uint64_t seed, int family, cudaStream_t s) {
-  const int64_t ntiles = (int64_t)N * (N + 1) / 2;
+cudaError_t launch_generate(double* tiles, int64_t n, int nb, int N, uint64_t seed, int family, cudaStream_t s,
+                            const int* slot_tile, int64_t nslots) {
+  const int64_t ntiles = slot_tile ? nslots : (int64_t)N * (N + 1) / 2;
   for (int64_t t0 = 0; t0 < ntiles; t0 += 65535) {
     const int64_t cnt = ntiles - t0 < 65535 ? ntiles - t0 : 65535;
-    k_generate<<<dim3(64, (unsigned)cnt), 256, 0, s>>>(tiles, n, nb, N, seed, family, t0);
+    k_generate<<<dim3(64, (unsigned)cnt), 256, 0, s>>>(tiles, n, nb, N, seed, family, t0, slot_tile);
   }
   return cudaGetLastError();
 }

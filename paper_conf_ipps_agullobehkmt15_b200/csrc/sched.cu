@@ -36,7 +36,9 @@ constexpr int kQStride = 32;           // ints between queue heads (separate 128
 // default plan); POTRF inner: J_DIAG potf2 of block (b,b), J_PANEL solve of block (r,b),
 // J_PUPD K=BS update of block (r,q); TRSM right-looking: J_TS solve of block (s,c) of
 // A_ik against L_kk[c,c], J_TU K=BS update A_ik[s,c'] -= A_ik[s,c] L_kk[c',c]^T.
-enum JobType : int16_t { J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6 };
+// Multi-GPU: J_RECV copies row slab a of remote panel tile (i, j) from its owner b (peer
+// memory over NVLink) into this rank's cache slot.
+enum JobType : int16_t { J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6, J_RECV = 7 };
 struct Job {
   int16_t type, i, j, k, a, b, c, pad;
 };
@@ -64,6 +66,18 @@ struct DevSched {
   int total_nodes;
   int latency_workers;     // STATIC: CTAs [0, latency_workers) serve the pinned queues only
   int policy;
+  // ---- multi-GPU (null / 0 on one GPU)
+  const int* slot_map;        // local slot of each tile
+  const int* owner_slot;      // slot of each tile in its owner's store
+  double* const* peer_slots;  // [nranks] slot stores (IPC-mapped; own entry = local)
+  int* const* peer_flags;     // [nranks] per-tile "final at epoch" flags of each rank
+  int* my_flags;              // this rank's flags (== peer_flags[rank])
+  const int* node_publish;    // tile made final by the node (published to the other ranks), -1
+  const int4* watch;          // RECV nodes to fire: {node, owner rank, tile, 0}, sorted by step
+  int* watch_fired;           // per watch entry
+  int nwatch;
+  unsigned epoch;             // factorization number (flags hold the epoch they became final in)
+  int nb;
 };
 
 // ------------------------------------------------------------------ device queue ops
@@ -161,17 +175,17 @@ __device__ void producer_loop(Ctx<BS>& c) {
         int64_t ta, tb, tcb;
         int ra, rb, kb, nst, cr, cc;
         if (type == J_UPD) {  // GEMM/SYRK block (i, j, k, bm, bn)
-          ta = tile_index(d0.z, d1.x); ra = d1.y * BS;
-          tb = tile_index(d0.w, d1.x); rb = d1.z * BS;
+          ta = c.slot(d0.z, d1.x); ra = d1.y * BS;
+          tb = c.slot(d0.w, d1.x); rb = d1.z * BS;
           kb = 0; nst = c.nb / BK;
-          tcb = tile_index(d0.z, d0.w); cr = d1.y * BS; cc = d1.z * BS;
+          tcb = c.slot(d0.z, d0.w); cr = d1.y * BS; cc = d1.z * BS;
         } else if (type == J_PUPD) {  // POTRF update block (k, b, r, q)
-          ta = tb = tcb = tile_index(d1.x, d1.x);
+          ta = tb = tcb = c.slot(d1.x, d1.x);
           ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
           cr = ra; cc = rb;
         } else {  // TRSM update (i, k, c, s, c'): A_ik[s, c'] -= A_ik[s, c] L_kk[c', c]^T
-          ta = tcb = tile_index(d0.z, d1.x);
-          tb = tile_index(d1.x, d1.x);
+          ta = tcb = c.slot(d0.z, d1.x);
+          tb = c.slot(d1.x, d1.x);
           ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
           cr = ra; cc = rb;
         }
@@ -189,7 +203,7 @@ __device__ void producer_loop(Ctx<BS>& c) {
           ++tcount;
           fence_proxy_async();
           const int nst = cb * BS / BK;
-          produce_range(c, pit, nst, tile_index(d0.z, d1.x), d1.y * BS, tile_index(d1.x, d1.x), cb * BS, 0, 0, nst);
+          produce_range(c, pit, nst, c.slot(d0.z, d1.x), d1.y * BS, c.slot(d1.x, d1.x), cb * BS, 0, 0, nst);
           pit += nst;
         }
       }
@@ -199,9 +213,78 @@ __device__ void producer_loop(Ctx<BS>& c) {
   }
 }
 
+// ---- multi-GPU receive: peer (NVLink) -> local cache, 16-byte loads, 8 in flight per thread
+template <int BS>
+__device__ __forceinline__ void recv_slab(Ctx<BS>& c, const DevSched& d, int i, int j, int sl, int owner) {
+  const int64_t t = tile_index(i, j);
+  const int64_t tile_elems = (int64_t)c.nb * c.nb, off = (int64_t)sl * BS * c.nb;
+  const double2* src = reinterpret_cast<const double2*>(d.peer_slots[owner] + (int64_t)d.owner_slot[t] * tile_elems + off);
+  double2* dst = reinterpret_cast<double2*>(c.tiles + c.slot(i, j) * tile_elems + off);
+  const int n2 = BS * c.nb / 2;
+  constexpr int U = 8;
+  for (int base = threadIdx.x; base < n2; base += U * kComputeThreads) {
+    double2 v[U];
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      const int idx = base + u * kComputeThreads;
+      if (idx < n2) v[u] = __ldcg(src + idx);
+    }
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      const int idx = base + u * kComputeThreads;
+      if (idx < n2) __stcg(dst + idx, v[u]);
+    }
+  }
+}
+
+// ---- multi-GPU watcher (warp 10 of CTA 0): fires the RECV nodes whose remote tile became
+// final (owner's flag == epoch), in step order, with a 64-entry sliding window.
+__device__ void watcher_loop(const DevSched& d) {
+  const int lane = threadIdx.x & 31;
+  int w0 = 0;
+  unsigned backoff = 64;
+  while (w0 < d.nwatch) {
+    bool fired_any = false;
+#pragma unroll
+    for (int h = 0; h < 2; ++h) {
+      const int e = w0 + h * 32 + lane;
+      bool fire = false;
+      int4 w = make_int4(0, 0, 0, 0);
+      if (e < d.nwatch && !ld_volatile(&d.watch_fired[e])) {
+        w = d.watch[e];
+        unsigned f;
+        asm volatile("ld.acquire.sys.global.u32 %0, [%1];" : "=r"(f) : "l"(d.peer_flags[w.y] + w.z) : "memory");
+        fire = (f == d.epoch);
+      }
+      if (fire) {
+        d.watch_fired[e] = 1;
+        __threadfence();
+        if (atomicSub(&d.node_deps[w.x], 1) == 1) push_node(d, w.x);
+      }
+      fired_any |= __any_sync(0xffffffffu, fire);
+    }
+    // advance past the fired prefix
+    while (true) {
+      const int e = w0 + lane;
+      const bool f = e >= d.nwatch || ld_volatile(&d.watch_fired[e]);
+      const unsigned m = __ballot_sync(0xffffffffu, f);
+      const int adv = (m == 0xffffffffu) ? 32 : __ffs(~m) - 1;
+      w0 += adv;
+      if (adv < 32 || w0 >= d.nwatch) break;
+    }
+    if (!fired_any) {
+      __nanosleep(backoff);
+      backoff = backoff < 1024 ? backoff * 2 : 1024;
+    } else {
+      backoff = 64;
+    }
+  }
+}
+
 // ---- compute warps: run the job's consumer side
 template <int BS>
-__device__ __forceinline__ void compute_job(Ctx<BS>& c, int type, const int4& d0, const int4& d1, int* info) {
+__device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int type, const int4& d0, const int4& d1,
+                                            int* info) {
   Acc<BS> acc;
   if (type == J_UPD) {
     const int i = d0.z, j = d0.w, k = d1.x, bm = d1.y, bn = d1.z;
@@ -235,6 +318,10 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, int type, const int4& d0
     const int i = d0.z, k = d1.x, cb = d1.y, sl = d1.z;
     solve_block(c, acc, false, c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
                 c.tile(k, k) + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+  } else if (type == J_RECV) {  // copy BS rows of a remote panel tile into the local cache
+    const int i = d0.z, j = d0.w, sl = d1.y, owner = d1.z;
+    (void)owner;
+    recv_slab(c, d, i, j, sl, owner);
   } else if (type == J_DIAG) {
     sub_potrf_diag(c, d1.x, d1.y, info);
   } else if (type == J_PANEL) {
@@ -243,7 +330,7 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, int type, const int4& d0
 }
 
 template <int BS>
-__device__ void compute_loop(Ctx<BS>& c, int* info) {
+__device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
   uint32_t q = 0;
   while (true) {
     const int e = q & 1;
@@ -255,7 +342,7 @@ __device__ void compute_loop(Ctx<BS>& c, int* info) {
       c.jdesc[e * 3 + 2] = make_int4((int)(t0 & 0xffffffffull), (int)(t0 >> 32), 0, 0);
     }
     const int type = d0.y & 0xff, skip = d0.y >> 8;
-    if (!skip) compute_job(c, type, d0, d1, info);
+    if (!skip) compute_job(c, d, type, d0, d1, info);
     __syncwarp();
     if (c.lane == 0) {
       mbar_arrive(c.lfree);  // lbuf (C block / L block / rdiag) no longer needed
@@ -275,7 +362,7 @@ __device__ __forceinline__ void complete_job(const DevSched& d, const StepParams
                                              uint64_t t1_abs) {
   __threadfence();  // the compute warps' stores (acquired through jdone) before the counters
   const int node = d.job_node[job];
-  if (sp.tr_t0) {
+  if (sp.tr_t0 && d.node_paper[node] >= 0) {
     const uint64_t base = *sp.tr_base;
     const uint64_t t0 = t0_abs - base, t_end = t1_abs - base;
     const int pt = d.node_paper[node];
@@ -289,6 +376,13 @@ __device__ __forceinline__ void complete_job(const DevSched& d, const StepParams
   }
   if (atomicSub(&d.node_left[node], 1) == 1) {
     __threadfence();
+    if (d.node_publish) {
+      const int pt = d.node_publish[node];
+      if (pt >= 0) {  // panel tile final: release it to every rank (system scope, NVLink)
+        __threadfence_system();
+        asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(d.my_flags + pt), "r"(d.epoch) : "memory");
+      }
+    }
     for (int e = d.succ_off[node]; e < d.succ_off[node + 1]; ++e) {
       const int s = d.succ[e];
       if (atomicSub(&d.node_deps[s], 1) == 1) push_node(d, s);
@@ -357,7 +451,7 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
 template <int BS>
 __global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__ CUtensorMap map, StepParams sp,
                                                          DevSched d) {
-  auto c = make_ctx<BS>(&map, sp.tiles, sp.nb, sp.N);
+  auto c = make_ctx<BS>(&map, sp.tiles, sp.nb, sp.N, d.slot_map);
   const bool latency_worker = d.policy == 2 && (int)blockIdx.x < d.latency_workers;
   if (c.warp >= kComputeWarps) {
     asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(kRegsControl));
@@ -365,11 +459,13 @@ __global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__
       if (c.lane == 0) producer_loop(c);
     } else if (c.warp == kSchedWarp) {
       scheduler_loop(c, d, sp, latency_worker);
+    } else if (c.warp == kSchedWarp + 1 && blockIdx.x == 0 && d.nwatch > 0) {
+      watcher_loop(d);
     }
     return;
   }
   asm volatile("setmaxnreg.inc.sync.aligned.u32 %0;\n" ::"n"(kRegsCompute));
-  compute_loop(c, sp.info);
+  compute_loop(c, d, sp.info);
 }
 
 __global__ void k_sched_init(DevSched d, const int* roots, int nroots) {
@@ -389,7 +485,8 @@ struct SchedState {
   void* dev_pristine = nullptr; // initial node_deps / node_left
   size_t pristine_bytes = 0;
   int* roots = nullptr;
-  uint64_t* job_trace = nullptr;           // device, 3 per job (trace == 2)
+  int nrecv_jobs = 0;
+  uint64_t* job_trace = nullptr;           // device, 4 per job (trace == 2)
   std::vector<int16_t> h_job_type;         // host copies for chol_job_trace
   std::vector<int> h_job_paper;
 };
@@ -429,7 +526,7 @@ struct Builder {
 }  // namespace
 
 int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts,
-                 cudaStream_t s) {
+                 cudaStream_t s, const DistInfo* dist) {
   auto* st = new SchedState();
   st->N = N;
   st->nb = nb;
@@ -442,11 +539,16 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // (CHOL_TRSM_BLOCKS=1, development switch; measured 2.5% slower at n=19200).
   const char* ev = getenv("CHOL_TRSM_BLOCKS");
   const bool trsm_slab = !(ev && ev[0] == '1');
+  // Multi-GPU: this rank creates the nodes of the tasks that overwrite the tiles it owns
+  // (owner-computes), plus one RECV node per remote panel tile it reads.
+  auto mine = [&](int64_t i, int64_t j) { return !dist || tile_owner(i, j, dist->p, dist->q) == dist->rank; };
+  std::vector<int> publish;  // per node: tile made final (published to other ranks) or -1
   // ---- nodes and jobs, Algorithm 1 order
-  std::vector<int> first_node(n_tasks(N)), last_node(n_tasks(N));
+  std::vector<int> first_node(n_tasks(N), -1), last_node(n_tasks(N), -1);
   for (int k = 0; k < N; ++k) {
     const int pid = (int)id_potrf(N, k);
     int prev = -1;
+    if (mine(k, k)) {
     for (int b = 0; b < nbb; ++b) {
       const int dn = B.add_node(pid, T_POTRF, k, k);
       B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
@@ -468,7 +570,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       }
     }
     last_node[pid] = prev;
+    }
     for (int i = k + 1; i < N; ++i) {
+      if (!mine(i, k)) continue;
       if (trsm_slab) {  // one left-looking row-slab job per BS rows
         const int tid = (int)id_trsm(N, i, k);
         const int n = B.add_node(tid, T_TRSM, i, k);
@@ -502,12 +606,15 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     }
     for (int j = k + 1; j < N; ++j) {
       const int sid = (int)id_syrk(N, j, k);
-      const int n = B.add_node(sid, T_SYRK, j, k);
-      for (int bm = 0; bm < nbb; ++bm)
-        for (int bn = 0; bn <= bm; ++bn)
-          B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
-      first_node[sid] = last_node[sid] = n;
+      if (mine(j, j)) {
+        const int n = B.add_node(sid, T_SYRK, j, k);
+        for (int bm = 0; bm < nbb; ++bm)
+          for (int bn = 0; bn <= bm; ++bn)
+            B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
+        first_node[sid] = last_node[sid] = n;
+      }
       for (int i = j + 1; i < N; ++i) {
+        if (!mine(i, j)) continue;
         const int gid = (int)id_gemm(N, i, j, k);
         const int g = B.add_node(gid, T_GEMM, i, k);
         for (int bm = 0; bm < nbb; ++bm)
@@ -520,10 +627,65 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
 
   // ---- task edges: direct data dependencies of Algorithm 1 (dag.cpp, L213-220),
   // mapped onto the nodes (POTRF_k enters at its first inner node, leaves at its last).
-  std::vector<std::pair<int64_t, int64_t>> E;
-  std::vector<int> type_of;
-  build_task_dag(N, E, type_of);
-  for (auto& e : E) B.edge(last_node[e.first], first_node[e.second]);
+  std::vector<int4> watch;  // multi-GPU: {RECV node, owner, tile, step}
+  if (!dist) {
+    std::vector<std::pair<int64_t, int64_t>> E;
+    std::vector<int> type_of;
+    build_task_dag(N, E, type_of);
+    for (auto& e : E) B.edge(last_node[e.first], first_node[e.second]);
+  } else {
+    // Same last-writer rule over the tiles an owned task touches: an owned tile's last
+    // writer is an owned task; a remote tile (always a final panel tile L_kk / L_ik) is
+    // reached through this rank's RECV node for it, fired by the watcher when the owner
+    // publishes the tile.
+    std::vector<int64_t> last_writer((size_t)(N * (N + 1) / 2), -1);
+    std::vector<int> recv_node((size_t)(N * (N + 1) / 2), -1);
+    std::vector<int> preds;
+    auto visit = [&](int64_t task, std::initializer_list<std::pair<int64_t, int64_t>> touched, int64_t wi,
+                     int64_t wj) {
+      const int64_t wt = tile_index(wi, wj);
+      if (mine(wi, wj)) {
+        preds.clear();
+        for (auto& ij : touched) {
+          const int64_t t = tile_index(ij.first, ij.second);
+          int pn = -1;
+          if (mine(ij.first, ij.second)) {
+            if (last_writer[t] >= 0) pn = last_node[last_writer[t]];
+          } else {
+            if (recv_node[t] < 0) {
+              const int owner = tile_owner(ij.first, ij.second, dist->p, dist->q);
+              const int rn = B.add_node(-1, -1, (int)ij.first, (int)ij.second);
+              for (int sl = 0; sl < nbb; ++sl)
+                B.add_job(rn, Job{J_RECV, (int16_t)ij.first, (int16_t)ij.second, 0, (int16_t)sl, (int16_t)owner, 0, 0});
+              B.deps[rn] += 1;  // fired by the watcher (remote readiness)
+              recv_node[t] = rn;
+              watch.push_back(make_int4(rn, owner, (int)t, (int)ij.second));
+            }
+            pn = recv_node[t];
+          }
+          if (pn >= 0 && std::find(preds.begin(), preds.end(), pn) == preds.end()) preds.push_back(pn);
+        }
+        for (int pn : preds) B.edge(pn, first_node[task]);
+      }
+      last_writer[wt] = task;
+    };
+    for (int64_t k = 0; k < N; ++k) {
+      visit(id_potrf(N, k), {{k, k}}, k, k);
+      for (int64_t i = k + 1; i < N; ++i) visit(id_trsm(N, i, k), {{k, k}, {i, k}}, i, k);
+      for (int64_t j = k + 1; j < N; ++j) {
+        visit(id_syrk(N, j, k), {{j, k}, {j, j}}, j, j);
+        for (int64_t i = j + 1; i < N; ++i) visit(id_gemm(N, i, j, k), {{i, k}, {j, k}, {i, j}}, i, j);
+      }
+    }
+    std::stable_sort(watch.begin(), watch.end(), [](const int4& a, const int4& b) { return a.w < b.w; });
+    // panel tiles this rank finalises are published (their final node)
+    publish.assign(B.deps.size(), -1);
+    for (int64_t k = 0; k < N; ++k) {
+      if (mine(k, k)) publish[last_node[id_potrf(N, k)]] = (int)tile_index(k, k);
+      for (int64_t i = k + 1; i < N; ++i)
+        if (mine(i, k)) publish[last_node[id_trsm(N, i, k)]] = (int)tile_index(i, k);
+    }
+  }
 
   // ---- priorities: bottom-level of each Algorithm 1 task (HEFT / dmdas, L299-301,
   // L655-660; reading R13) with latency-estimate weights, quantised into kBuckets;
@@ -536,7 +698,8 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   for (int v = 0; v < nnodes; ++v) {
     int bucket = 0;
     if (opts->policy != CHOL_POLICY_DYNAMIC)
-      bucket = std::min(kBuckets - 1, (int)(kBuckets * bl[B.paper[v]] / blmax));
+      bucket = B.paper[v] < 0 ? kBuckets - 1  // RECV: gates local work
+                              : std::min(kBuckets - 1, (int)(kBuckets * bl[B.paper[v]] / blmax));
     bool pinned = false;
     if (opts->policy == CHOL_POLICY_STATIC) {
       if (B.ptype[v] == T_POTRF) pinned = true;
@@ -582,6 +745,8 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   const size_t o_nq = off; off = align(off + nnodes * 4);
   const size_t o_qbase = off; off = align(off + kQueues * 4);
   const size_t o_roots = off; off = align(off + std::max<size_t>(roots.size(), 1) * 4);
+  const size_t o_pub = off; off = align(off + (publish.empty() ? 4 : publish.size() * 4));
+  const size_t o_watch = off; off = align(off + std::max<size_t>(watch.size(), 1) * 16);
   const size_t static_bytes = off;
   std::vector<char> h(static_bytes, 0);
   memcpy(h.data() + o_jobs, B.jobs.data(), B.jobs.size() * sizeof(Job));
@@ -594,6 +759,8 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   memcpy(h.data() + o_nq, node_queue.data(), nnodes * 4);
   memcpy(h.data() + o_qbase, qbase.data(), kQueues * 4);
   if (!roots.empty()) memcpy(h.data() + o_roots, roots.data(), roots.size() * 4);
+  if (!publish.empty()) memcpy(h.data() + o_pub, publish.data(), publish.size() * 4);
+  if (!watch.empty()) memcpy(h.data() + o_watch, watch.data(), watch.size() * 16);
 
   // dynamic part: node_deps, node_left, q_items, q_head, q_tail, done, finished
   size_t doff = 0;
@@ -606,6 +773,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   const size_t d_tail = doff; doff = align(doff + kQueues * kQStride * 4);
   const size_t d_done = doff; doff = align(doff + 4);
   const size_t d_fin = doff; doff = align(doff + 4);
+  const size_t d_fired = doff; doff = align(doff + std::max<size_t>(watch.size(), 1) * 4);
   std::vector<char> hp(pristine, 0);
   memcpy(hp.data() + d_deps, B.deps.data(), nnodes * 4);
   memcpy(hp.data() + d_left, B.jcnt.data(), nnodes * 4);
@@ -646,6 +814,13 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   d.done_nodes = reinterpret_cast<int*>(D + d_done);
   d.finished = reinterpret_cast<int*>(D + d_fin);
   d.total_nodes = nnodes;
+  d.node_publish = publish.empty() ? nullptr : reinterpret_cast<const int*>(S + o_pub);
+  d.watch = reinterpret_cast<const int4*>(S + o_watch);
+  d.nwatch = (int)watch.size();
+  d.watch_fired = reinterpret_cast<int*>(D + d_fired);
+  d.nb = (int)nb;
+  st->nrecv_jobs = 0;
+  for (const Job& jb : B.jobs) st->nrecv_jobs += jb.type == J_RECV;
   if (opts->trace == 2) {
     if ((e = cudaMalloc(&st->job_trace, (size_t)st->njobs * 4 * sizeof(uint64_t)))) {
       cudaGetLastError();
@@ -680,7 +855,19 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   return 0;
 }
 
-int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch) {
+int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slot, double* const* d_peer_slots,
+                   int* const* d_peer_flags, int* d_my_flags) {
+  st->d.slot_map = d_slot_map;
+  st->d.owner_slot = d_owner_slot;
+  st->d.peer_slots = d_peer_slots;
+  st->d.peer_flags = d_peer_flags;
+  st->d.my_flags = d_my_flags;
+  return 0;
+}
+
+int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch,
+              unsigned epoch) {
+  st->d.epoch = epoch;
   cudaError_t e;
   if ((e = cudaMemcpyAsync(st->dev_dynamic, st->dev_pristine, st->pristine_bytes, cudaMemcpyDeviceToDevice, s)))
     return -100 - (int)e;

@@ -8,8 +8,21 @@
 
 namespace chol {
 struct SchedState;
-int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts, cudaStream_t s);
-int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch);
+
+// Multi-GPU (2D block-cyclic owner-computes): what this rank owns.
+struct DistInfo {
+  int p, q, rank, nranks;
+  const int* h_slot_map;  // host, N(N+1)/2 entries: local slot of tile t (owned or cached), -1 = absent
+};
+__host__ __device__ inline int tile_owner(int i, int j, int p, int q) { return (i % p) * q + (j % q); }
+
+int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts, cudaStream_t s,
+                 const DistInfo* dist = nullptr);
+// device pointers of the distributed plan, known after the IPC handle exchange
+int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slot, double* const* d_peer_slots,
+                   int* const* d_peer_flags, int* d_my_flags);
+int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch,
+              unsigned epoch = 1);
 int sched_workers(const SchedState* st);
 int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* njobs);
 void sched_destroy(SchedState* st);

@@ -69,18 +69,25 @@ struct Ctx {
   uint32_t cphase; // parity of the next cbar completion
   int warp, lane;
 
-  __device__ double* tile(int i, int j) const { return tiles + tile_index(i, j) * (int64_t)nb * nb; }
+  const int* slot_map;  // multi-GPU: store slot of tile (i,j) (tile_index order); null = identity
+  __device__ int64_t slot(int i, int j) const {
+    const int64_t t = tile_index(i, j);
+    return slot_map ? (int64_t)__ldg(slot_map + t) : t;
+  }
+  __device__ double* tile(int i, int j) const { return tiles + slot(i, j) * (int64_t)nb * nb; }
   __device__ bool issuer() const { return threadIdx.x == 0; }
 };
 
 template <int BS>
-__device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tiles, int nb, int N) {
+__device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tiles, int nb, int N,
+                                            const int* slot_map = nullptr) {
   extern __shared__ __align__(1024) char smem_raw[];
   using C = Cfg<BS>;
   Ctx<BS> c;
   char* base = reinterpret_cast<char*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
   c.map = map;
   c.tiles = tiles;
+  c.slot_map = slot_map;
   c.nb = nb;
   c.N = N;
   c.pipe = base;
@@ -562,8 +569,8 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
 template <int BS>
 __device__ __forceinline__ void sub_update(Ctx<BS>& c, int i, int j, int k, int bm, int bn) {
   Acc<BS> acc;
-  const CPrefetch cp{tile_index(i, j), bm * BS, bn * BS};
-  gemm_mainloop(c, tile_index(i, k), bm * BS, tile_index(j, k), bn * BS, 0, c.nb, acc, &cp);
+  const CPrefetch cp{c.slot(i, j), bm * BS, bn * BS};
+  gemm_mainloop(c, c.slot(i, k), bm * BS, c.slot(j, k), bn * BS, 0, c.nb, acc, &cp);
   epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
 }
 
@@ -576,7 +583,7 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
   const double* L = c.tile(k, k);
   for (int cb = 0; cb < nbb; ++cb) {
     Acc<BS> acc;
-    if (cb > 0) gemm_mainloop(c, tile_index(i, k), slab * BS, tile_index(k, k), cb * BS, 0, cb * BS, acc);
+    if (cb > 0) gemm_mainloop(c, c.slot(i, k), slab * BS, c.slot(k, k), cb * BS, 0, cb * BS, acc);
     solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
     // X[:, cb] (generic stores) is read by TMA in the next block: complete the stores
     // at L2 (gpu-scope fence), then order them before async-proxy accesses.
@@ -604,7 +611,7 @@ __device__ __forceinline__ void sub_potrf_panel(Ctx<BS>& c, int k, int b, int r)
 template <int BS>
 __device__ __forceinline__ void sub_potrf_update(Ctx<BS>& c, int k, int b, int r, int q) {
   Acc<BS> acc;
-  const int64_t t = tile_index(k, k);
+  const int64_t t = c.slot(k, k);
   const CPrefetch cp{t, r * BS, q * BS};
   gemm_mainloop(c, t, r * BS, t, q * BS, b * BS, (b + 1) * BS, acc, &cp);
   epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);

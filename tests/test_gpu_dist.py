@@ -1,0 +1,84 @@
+"""Multi-GPU path on ONE GPU: R logical ranks (one plan each, workers = SMs / R, same
+process, plain device pointers instead of IPC) run the distributed persistent schedulers
+concurrently; the panel tiles travel between ranks through the RECV jobs exactly as they
+would over NVLink.  Checked against the oracle."""
+import numpy as np
+import pytest
+
+import oracle
+import spdgen
+
+pytestmark = pytest.mark.gpu
+torch = pytest.importorskip("torch")
+
+
+def _lib():
+    import paper_conf_ipps_agullobehkmt15_b200 as c
+    return c
+
+
+def run_logical(n, nb, p, q, seed=0, family=0, A=None, policy=1):
+    c = _lib()
+    R = p * q
+    sms = torch.cuda.get_device_properties(0).multi_processor_count
+    plans = [c.DistPlan(n, nb, R, r, grid_p=p, grid_q=q, workers=sms // R, policy=policy) for r in range(R)]
+    c.DistPlan.connect_local(plans)
+    if A is None:
+        for pl in plans:
+            c.chol_generate(pl.h, seed, family)
+    else:
+        dA = torch.from_numpy(np.ascontiguousarray(A)).cuda()
+        for pl in plans:
+            c.chol_scatter(pl.h, dA, n)
+    for pl in plans:
+        c.chol_factor_async(pl.h)
+    infos = [c.chol_wait(pl.h) for pl in plans]
+    out = torch.zeros((n, n), dtype=torch.float64, device="cuda")
+    for pl in plans:
+        c.chol_gather(pl.h, out, n)
+    torch.cuda.synchronize()
+    for pl in plans:
+        pl.close()
+    nz = [i for i in infos if i]
+    return out.cpu().numpy(), (min(nz) if nz else 0)
+
+
+@pytest.mark.parametrize("n,nb,p,q", [(1920, 96, 1, 2), (1920, 96, 2, 2), (2880, 96, 1, 3), (3840, 960, 2, 2),
+                                      (2304, 96, 2, 4)])
+def test_dist_matches_oracle(n, nb, p, q):
+    A = spdgen.uniform_spd(n, seed=n + p + q)
+    L, info = run_logical(n, nb, p, q, A=A)
+    ref, rinfo = oracle.chol_tiled(A, nb)
+    assert info == rinfo == 0
+    d = oracle.rel_diff(L, ref)
+    assert d["max_rel_floored"] <= 1e-10, d
+    assert oracle.backward_error(A, L) <= 10.0
+
+
+@pytest.mark.parametrize("p,q", [(1, 2), (2, 2)])
+def test_dist_integer_family_bitwise(p, q):
+    n, nb = 1920, 96
+    L, info = run_logical(n, nb, p, q, seed=4, family=1)
+    assert info == 0
+    assert np.array_equal(L, spdgen.integer_L0(n, 4))
+
+
+def test_dist_bitwise_equals_single_gpu():
+    """Reading R15 extended: the distribution does not change any tile's update order."""
+    c = _lib()
+    n, nb = 1920, 96
+    A = spdgen.uniform_spd(n, seed=11)
+    L2, _ = run_logical(n, nb, 2, 2, A=A)
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+        dA = torch.from_numpy(A.copy()).cuda()
+        assert p.factor(dA) == 0
+        L1 = dA.cpu().numpy()
+    assert np.array_equal(L1, L2)
+
+
+def test_dist_non_spd_info():
+    n, nb = 1920, 96
+    L0 = spdgen.integer_L0(n, 6)
+    A = spdgen.make_non_spd(spdgen.integer_spd(n, 6), L0, 1000, "zero")
+    _, info = run_logical(n, nb, 2, 2, A=A)
+    assert info == 1001
