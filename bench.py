@@ -9,8 +9,11 @@ n = 19200 as 20 x 20 tiles of nb = 960 on 1 B200.
 
 Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
        [--n 19200] [--nb 960] [--policy cp|dynamic|static] [--executor sched|host]
-Under torchrun (N > 1) each rank factors its own matrix (replicas, see DESIGN.md
-"Multi-GPU"); rank 0 prints ONE JSON line.
+       [--logical-ranks R --grid PxQ]
+Under torchrun (N > 1) the N ranks factor ONE matrix together (2D block-cyclic
+owner-computes, panel tiles pulled over NVLink peer memory; strong scaling); rank 0
+prints ONE JSON line.  --logical-ranks R runs the distributed path with R ranks sharing
+one GPU (tests the multi-GPU machinery; not a scaling number).
 """
 from __future__ import annotations
 
@@ -47,6 +50,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-bounds", action="store_true")
     ap.add_argument("--cpu-sample-n", type=int, default=7680)
+    ap.add_argument("--grid", default="", help="process grid PxQ (default 1xN; SURVEY §8e prefers p <= q)")
+    ap.add_argument("--logical-ranks", type=int, default=0)
     return ap.parse_args()
 
 
@@ -220,6 +225,108 @@ def calibrate(c, args, workers):
     return T_lat, T_thr
 
 
+def grid_of(args, R):
+    if args.grid:
+        p, q = (int(x) for x in args.grid.lower().split("x"))
+        assert p * q == R, "grid must have R ranks"
+        return p, q
+    p = 1
+    for cand in range(int(R ** 0.5), 0, -1):  # p <= q, as square as possible
+        if R % cand == 0:
+            p = cand
+            break
+    return p, R // p
+
+
+def run_dist(args, ws, rank, local):
+    """Multi-GPU strong scaling: one factorization of A (n x n) on ws ranks."""
+    import torch
+    import torch.distributed as dist
+    import paper_conf_ipps_agullobehkmt15_b200 as c
+
+    n, nb = args.n, args.nb
+    flops = n ** 3 / 3.0
+    p, q = grid_of(args, ws)
+
+    def allgather(blob):
+        out = [None] * ws
+        dist.all_gather_object(out, blob)
+        return out
+
+    plan = c.DistPlan(n, nb, ws, rank, allgather=allgather, grid_p=p, grid_q=q, policy=POLICIES[args.policy])
+    for _ in range(args.warmup):
+        c.chol_generate(plan.h, args.seed, 0)
+        barrier(ws)
+        c.chol_factor_inplace(plan.h)
+    torch.cuda.synchronize()
+    times, launches = [], 0
+    with ClockSampler(local) as clk:
+        for _ in range(args.steps):
+            c.chol_generate(plan.h, args.seed, 0)
+            barrier(ws)
+            torch.cuda.synchronize()
+            info = c.chol_factor_inplace(plan.h)
+            torch.cuda.synchronize()
+            assert info == 0, info
+            times.append(allmax(ws, c.chol_last_times(plan.h)[0]))
+            launches += c.chol_last_launches(plan.h)
+    clocks = clk.summary()
+    d = c.chol_get_dist(plan.h)
+    plan.close()
+    t_step = sum(times) / len(times)
+    value = flops / t_step / 1e12
+    line = {
+        "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": ws, "steps": args.steps,
+        "warmup": args.warmup, "ms_per_step": 1e3 * t_step, "higher_is_better": True, "scaling": "strong",
+        "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": {"workload": f"FP64 SPD n={n} as {n // nb}x{n // nb} tiles of nb={nb}", "n": n, "nb": nb,
+                   "parallelism": f"2D block-cyclic {p}x{q}, owner-computes, NVLink peer pulls of panel tiles",
+                   "policy": args.policy, "tiles_owned_rank0": d["nowned"],
+                   "tiles_cached_rank0": d["nslots"] - d["nowned"],
+                   "timing": "CUDA events per rank around each factorization, max over ranks"},
+        "pct_fp64_peak": 100.0 * value / (ws * FP64_PEAK_TFLOPS),
+        "roofline": {"bound": "tensor", "achieved": value / ws, "peak": FP64_PEAK_TFLOPS, "unit": "TFLOP/s",
+                     "frac": value / ws / FP64_PEAK_TFLOPS, "traffic": None,
+                     "kernel": "k_sched per GPU (achieved = whole-job rate / GPUs)",
+                     "peak_source": "measured FP64 DMMA microbenchmark"},
+        "clocks": clocks, "gpu_launches": launches,
+    }
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+
+
+def run_logical(args):
+    """R logical ranks sharing this GPU (workers = SMs / R each): the distributed machinery
+    (owner map, RECV jobs, publish/watch flags) exercised on one device."""
+    import torch
+    import paper_conf_ipps_agullobehkmt15_b200 as c
+
+    n, nb, R = args.n, args.nb, args.logical_ranks
+    p, q = grid_of(args, R)
+    sms = torch.cuda.get_device_properties(0).multi_processor_count
+    plans = [c.DistPlan(n, nb, R, r, grid_p=p, grid_q=q, workers=sms // R, policy=POLICIES[args.policy])
+             for r in range(R)]
+    c.DistPlan.connect_local(plans)
+    times = []
+    for it in range(args.warmup + args.steps):
+        for pl in plans:
+            c.chol_generate(pl.h, args.seed, 0)
+        torch.cuda.synchronize()
+        t0 = time.perf_counter()
+        for pl in plans:
+            c.chol_factor_async(pl.h)
+        infos = [c.chol_wait(pl.h) for pl in plans]
+        dt = time.perf_counter() - t0
+        assert not any(infos)
+        if it >= args.warmup:
+            times.append(max(c.chol_last_times(pl.h)[0] for pl in plans))
+    t = sum(times) / len(times)
+    print(json.dumps({"metric": METRIC, "value": n ** 3 / 3 / t / 1e12, "unit": "TFLOP/s", "n_gpus": 1,
+                      "logical_ranks": R, "grid": f"{p}x{q}", "ms_per_step": 1e3 * t, "steps": args.steps,
+                      "warmup": args.warmup, "note": "distributed path on one GPU (not a scaling number)",
+                      "config": {"n": n, "nb": nb}}), flush=True)
+
+
 def run_ours(args, ws, rank, local):
     import torch
     import paper_conf_ipps_agullobehkmt15_b200 as c
@@ -332,6 +439,10 @@ def main():
     ws, rank, local = dist_setup()
     if args.impl == "reference":
         run_reference(args, ws, rank)
+    elif args.logical_ranks > 1:
+        run_logical(args)
+    elif ws > 1:
+        run_dist(args, ws, rank, local)
     else:
         run_ours(args, ws, rank, local)
     if ws > 1:
