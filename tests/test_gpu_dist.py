@@ -82,3 +82,16 @@ def test_dist_non_spd_info():
     A = spdgen.make_non_spd(spdgen.integer_spd(n, 6), L0, 1000, "zero")
     _, info = run_logical(n, nb, 2, 2, A=A)
     assert info == 1001
+
+
+def test_two_processes_share_gpu_through_ipc():
+    """The real multi-process path (CUDA IPC export/open of the tile stores and flags,
+    peer pulls, publish/watch) with two OS processes on cuda:0."""
+    import subprocess
+    import sys
+    import os
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    r = subprocess.run([sys.executable, os.path.join(root, "tools", "two_proc_one_gpu.py"), "960"],
+                       capture_output=True, text=True, timeout=240)
+    assert r.returncode == 0, r.stderr[-2000:]
+    assert "'infos': [0, 0], 'exact': True" in r.stdout, r.stdout
