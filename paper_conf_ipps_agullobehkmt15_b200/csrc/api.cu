@@ -8,6 +8,7 @@
 #include <cstring>
 #include <new>
 #include <thread>
+#include <chrono>
 #include <vector>
 
 #include <unistd.h>
@@ -51,6 +52,13 @@ struct chol_plan_s {
   int** d_peer_flags = nullptr;
   std::vector<void*> ipc_opened;
   unsigned epoch = 0;
+  // ---- single GPU, persistent scheduler: streamed host input / output (chol_factor)
+  int* d_in_flags = nullptr;   // per tile: epoch in which its input copy landed (device)
+  int* h_out_flags = nullptr;  // per tile: epoch in which it became final (host-mapped)
+  int* d_out_flags = nullptr;  // device alias of h_out_flags
+  int* h_epoch = nullptr;      // pinned source of the 4-byte arrival-flag copies
+  cudaStream_t s_in = nullptr, s_out = nullptr;
+  bool streamed_run = false;
 };
 
 #define CUDA_TRY(x)                                   \
@@ -121,6 +129,11 @@ extern "C" int chol_destroy(chol_plan_t p) {
   cudaFree(p->d_flags);
   cudaFree(p->d_peer_slots);
   cudaFree(p->d_peer_flags);
+  cudaFree(p->d_in_flags);
+  if (p->h_out_flags) cudaFreeHost(p->h_out_flags);
+  if (p->h_epoch) cudaFreeHost(p->h_epoch);
+  if (p->s_in) cudaStreamDestroy(p->s_in);
+  if (p->s_out) cudaStreamDestroy(p->s_out);
   cudaFree(p->tiles);
   cudaFree(p->d_info);
   cudaFree(p->d_base);
@@ -195,6 +208,19 @@ extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t*
   if ((e = prepare_kernels(p->bs))) return fail(-100 - (int)e);
   if (opts.executor == CHOL_EXEC_SCHEDULER) {
     if ((st = sched_create(&p->sched, p->N, p->nb, p->bs, p->sms, &p->opts, p->stream))) return fail(st);
+    // arrival flags (device), publish flags (host-mapped, polled by chol_factor), copy streams
+    if ((e = cudaMalloc(&p->d_in_flags, p->ntiles * sizeof(int))) ||
+        (e = cudaHostAlloc(&p->h_out_flags, p->ntiles * sizeof(int), cudaHostAllocMapped)) ||
+        (e = cudaHostGetDevicePointer(&p->d_out_flags, p->h_out_flags, 0)) ||
+        (e = cudaHostAlloc(&p->h_epoch, sizeof(int), cudaHostAllocDefault)) ||
+        (e = cudaMalloc(&p->d_peer_flags, sizeof(int*))) ||
+        (e = cudaStreamCreateWithFlags(&p->s_in, cudaStreamNonBlocking)) ||
+        (e = cudaStreamCreateWithFlags(&p->s_out, cudaStreamNonBlocking)))
+      return fail(-100 - (int)e);
+    memset(p->h_out_flags, 0, p->ntiles * sizeof(int));
+    cudaMemset(p->d_in_flags, 0, p->ntiles * sizeof(int));
+    cudaMemcpy(p->d_peer_flags, &p->d_in_flags, sizeof(int*), cudaMemcpyHostToDevice);
+    sched_set_dist(p->sched, nullptr, nullptr, nullptr, p->d_peer_flags, p->d_out_flags);
   }
   *out = p;
   return 0;
@@ -541,6 +567,8 @@ static int factor_launch(chol_plan_s* p) {
   int st = 0;
   if (p->dist && !p->connected) return -8;
   ++p->epoch;
+  if (!p->dist && p->sched && !p->streamed_run)  // input already resident: every tile has arrived
+    CUDA_TRY(launch_fill_flags(p->d_in_flags, p->ntiles, (int)p->epoch, p->stream));
   if (p->opts.executor == CHOL_EXEC_HOST)
     st = run_host_sequenced(p, &nl);
   else
@@ -583,10 +611,104 @@ extern "C" int chol_factor_inplace(chol_plan_t p, int* info) {
   return finish_info(p, info);
 }
 
+// chol_factor from HOST memory with the persistent scheduler: the factorization starts
+// on the first tile while the rest is still being copied in (per-tile arrival flags
+// gate each tile's first task), and every off-diagonal L tile is copied out as soon as
+// its TRSM publishes it; only the diagonal tiles are copied after the kernel ends.
+static int factor_streamed(chol_plan_s* p, const double* A, int64_t lda, double* L, int64_t ldl, int* info) {
+  const int64_t nb = p->nb, N = p->N, n = p->n;
+  CUDA_TRY(cudaEventRecord(p->ev2, p->stream));
+  p->streamed_run = true;
+  const int st = factor_launch(p);  // epoch++, scheduler kernel waits on the arrival flags
+  p->streamed_run = false;
+  if (st) return st;
+  *p->h_epoch = (int)p->epoch;
+  CUDA_TRY(cudaStreamWaitEvent(p->s_in, p->ev2, 0));
+  CUDA_TRY(cudaStreamWaitEvent(p->s_out, p->ev2, 0));
+  auto copy_in = [&](int64_t i, int64_t j) -> int {
+    const int64_t t = tile_index(i, j);
+    CUDA_TRY(cudaMemcpy2DAsync(p->tiles + t * nb * nb, nb * 8, A + i * nb * lda + j * nb, lda * 8, nb * 8, nb,
+                               cudaMemcpyDefault, p->s_in));
+    CUDA_TRY(cudaMemcpyAsync(p->d_in_flags + t, p->h_epoch, sizeof(int), cudaMemcpyHostToDevice, p->s_in));
+    return 0;
+  };
+  // first-use order of Algorithm 1 (must match the scheduler's watch order): column 0
+  // (POTRF_0, TRSM_i_0), then for each j the diagonal tile (SYRK_j_0) and column j
+  // below it (GEMM_i_j_0)
+  int s = copy_in(0, 0);
+  for (int64_t i = 1; i < N && !s; ++i) s = copy_in(i, 0);
+  for (int64_t j = 1; j < N && !s; ++j) {
+    s = copy_in(j, j);
+    for (int64_t i = j + 1; i < N && !s; ++i) s = copy_in(i, j);
+  }
+  if (s) return s;
+  std::thread zero_upper([=] { host_zero_upper_tiles(L, ldl, n, nb); });
+  // stream out the off-diagonal tiles as they become final (published by their TRSM)
+  std::vector<int64_t> pending;
+  for (int64_t k = 0; k < N; ++k)
+    for (int64_t i = k + 1; i < N; ++i) pending.push_back(tile_index(i, k));
+  std::vector<int> row_of(p->ntiles), col_of(p->ntiles);
+  for (int64_t i = 0; i < N; ++i)
+    for (int64_t j = 0; j <= i; ++j) {
+      row_of[tile_index(i, j)] = (int)i;
+      col_of[tile_index(i, j)] = (int)j;
+    }
+  const volatile int* outf = p->h_out_flags;
+  size_t head = 0;
+  int rc = 0;
+  while (head < pending.size() && !rc) {
+    bool progressed = false;
+    for (size_t w = head; w < pending.size() && w < head + 256; ++w) {
+      const int64_t t = pending[w];
+      if (t < 0 || outf[t] != (int)p->epoch) continue;
+      const int64_t i = row_of[t], j = col_of[t];
+      const cudaError_t e = cudaMemcpy2DAsync(L + i * nb * ldl + j * nb, ldl * 8, p->tiles + t * nb * nb, nb * 8,
+                                              nb * 8, nb, cudaMemcpyDefault, p->s_out);
+      if (e) rc = -100 - (int)e;
+      pending[w] = -1;
+      progressed = true;
+    }
+    while (head < pending.size() && pending[head] < 0) ++head;
+    if (!progressed) {
+      if (cudaStreamQuery(p->stream) == cudaSuccess) {  // kernel done: take the rest
+        for (size_t w = head; w < pending.size(); ++w)
+          if (pending[w] >= 0) {
+            const int64_t t = pending[w], i = row_of[t], j = col_of[t];
+            cudaMemcpy2DAsync(L + i * nb * ldl + j * nb, ldl * 8, p->tiles + t * nb * nb, nb * 8, nb * 8, nb,
+                              cudaMemcpyDefault, p->s_out);
+            pending[w] = -1;
+          }
+        head = pending.size();
+      } else {
+        std::this_thread::yield();
+      }
+    }
+  }
+  // diagonal tiles after the factorization: zero their upper triangles, copy out
+  CUDA_TRY(launch_zero_upper_diag(p->tiles, (int)nb, (int)N, p->stream));
+  for (int64_t k = 0; k < N && !rc; ++k) {
+    const cudaError_t e = cudaMemcpy2DAsync(L + k * nb * ldl + k * nb, ldl * 8, p->tiles + tile_index(k, k) * nb * nb,
+                                            nb * 8, nb * 8, nb, cudaMemcpyDefault, p->stream);
+    if (e) rc = -100 - (int)e;
+  }
+  CUDA_TRY(cudaEventRecord(p->ev3, p->stream));
+  const int st2 = finish_info(p, info);
+  CUDA_TRY(cudaStreamSynchronize(p->s_in));
+  CUDA_TRY(cudaStreamSynchronize(p->s_out));
+  zero_upper.join();
+  if (rc) return rc;
+  if (st2) return st2;
+  float tot = 0.f;
+  CUDA_TRY(cudaEventElapsedTime(&tot, p->ev2, p->ev3));
+  p->last_layout_s = tot * 1e-3 - p->last_factor_s;  // exposed (non-overlapped) transfer time
+  return 0;
+}
+
 extern "C" int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* L, int64_t ldl, int* info) {
   if (!p || !A || !L || (reinterpret_cast<uintptr_t>(A) & 7) || (reinterpret_cast<uintptr_t>(L) & 7)) return -4;
   if (lda < p->n || ldl < p->n) return -5;
   cudaSetDevice(p->device);
+  if (!p->dist && p->sched && !is_device_ptr(A) && !is_device_ptr(L)) return factor_streamed(p, A, lda, L, ldl, info);
   CUDA_TRY(cudaEventRecord(p->ev2, p->stream));
   int st = scatter_impl(p, A, lda);
   if (st) return st;

@@ -118,6 +118,12 @@ __global__ void k_stamp(uint64_t* base) { *base = globaltimer_ns(); }
 
 __global__ void k_init_info(int* info) { *info = INT_MAX; }
 
+// mark every input tile as arrived (factorizations whose input is already resident)
+__global__ void k_fill_flags(int* flags, int64_t n, int value) {
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < n; i += (int64_t)gridDim.x * blockDim.x)
+    flags[i] = value;
+}
+
 // zero the strictly upper triangle of every diagonal tile
 // slots: store slots of the diagonal tiles to clean (null: tile k at tile_index(k, k))
 __global__ void k_zero_upper_diag(double* tiles, int nb, int N, const int* slots) {
@@ -281,6 +287,10 @@ cudaError_t launch_update(int bs, const CUtensorMap& map, const StepParams& p, i
 
 cudaError_t launch_stamp(uint64_t* base, cudaStream_t s) {
   k_stamp<<<1, 1, 0, s>>>(base);
+  return cudaGetLastError();
+}
+cudaError_t launch_fill_flags(int* flags, int64_t n, int value, cudaStream_t s) {
+  k_fill_flags<<<(unsigned)((n + 255) / 256 < 1024 ? (n + 255) / 256 : 1024), 256, 0, s>>>(flags, n, value);
   return cudaGetLastError();
 }
 cudaError_t launch_init_info(int* info, cudaStream_t s) {

@@ -26,6 +26,7 @@ cudaError_t launch_trsm(int bs, const CUtensorMap& map, const StepParams& p, int
 cudaError_t launch_update(int bs, const CUtensorMap& map, const StepParams& p, int ntask, cudaStream_t s, int* nl);
 cudaError_t launch_stamp(uint64_t* base, cudaStream_t s);
 cudaError_t launch_init_info(int* info, cudaStream_t s);
+cudaError_t launch_fill_flags(int* flags, int64_t n, int value, cudaStream_t s);
 cudaError_t launch_zero_upper_diag(double* tiles, int nb, int N, cudaStream_t s, const int* slots = nullptr,
                                    int count = -1);
 cudaError_t launch_generate(double* tiles, int64_t n, int nb, int N, uint64_t seed, int family, cudaStream_t s,

@@ -633,6 +633,32 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     std::vector<int> type_of;
     build_task_dag(N, E, type_of);
     for (auto& e : E) B.edge(last_node[e.first], first_node[e.second]);
+    // Streamed input (chol_factor from host memory): the first task touching a tile
+    // waits for the tile's arrival flag (the copy engine writes it after the tile);
+    // watch order = first-use order = the order the tiles are copied in.
+    std::vector<char> seen((size_t)(N * (N + 1) / 2), 0);
+    int order = 0;
+    auto first_touch = [&](int64_t task, int64_t i, int64_t j) {
+      const int64_t t = tile_index(i, j);
+      if (seen[t]) return;
+      seen[t] = 1;
+      B.deps[first_node[task]] += 1;
+      watch.push_back(make_int4(first_node[task], 0, (int)t, order++));
+    };
+    for (int64_t k = 0; k < N; ++k) {
+      first_touch(id_potrf(N, k), k, k);
+      for (int64_t i = k + 1; i < N; ++i) first_touch(id_trsm(N, i, k), i, k);
+      for (int64_t j = k + 1; j < N; ++j) {
+        first_touch(id_syrk(N, j, k), j, j);
+        for (int64_t i = j + 1; i < N; ++i) first_touch(id_gemm(N, i, j, k), i, j);
+      }
+    }
+    // Streamed output: every final panel tile is published (host-mapped flags)
+    publish.assign(B.deps.size(), -1);
+    for (int64_t k = 0; k < N; ++k) {
+      publish[last_node[id_potrf(N, k)]] = (int)tile_index(k, k);
+      for (int64_t i = k + 1; i < N; ++i) publish[last_node[id_trsm(N, i, k)]] = (int)tile_index(i, k);
+    }
   } else {
     // Same last-writer rule over the tiles an owned task touches: an owned tile's last
     // writer is an owned task; a remote tile (always a final panel tile L_kk / L_ik) is
