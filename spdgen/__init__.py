@@ -29,8 +29,8 @@ M2 = np.uint64(0x94D049BB133111EB)
 INT_SALT = np.uint64(0xD1B54A32D192ED03)  # separates the integer family's stream
 BW = 3  # bandwidth of L0 in the integer family
 
-__all__ = ["splitmix64", "uniform_spd", "integer_L0", "integer_spd", "make_non_spd",
-           "BW"]
+__all__ = ["splitmix64", "uniform_spd", "uniform_entries", "integer_L0", "integer_L0_bands", "integer_spd",
+           "make_non_spd", "BW"]
 
 
 def splitmix64(x: np.ndarray) -> np.ndarray:
@@ -78,6 +78,16 @@ def uniform_spd(n: int, seed: int = 0, *, rows: slice | None = None,
                 blk[mask] = np.nan if upper == "nan" else 0.0
             out[a - r0:b - r0] = blk
     return out
+
+
+def uniform_entries(n: int, seed: int, i: np.ndarray, j: np.ndarray) -> np.ndarray:
+    """Entries A[i, j] of the ``uniform`` family for index arrays (any size n)."""
+    i = np.asarray(i, dtype=np.uint64)
+    j = np.asarray(j, dtype=np.uint64)
+    with np.errstate(over="ignore"):
+        key = np.uint64(seed) * GOLDEN + np.maximum(i, j) * np.uint64(n) + np.minimum(i, j)
+    v = _u01(splitmix64(key)) - 0.5
+    return np.where(i == j, v + float(n), v)
 
 
 def _int_hash(n: int, seed: int, i: np.ndarray, j: np.ndarray) -> np.ndarray:

@@ -35,3 +35,12 @@ def test_integer_family_structure():
     assert np.all(np.tril(L0, -spdgen.BW - 1) == 0)
     A = spdgen.integer_spd(200, 3)
     assert np.array_equal(A, L0 @ L0.T)
+
+
+def test_uniform_entries_match_dense():
+    n = 77
+    A = spdgen.uniform_spd(n, seed=3)
+    rng = np.random.default_rng(0)
+    i = rng.integers(0, n, 500)
+    j = rng.integers(0, n, 500)
+    assert np.array_equal(spdgen.uniform_entries(n, 3, i, j), A[i, j])
