@@ -377,89 +377,98 @@ __device__ __forceinline__ void panel_to_frag(const Ctx<BS>& c, Acc<BS>& x, int 
   }
 }
 
+// ---- row layout for the in-block solves: warp w < BS/16 owns rows 16w .. 16w+15 and
+// all columns; x[mi][cb] = {X[16w+8mi+g][8cb+2t], X[16w+8mi+g][8cb+2t+1]}.  Rows are
+// independent in X L^{-T}, so a warp never waits for another, and the pair a thread
+// holds is directly the A operand of a DMMA with k-slot t <-> column 8p+2t (+1).
+template <int BS>
+struct RowX {
+  static constexpr int NB = BS / 8;
+  double v[2][NB][2];
+};
+
 // X <- (X - acc) * Ld^{-T} for one BS x BS block X (ld ldx) against the lower
 // triangular BS x BS diagonal block Ld (ld ldl): the in-block part of TRSM
 // (L200-202), forward substitution x_c = (b_c - sum_{m<c} x_m L[c][m]) / L[c][c]
-// per row.  Register-resident, blocked right-looking over 8-column panels: X stays
-// in the accumulator fragments; for each panel the owner warps copy it to a shared
-// panel buffer, one thread per row solves it against the 8x8 diagonal block of L,
-// and every warp updates its trailing column blocks with FP64 DMMA
-// (X[:, later] -= X[:, panel] L[later, panel]^T).  On entry x holds acc (has_acc) or
-// scratch; it is overwritten with the solved block.
+// per row, blocked right-looking over 8-column panels: a panel is solved by the four
+// lanes of a quad that hold a row (shuffles), then the warp updates its later column
+// blocks with FP64 DMMA (X[:, later] -= X[:, panel] L[later, panel]^T).  No CTA
+// barrier inside the panel loop.  On entry acc holds the GEMM part (has_acc) or is
+// unused; the block is written back to X.
 template <int BS>
-__device__ __forceinline__ void solve_block(const Ctx<BS>& c, Acc<BS>& x, bool has_acc, double* X, int ldx,
+__device__ __forceinline__ void solve_block(const Ctx<BS>& c, Acc<BS>& acc, bool has_acc, double* X, int ldx,
                                             const double* Ld, int ldl) {
   using C = Cfg<BS>;
-  constexpr int P = C::kPitch;
-  const int tid = threadIdx.x, wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  constexpr int P = C::kPitch, NB = BS / 8;
+  const int tid = threadIdx.x, g = c.lane >> 2, t = c.lane & 3;
   double* lb = c.lbuf;  // L block; column BS holds 1/L[c][c]
-  double* pans = c.pans; // 2 panels of BS x kPanelPitch
-  // x := X - acc in place (acc is consumed; one 72-register array live)
-  {
-    const int wm0 = wm * C::WM, wn0 = wn * C::WN;
+  // every warp must be done with lbuf (previous job / previous column block)
+  bar_sync(kBarCompute, kComputeThreads);
+  if (has_acc) {  // X -= acc in the GEMM's fragment layout, through global memory (L2)
+    const int wm = c.warp >> 2, wn = c.warp & 3;
 #pragma unroll
     for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) {
-        const double2 v = __ldcg(reinterpret_cast<const double2*>(X + (int64_t)(wm0 + mi * 8 + g) * ldx + wn0 +
-                                                                  ni * 8 + 2 * t));
-        x[mi][ni][0] = has_acc ? v.x - x[mi][ni][0] : v.x;
-        x[mi][ni][1] = has_acc ? v.y - x[mi][ni][1] : v.y;
+        double2* px = reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN + ni * 8 +
+                                                 2 * t);
+        double2 v = __ldcg(px);
+        v.x -= acc[mi][ni][0];
+        v.y -= acc[mi][ni][1];
+        __stcg(px, v);
       }
   }
-  // buf/lbuf reuse: every warp must be done with the TMA ring and the previous lbuf use.
-  bar_sync(kBarCompute, kComputeThreads);
   load_block<BS>(lb, Ld, ldl);
   if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
-#pragma unroll 1
-  for (int p = 0; p < BS / 8; ++p) {
-    const int c0 = 8 * p;
-    double* pan = pans + (p & 1) * BS * kPanelPitch;
-    frag_to_panel(c, x, p, pan);
-    bar_sync(kBarCompute, kComputeThreads);  // (also publishes lb on p == 0)
-    if (tid < BS) {  // substitution of row tid against L[c0:c0+8, c0:c0+8]
-      double v[8];
-      double* pr = pan + tid * kPanelPitch;
+  bar_sync(kBarCompute, kComputeThreads);
+  if (c.warp < BS / 16) {
+    RowX<BS> x;
+    const int r0 = 16 * c.warp;
 #pragma unroll
-      for (int j = 0; j < 8; j += 2) {
-        const double2 q = *reinterpret_cast<const double2*>(pr + j);
-        v[j] = q.x;
-        v[j + 1] = q.y;
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb) {
+        const double2 v =
+            __ldcg(reinterpret_cast<const double2*>(X + (int64_t)(r0 + 8 * mi + g) * ldx + 8 * cb + 2 * t));
+        x.v[mi][cb][0] = v.x;
+        x.v[mi][cb][1] = v.y;
       }
+    const int qbase = c.lane & ~3;
+#pragma unroll
+    for (int p = 0; p < NB; ++p) {
+      const int c0 = 8 * p;
+      // (a) substitution inside the panel: column c0+j is held by lane t = j/2, slot j%2
 #pragma unroll
       for (int j = 0; j < 8; ++j) {
-        v[j] *= lb[(c0 + j) * P + BS];
+        const double rd = lb[(c0 + j) * P + BS];
+        const double l0 = lb[(c0 + 2 * t) * P + c0 + j], l1 = lb[(c0 + 2 * t + 1) * P + c0 + j];
 #pragma unroll
-        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], lb[(c0 + j2) * P + c0 + j], v[j2]);
+        for (int mi = 0; mi < 2; ++mi) {
+          const double xj = __shfl_sync(0xffffffffu, x.v[mi][p][j & 1], qbase | (j >> 1)) * rd;
+          if (t == (j >> 1)) x.v[mi][p][j & 1] = xj;
+          if (2 * t > j) x.v[mi][p][0] = fma(-xj, l0, x.v[mi][p][0]);
+          if (2 * t + 1 > j) x.v[mi][p][1] = fma(-xj, l1, x.v[mi][p][1]);
+        }
       }
+      // (b) later column blocks: x[:, cb] -= x[:, p] L[cb rows, p cols]^T
 #pragma unroll
-      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(pr + j) = make_double2(v[j], v[j + 1]);
-    }
-    bar_sync(kBarCompute, kComputeThreads);
-    panel_to_frag(c, x, p, pan);
-    // trailing update of this warp's column blocks cb > p
-    double a[C::MI][2];
+      for (int cb = p + 1; cb < NB; ++cb) {
+        const double2 bv = *reinterpret_cast<const double2*>(lb + (8 * cb + g) * P + c0 + 2 * t);
 #pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) {
-      const double* pr = pan + (wm * C::WM + mi * 8 + g) * kPanelPitch;
-      a[mi][0] = -pr[t];
-      a[mi][1] = -pr[t + 4];
-    }
-#pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) {
-      const int cb = wn * C::NI + ni;
-      if (cb <= p) continue;
-      const double* lr = lb + (cb * 8 + g) * P + c0;
-      const double b0 = lr[t], b1 = lr[t + 4];
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) {
-        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][0], b0);
-        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][1], b1);
+        for (int mi = 0; mi < 2; ++mi) {
+          dmma884(x.v[mi][cb][0], x.v[mi][cb][1], -x.v[mi][p][0], bv.x);
+          dmma884(x.v[mi][cb][0], x.v[mi][cb][1], -x.v[mi][p][1], bv.y);
+        }
       }
     }
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb)
+        __stcg(reinterpret_cast<double2*>(X + (int64_t)(r0 + 8 * mi + g) * ldx + 8 * cb + 2 * t),
+               make_double2(x.v[mi][cb][0], x.v[mi][cb][1]));
   }
-  frag_store(c, x, X, ldx, false);
-  bar_sync(kBarCompute, kComputeThreads);  // buf / lbuf free for the next user
+  bar_sync(kBarCompute, kComputeThreads);  // lbuf free for the next user; X stores issued
 }
 
 // Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
@@ -485,32 +494,32 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
     double* pan = pans + (p & 1) * BS * kPanelPitch;
     frag_to_panel(c, x, p, pan);
     bar_sync(kBarCompute, kComputeThreads);
-    if (c.warp == 0) {  // 8x8 diagonal block in registers: lane r < 8 holds row c0 + r
-      double v[8];
-      double* pr = pan + (c0 + (lane & 7)) * kPanelPitch;
+    if (tid == 0) {  // 8x8 diagonal block: one thread, all 36 entries in registers
+      double v[8][8];
 #pragma unroll
-      for (int j = 0; j < 8; ++j) v[j] = pr[j];
+      for (int r = 0; r < 8; ++r)
+#pragma unroll
+        for (int q = 0; q <= r; ++q) v[r][q] = pan[(c0 + r) * kPanelPitch + q];
 #pragma unroll
       for (int j = 0; j < 8; ++j) {
-        const double d = __shfl_sync(0xffffffffu, v[j], j);
-        if (lane == 0 && !(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
-        // one rsqrt on the column's dependency chain instead of sqrt followed by a
-        // division: L[j][j] = d * d^{-1/2}, scale = d^{-1/2} (exact for the perfect
-        // squares of the integer family; within an ulp otherwise)
+        const double d = v[j][j];
+        if (!(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
+        // one rsqrt on the column's dependency chain: L[j][j] = d * d^{-1/2}, scale = d^{-1/2}
+        // (exact for the perfect squares of the integer family; within an ulp otherwise)
         const double rl = rsqrt(d);
-        const double ljj = d * rl;
-        if (lane == j) v[j] = ljj;
-        if (lane > j) v[j] *= rl;
-        if (lane == 0) rdiag[j] = rl;
+        v[j][j] = d * rl;
+        rdiag[j] = rl;
 #pragma unroll
-        for (int q = j + 1; q < 8; ++q) {
-          const double lqj = __shfl_sync(0xffffffffu, v[j], q);
-          if (lane >= q) v[q] = fma(-v[j], lqj, v[q]);
-        }
+        for (int r = j + 1; r < 8; ++r) v[r][j] *= rl;
+#pragma unroll
+        for (int r = j + 1; r < 8; ++r)
+#pragma unroll
+          for (int q = j + 1; q <= r; ++q) v[r][q] = fma(-v[r][j], v[q][j], v[r][q]);
       }
-      if (lane < 8)
 #pragma unroll
-        for (int j = 0; j < 8; ++j) pr[j] = v[j];
+      for (int r = 0; r < 8; ++r)
+#pragma unroll
+        for (int q = 0; q <= r; ++q) pan[(c0 + r) * kPanelPitch + q] = v[r][q];
     }
     bar_sync(kBarCompute, kComputeThreads);
     const int r = c0 + 8 + tid;
