@@ -11,7 +11,7 @@ import ctypes
 import os
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libchol_b200.so")
+LIB_PATH = os.environ.get("CHOL_LIB_OVERRIDE") or os.path.join(_HERE, "libchol_b200.so")  # override: A/B experiments only
 
 POLICY_DYNAMIC, POLICY_CP_PRIORITY, POLICY_STATIC = 0, 1, 2
 EXEC_SCHEDULER, EXEC_HOST = 0, 1

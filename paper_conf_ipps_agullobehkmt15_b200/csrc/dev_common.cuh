@@ -68,6 +68,9 @@ __device__ __forceinline__ double2 lds128(uint32_t addr) {
 }
 
 // ---------------------------------------------------------------- named barriers
+__device__ __forceinline__ void bar_arrive(uint32_t id, uint32_t nthreads) {
+  asm volatile("bar.arrive %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
+}
 __device__ __forceinline__ void bar_sync(uint32_t id, uint32_t nthreads) {
   asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
 }

@@ -162,11 +162,11 @@ __device__ __forceinline__ int* prod_issued_ptr(int4* jdesc) { return reinterpre
 template <int BS>
 __device__ void producer_loop(Ctx<BS>& c) {
   uint32_t q = 0, pit = 0, tcount = 0;
-  volatile int* issued = prod_issued_ptr(c.jdesc);
+  volatile int* issued = prod_issued_ptr(c.jdesc());
   while (true) {
     const int e = q & 1;
-    mbar_wait(&c.jfull[e], (q >> 1) & 1);
-    const int4 d0 = c.jdesc[e * 3], d1 = c.jdesc[e * 3 + 1];
+    mbar_wait(&c.jfull()[e], (q >> 1) & 1);
+    const int4 d0 = c.jdesc()[e * 3], d1 = c.jdesc()[e * 3 + 1];
     const int job = d0.x, type = d0.y & 0xff, skip = d0.y >> 8;
     if (job < 0) break;
     fence_proxy_async();  // operands written by generic stores (this or other SMs)
@@ -192,18 +192,23 @@ __device__ void producer_loop(Ctx<BS>& c) {
         // stages first (they only need ring space), then the C prefetch into lbuf once
         // the previous job has released lbuf, then the rest
         produce_range(c, pit, nst, ta, ra, tb, rb, kb, 0, kStages);
-        if (q > 0) mbar_wait(c.lfree, (q - 1) & 1);
+        if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
         prefetch_c_issue(c, tcb, cr, cc);
         produce_range(c, pit, nst, ta, ra, tb, rb, kb, kStages, nst);
         pit += nst;
       } else if (type == J_TRSM) {  // row slab (i, k, slab): mainloop cb reads X[:, :cb] (solved)
         const int nbb = c.nb / BS;
         for (int cb = 1; cb < nbb; ++cb) {
-          mbar_wait(c.tstep, tcount & 1);
+          // K chunks of the column blocks solved before cb-1 are final already: stream
+          // them into the ring while the compute warps still solve block cb-1; only the
+          // last BS/BK stages (column block cb-1) wait for its tstep.  Same K order.
+          const int nst = cb * BS / BK, nold = (cb - 1) * BS / BK;
+          const int64_t ta = c.slot(d0.z, d1.x), tb = c.slot(d1.x, d1.x);
+          produce_range(c, pit, nst, ta, d1.y * BS, tb, cb * BS, 0, 0, nold);
+          mbar_wait(c.tstep(), tcount & 1);
           ++tcount;
           fence_proxy_async();
-          const int nst = cb * BS / BK;
-          produce_range(c, pit, nst, c.slot(d0.z, d1.x), d1.y * BS, c.slot(d1.x, d1.x), cb * BS, 0, 0, nst);
+          produce_range(c, pit, nst, ta, d1.y * BS, tb, cb * BS, 0, nold, nst);
           pit += nst;
         }
       }
@@ -285,38 +290,44 @@ __device__ void watcher_loop(const DevSched& d) {
 template <int BS>
 __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int type, const int4& d0, const int4& d1,
                                             int* info) {
-  Acc<BS> acc;
+  // accumulators are declared per branch: one function-wide Acc makes ptxas keep its
+  // registers reserved across the register-hungry in-block routines (spills)
   if (type == J_UPD) {
+    Acc<BS> acc;
     const int i = d0.z, j = d0.w, k = d1.x, bm = d1.y, bn = d1.z;
     gemm_consume(c, c.nb / BK, acc);
     epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
     (void)k;
   } else if (type == J_PUPD) {
+    Acc<BS> acc;
     const int k = d1.x, r = d1.z, q = d1.w;
     gemm_consume(c, BS / BK, acc);
     epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);
   } else if (type == J_TRSM) {
+    Acc<BS> acc;
     const int i = d0.z, k = d1.x, slab = d1.y, nbb = c.nb / BS;
     double* X = c.tile(i, k) + (int64_t)slab * BS * c.nb;
     const double* L = c.tile(k, k);
     for (int cb = 0; cb < nbb; ++cb) {
       if (cb > 0) gemm_consume(c, cb * BS / BK, acc);
-      solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+      if (cb > 0) acc_sub_global(c, acc, X + cb * BS, c.nb);
+      solve_block(c, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
       if (cb + 1 < nbb) {
         // X[:, cb] is read by the producer's TMA for the next column block
         __threadfence();
         fence_proxy_async();
         __syncwarp();
-        if (c.lane == 0) mbar_arrive(c.tstep);
+        if (c.lane == 0) mbar_arrive(c.tstep());
       }
     }
   } else if (type == J_TU) {
+    Acc<BS> acc;
     const int i = d0.z, k = d1.x, sl = d1.z, c2 = d1.w;
     gemm_consume(c, BS / BK, acc);
     epi_sub_global(c, acc, c.tile(i, k) + (int64_t)sl * BS * c.nb + c2 * BS, c.nb, false);
   } else if (type == J_TS) {
     const int i = d0.z, k = d1.x, cb = d1.y, sl = d1.z;
-    solve_block(c, acc, false, c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
+    solve_block(c, c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
                 c.tile(k, k) + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
   } else if (type == J_RECV) {  // copy BS rows of a remote panel tile into the local cache
     const int i = d0.z, j = d0.w, sl = d1.y, owner = d1.z;
@@ -334,24 +345,24 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
   uint32_t q = 0;
   while (true) {
     const int e = q & 1;
-    mbar_wait(&c.jfull[e], (q >> 1) & 1);
-    const int4 d0 = c.jdesc[e * 3], d1 = c.jdesc[e * 3 + 1];
+    mbar_wait(&c.jfull()[e], (q >> 1) & 1);
+    const int4 d0 = c.jdesc()[e * 3], d1 = c.jdesc()[e * 3 + 1];
     if (d0.x < 0) break;
     if (c.warp == 0 && c.lane == 0) {
       const unsigned long long t0 = globaltimer_ns();
-      c.jdesc[e * 3 + 2] = make_int4((int)(t0 & 0xffffffffull), (int)(t0 >> 32), 0, 0);
+      c.jdesc()[e * 3 + 2] = make_int4((int)(t0 & 0xffffffffull), (int)(t0 >> 32), 0, 0);
     }
     const int type = d0.y & 0xff, skip = d0.y >> 8;
     if (!skip) compute_job(c, d, type, d0, d1, info);
     __syncwarp();
     if (c.lane == 0) {
-      mbar_arrive(c.lfree);  // lbuf (C block / L block / rdiag) no longer needed
+      mbar_arrive(c.lfree());  // lbuf (C block / L block / rdiag) no longer needed
       if (c.warp == 0) {     // end time of the job as seen by warp 0
         const unsigned long long t1 = globaltimer_ns();
-        c.jdesc[e * 3 + 2].z = (int)(t1 & 0xffffffffull);
-        c.jdesc[e * 3 + 2].w = (int)(t1 >> 32);
+        c.jdesc()[e * 3 + 2].z = (int)(t1 & 0xffffffffull);
+        c.jdesc()[e * 3 + 2].w = (int)(t1 >> 32);
       }
-      mbar_arrive(&c.jdone[e]);  // the job's global stores precede this release
+      mbar_arrive(&c.jdone()[e]);  // the job's global stores precede this release
     }
     ++q;
   }
@@ -404,9 +415,9 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
     // 1. retire finished jobs in order
     while (q_done < q_issue) {
       const int e = q_done & 1;
-      if (!mbar_try_wait(smem_u32(&c.jdone[e]), (q_done >> 1) & 1)) break;
+      if (!mbar_try_wait(smem_u32(&c.jdone()[e]), (q_done >> 1) & 1)) break;
       if (lane == 0) {
-        const int4 tt = c.jdesc[e * 3 + 2];
+        const int4 tt = c.jdesc()[e * 3 + 2];
         const uint64_t t0 = (uint64_t)(uint32_t)tt.x | ((uint64_t)(uint32_t)tt.y << 32);
         const uint64_t t1 = (uint64_t)(uint32_t)tt.z | ((uint64_t)(uint32_t)tt.w << 32);
         complete_job(d, sp, pending[e], t0, t1);
@@ -416,15 +427,15 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
     }
     // 2. claim the next job once the ring has room and the producer is done with the
     //    running job's loads (late claim keeps critical-path hops short)
-    if (q_issue - q_done < 2 && (q_issue == q_done || ld_volatile(prod_issued_ptr(c.jdesc)) >= (int)q_issue)) {
+    if (q_issue - q_done < 2 && (q_issue == q_done || ld_volatile(prod_issued_ptr(c.jdesc())) >= (int)q_issue)) {
       const int job = try_pop(d, latency_worker, lane);
       if (job >= 0) {
         const int e = q_issue & 1;
         if (lane == 0) {
           __threadfence();  // acquire: the job's inputs were published before it was enqueued
           const Job jb = d.jobs[job];
-          write_desc(&c.jdesc[e * 3], job, jb, ld_volatile(sp.info) != INT_MAX);
-          mbar_arrive(&c.jfull[e]);
+          write_desc(&c.jdesc()[e * 3], job, jb, ld_volatile(sp.info) != INT_MAX);
+          mbar_arrive(&c.jfull()[e]);
         }
         __syncwarp();
         pending[e] = job;
@@ -437,8 +448,8 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
     if (q_done == q_issue && ld_volatile(d.finished)) {
       if (lane == 0) {
         const int e = q_issue & 1;
-        c.jdesc[e * 3] = make_int4(-1, 0, 0, 0);
-        mbar_arrive(&c.jfull[e]);
+        c.jdesc()[e * 3] = make_int4(-1, 0, 0, 0);
+        mbar_arrive(&c.jfull()[e]);
       }
       __syncwarp();
       break;

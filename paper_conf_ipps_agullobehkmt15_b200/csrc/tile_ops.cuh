@@ -25,6 +25,7 @@ constexpr int kStages = 5;
 constexpr int BK = 16;  // doubles per TMA box row (128 bytes)
 constexpr int kBarCompute = 1;  // named barrier id: compute warps only
 constexpr int kBarAll = 2;      // named barrier id: all warps
+constexpr int kBarDiag = 3;     // named barrier id: panel owner warp -> diagonal-factor warp (potf2_block)
 
 
 template <int BS>
@@ -52,19 +53,30 @@ struct Ctx {
   const CUtensorMap* map;
   double* tiles;
   int nb, N;
-  char* pipe;      // kStages x {A, B} operand buffers (1024-aligned)
-  double* buf;     // BS x kPitch solve/factor buffer (aliases pipe)
-  double* lbuf;    // BS x kPitch (transposed L block)
-  uint64_t* full;  // kStages
-  uint64_t* empty; // kStages
-  uint64_t* cbar;  // C-block prefetch (TMA -> lbuf)
+  // Shared-memory regions: fixed offsets from the 1024-aligned dynamic smem base,
+  // recomputed on use (the compiler rematerialises them instead of holding ~24
+  // registers of pointers live through the register-hungry in-block routines).
+  __device__ static char* base() {
+    extern __shared__ __align__(1024) char smem_raw[];
+    return reinterpret_cast<char*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
+  }
+  __device__ static char* bars() { return base() + Cfg<BS>::kPipeBytes + Cfg<BS>::kBufBytes + Cfg<BS>::kPanBytes; }
+  __device__ char* pipe() const { return base(); }  // kStages x {A, B} operand buffers
+  __device__ double* buf() const { return reinterpret_cast<double*>(base()); }  // solve buffer (aliases pipe)
+  __device__ double* lbuf() const { return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes); }  // BS x kPitch
+  __device__ double* pans() const {  // two BS x 8 panels for the in-block solves
+    return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes + Cfg<BS>::kBufBytes);
+  }
+  __device__ uint64_t* full() const { return reinterpret_cast<uint64_t*>(bars()); }  // kStages
+  __device__ uint64_t* empty() const { return full() + kStages; }                     // kStages
+  __device__ uint64_t* cbar() const { return empty() + kStages; }  // C-block prefetch (TMA -> lbuf)
   // warp-specialised persistent kernel only (sched.cu):
-  uint64_t* jfull; // [2] job descriptor ready (scheduler -> producer, compute)
-  uint64_t* jdone; // [2] job finished (compute -> scheduler)
-  uint64_t* lfree; // lbuf released by the current job (compute -> producer)
-  uint64_t* tstep; // TRSM column block solved and stored (compute -> producer)
-  int4* jdesc;     // [2] x 3 int4 job descriptors
-  double* pans;    // two BS x 8 panels for the in-block solves
+  __device__ uint64_t* jfull() const { return cbar() + 1; }  // [2] job descriptor ready
+  __device__ uint64_t* jdone() const { return jfull() + 2; } // [2] job finished (compute -> scheduler)
+  __device__ uint64_t* lfree() const { return jdone() + 2; } // lbuf released (compute -> producer)
+  __device__ uint64_t* tstep() const { return lfree() + 1; } // TRSM column block stored (compute -> producer)
+  // 2*kStages + 7 = 17 barriers = 136 bytes; then 2 x 3 int4 job descriptors + producer progress word
+  __device__ int4* jdesc() const { return reinterpret_cast<int4*>(bars() + 160); }
   uint32_t it;     // stages consumed so far
   uint32_t cphase; // parity of the next cbar completion
   int warp, lane;
@@ -81,45 +93,29 @@ struct Ctx {
 template <int BS>
 __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tiles, int nb, int N,
                                             const int* slot_map = nullptr) {
-  extern __shared__ __align__(1024) char smem_raw[];
-  using C = Cfg<BS>;
   Ctx<BS> c;
-  char* base = reinterpret_cast<char*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
   c.map = map;
   c.tiles = tiles;
   c.slot_map = slot_map;
   c.nb = nb;
   c.N = N;
-  c.pipe = base;
-  c.buf = reinterpret_cast<double*>(base);
-  c.lbuf = reinterpret_cast<double*>(base + C::kPipeBytes);
-  c.pans = reinterpret_cast<double*>(base + C::kPipeBytes + C::kBufBytes);
-  char* bars = base + C::kPipeBytes + C::kBufBytes + C::kPanBytes;  // kBarBytes
-  c.full = reinterpret_cast<uint64_t*>(bars);
-  c.empty = c.full + kStages;
-  c.cbar = c.empty + kStages;
-  c.jfull = c.cbar + 1;
-  c.jdone = c.jfull + 2;
-  c.lfree = c.jdone + 2;
-  c.tstep = c.lfree + 1;  // 2*kStages + 7 = 17 barriers = 136 bytes
-  c.jdesc = reinterpret_cast<int4*>(bars + 160);  // 2 x 3 int4 + producer progress word
-  if (threadIdx.x == 0) *reinterpret_cast<int*>(c.jdesc + 6) = 0;
+  if (threadIdx.x == 0) *reinterpret_cast<int*>(c.jdesc() + 6) = 0;
   c.it = 0;
   c.cphase = 0;
   c.warp = threadIdx.x >> 5;
   c.lane = threadIdx.x & 31;
   if (threadIdx.x == 0) {
     for (int s = 0; s < kStages; ++s) {
-      mbar_init(&c.full[s], 1);
-      mbar_init(&c.empty[s], kComputeWarps);
+      mbar_init(&c.full()[s], 1);
+      mbar_init(&c.empty()[s], kComputeWarps);
     }
-    mbar_init(c.cbar, 1);
+    mbar_init(c.cbar(), 1);
     for (int e = 0; e < 2; ++e) {
-      mbar_init(&c.jfull[e], 1);
-      mbar_init(&c.jdone[e], kComputeWarps);
+      mbar_init(&c.jfull()[e], 1);
+      mbar_init(&c.jdone()[e], kComputeWarps);
     }
-    mbar_init(c.lfree, kComputeWarps);
-    mbar_init(c.tstep, kComputeWarps);
+    mbar_init(c.lfree(), kComputeWarps);
+    mbar_init(c.tstep(), kComputeWarps);
     fence_mbar_init();
   }
   if (c.issuer() && map) tma_prefetch_desc(map);
@@ -145,10 +141,10 @@ struct CPrefetch {
 template <int BS>
 __device__ __forceinline__ void prefetch_c_issue(Ctx<BS>& c, int64_t tile, int r0, int c0) {
   fence_proxy_async();
-  mbar_arrive_expect_tx(c.cbar, BS * BS * 8);
-  char* dst = reinterpret_cast<char*>(c.lbuf);
+  mbar_arrive_expect_tx(c.cbar(), BS * BS * 8);
+  char* dst = reinterpret_cast<char*>(c.lbuf());
 #pragma unroll 1
-  for (int b = 0; b < BS / 16; ++b) tma_load_3d(dst + b * BS * 128, c.map, c.cbar, c0 + 16 * b, r0, (int)tile);
+  for (int b = 0; b < BS / 16; ++b) tma_load_3d(dst + b * BS * 128, c.map, c.cbar(), c0 + 16 * b, r0, (int)tile);
 }
 
 template <int BS>
@@ -160,11 +156,11 @@ template <int BS>
 __device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, int ra, int64_t tb, int rb, int kk) {
   using C = Cfg<BS>;
   const uint32_t st = q % kStages, ph = (q / kStages) & 1;
-  mbar_wait(&c.empty[st], ph ^ 1);  // the previous use of this buffer was released by all warps
-  mbar_arrive_expect_tx(&c.full[st], 2 * C::kOpBytes);
-  char* sa = c.pipe + st * 2 * C::kOpBytes;
-  tma_load_3d(sa, c.map, &c.full[st], kk, ra, (int)ta);
-  tma_load_3d(sa + C::kOpBytes, c.map, &c.full[st], kk, rb, (int)tb);
+  mbar_wait(&c.empty()[st], ph ^ 1);  // the previous use of this buffer was released by all warps
+  mbar_arrive_expect_tx(&c.full()[st], 2 * C::kOpBytes);
+  char* sa = c.pipe() + st * 2 * C::kOpBytes;
+  tma_load_3d(sa, c.map, &c.full()[st], kk, ra, (int)ta);
+  tma_load_3d(sa + C::kOpBytes, c.map, &c.full()[st], kk, rb, (int)tb);
 }
 
 // Consume one TMA stage: wait for it, DMMA it into acc, release it to the producer.
@@ -173,9 +169,9 @@ __device__ __forceinline__ void consume_stage(Ctx<BS>& c, uint32_t q, Acc<BS>& a
   using C = Cfg<BS>;
   const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
   const uint32_t st = q % kStages, ph = (q / kStages) & 1;
-  mbar_wait(&c.full[st], ph);
-  const uint32_t As = smem_u32(c.pipe) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
-  const uint32_t Bs = smem_u32(c.pipe) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
+  mbar_wait(&c.full()[st], ph);
+  const uint32_t As = smem_u32(c.pipe()) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
+  const uint32_t Bs = smem_u32(c.pipe()) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
   uint32_t dep = 0;
 #pragma unroll
   for (int h = 0; h < 2; ++h) {
@@ -207,7 +203,7 @@ __device__ __forceinline__ void consume_stage(Ctx<BS>& c, uint32_t q, Acc<BS>& a
   // cannot issue before the loads complete and a TMA refill can never overwrite
   // data a lane has not read yet.
   __syncwarp();
-  if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty[st]);
+  if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty()[st]);
 }
 
 template <int BS>
@@ -257,9 +253,9 @@ __device__ __forceinline__ void epi_sub_global(Ctx<BS>& c, const Acc<BS>& acc, d
                                                bool lower_only) {
   using C = Cfg<BS>;
   const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
-  mbar_wait(c.cbar, c.cphase);
+  mbar_wait(c.cbar(), c.cphase);
   c.cphase ^= 1;
-  const uint32_t cs = smem_u32(c.lbuf);
+  const uint32_t cs = smem_u32(c.lbuf());
 #pragma unroll
   for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
@@ -387,37 +383,42 @@ struct RowX {
   double v[2][NB][2];
 };
 
-// X <- (X - acc) * Ld^{-T} for one BS x BS block X (ld ldx) against the lower
+// X -= acc for one BS x BS block X (ld ldx), acc in the GEMM's fragment layout,
+// through global memory (L2): the GEMM part of a TRSM column block, applied before its
+// in-block solve (solve_block's barriers order these stores before the solve's loads).
+template <int BS>
+__device__ __forceinline__ void acc_sub_global(const Ctx<BS>& c, const Acc<BS>& acc, double* X, int ldx) {
+  using C = Cfg<BS>;
+  const int g = c.lane >> 2, t = c.lane & 3;
+  const int wm = c.warp >> 2, wn = c.warp & 3;
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      double2* px = reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN + ni * 8 +
+                                               2 * t);
+      double2 v = __ldcg(px);
+      v.x -= acc[mi][ni][0];
+      v.y -= acc[mi][ni][1];
+      __stcg(px, v);
+    }
+}
+
+// X <- X * Ld^{-T} for one BS x BS block X (ld ldx) against the lower
 // triangular BS x BS diagonal block Ld (ld ldl): the in-block part of TRSM
 // (L200-202), forward substitution x_c = (b_c - sum_{m<c} x_m L[c][m]) / L[c][c]
 // per row, blocked right-looking over 8-column panels: a panel is solved by the four
 // lanes of a quad that hold a row (shuffles), then the warp updates its later column
 // blocks with FP64 DMMA (X[:, later] -= X[:, panel] L[later, panel]^T).  No CTA
-// barrier inside the panel loop.  On entry acc holds the GEMM part (has_acc) or is
-// unused; the block is written back to X.
+// barrier inside the panel loop.  The block is written back to X.
 template <int BS>
-__device__ __forceinline__ void solve_block(const Ctx<BS>& c, Acc<BS>& acc, bool has_acc, double* X, int ldx,
-                                            const double* Ld, int ldl) {
+__device__ __forceinline__ void solve_block(const Ctx<BS>& c, double* X, int ldx, const double* Ld, int ldl) {
   using C = Cfg<BS>;
   constexpr int P = C::kPitch, NB = BS / 8;
   const int tid = threadIdx.x, g = c.lane >> 2, t = c.lane & 3;
-  double* lb = c.lbuf;  // L block; column BS holds 1/L[c][c]
+  double* lb = c.lbuf();  // L block; column BS holds 1/L[c][c]
   // every warp must be done with lbuf (previous job / previous column block)
   bar_sync(kBarCompute, kComputeThreads);
-  if (has_acc) {  // X -= acc in the GEMM's fragment layout, through global memory (L2)
-    const int wm = c.warp >> 2, wn = c.warp & 3;
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) {
-        double2* px = reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN + ni * 8 +
-                                                 2 * t);
-        double2 v = __ldcg(px);
-        v.x -= acc[mi][ni][0];
-        v.y -= acc[mi][ni][1];
-        __stcg(px, v);
-      }
-  }
   load_block<BS>(lb, Ld, ldl);
   if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
   bar_sync(kBarCompute, kComputeThreads);
@@ -452,7 +453,8 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, Acc<BS>& acc, bool
       }
       // (b) later column blocks: x[:, cb] -= x[:, p] L[cb rows, p cols]^T
 #pragma unroll
-      for (int cb = p + 1; cb < NB; ++cb) {
+      for (int cb = 1; cb < NB; ++cb) {  // constant trip count: fully unrolled, x stays in registers
+        if (cb <= p) continue;
         const double2 bv = *reinterpret_cast<const double2*>(lb + (8 * cb + g) * P + c0 + 2 * t);
 #pragma unroll
         for (int mi = 0; mi < 2; ++mi) {
@@ -471,101 +473,168 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, Acc<BS>& acc, bool
   bar_sync(kBarCompute, kComputeThreads);  // lbuf free for the next user; X stores issued
 }
 
+// One thread factors the 8x8 lower block dd (pitch 8) in registers, column by column
+// (SURVEY §8c column algorithm), writing L back to dd and 1/L[j][j] to rdv.
+__device__ __forceinline__ void factor_8x8(double* dd, double* rdv, int* info, int col) {
+  double v[8][8];
+#pragma unroll
+  for (int r = 0; r < 8; ++r)
+#pragma unroll
+    for (int q = 0; q <= r; ++q) v[r][q] = dd[r * 8 + q];
+#pragma unroll
+  for (int j = 0; j < 8; ++j) {
+    const double d = v[j][j];
+    if (!(d > 0.0)) atomicMin(info, col + j + 1);
+    // one rsqrt on the dependency chain: L[j][j] = d * d^{-1/2}, scale = d^{-1/2}
+    // (exact for the perfect squares of the integer family; within an ulp otherwise)
+    const double rl = rsqrt(d);
+    v[j][j] = d * rl;
+    rdv[j] = rl;
+#pragma unroll
+    for (int r = j + 1; r < 8; ++r) v[r][j] *= rl;
+#pragma unroll
+    for (int r = j + 1; r < 8; ++r)
+#pragma unroll
+      for (int q = j + 1; q <= r; ++q) v[r][q] = fma(-v[r][j], v[q][j], v[r][q]);
+  }
+#pragma unroll
+  for (int r = 0; r < 8; ++r)
+#pragma unroll
+    for (int q = 0; q <= r; ++q) dd[r * 8 + q] = v[r][q];
+}
+
 // Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
-// L196-199).  Register-resident like solve_block: for each 8-column panel, the owner
-// warps copy it to shared memory, warp 0 factors its 8x8 diagonal block in registers
-// (column algorithm of SURVEY §8c, lanes = rows, shuffles), one thread per row
-// solves the rows below, and every warp applies the rank-8 update to its lower
-// blocks with FP64 DMMA.  A pivot !(d > 0) records info = col0 + c + 1 with
-// atomicMin (LAPACK convention, reading R6).  The strictly upper blocks are never
-// stored; the upper halves of diagonal 8x8 blocks are scratch (never read).
+// L196-199), blocked right-looking over 8-column panels p, register resident in a
+// row layout with paired row blocks: warp w < NB/2 owns the 8-row blocks rb = w and
+// rb = NB-1-w (13 of the 78 lower 8x8 blocks each for BS = 96: balanced work, and
+// NB+1 fragment slots per thread instead of 2*NB -- column cb of the first block in
+// slot cb, of the second in slot NB-cb, disjoint since cb <= w < NB-cb).  Per panel:
+//   (1) the owner of the diagonal block updates it first and hands it to the idle
+//       warp 7 (named barrier kBarDiag), which factors it with one thread in
+//       registers (column algorithm of SURVEY §8c, one rsqrt per column) while the
+//       other warps finish their updates (one-panel lookahead);
+//   (2) after a compute barrier every warp solves its rows below against L_pp (quad
+//       shuffles) and publishes them to shared memory;
+//   (3) after a second barrier every warp applies the rank-8 update to its lower
+//       blocks with FP64 DMMA (A operand = its own solved fragments).
+// A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
+// reading R6).  Only the lower blocks are stored; the upper halves of the diagonal 8x8
+// blocks are never read (stored back as the input values).
 template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
-  using C = Cfg<BS>;
-  const int tid = threadIdx.x, lane = c.lane, wm = c.warp >> 2, wn = c.warp & 3, g = lane >> 2, t = lane & 3;
-  double* pans = c.pans;
-  double* rdiag = c.lbuf;  // 1/L[c][c] of the current panel (8 doubles)
-  Acc<BS> x;
-  frag_load(c, x, A, lda);
-  bar_sync(kBarCompute, kComputeThreads);  // buf / lbuf reuse
+  constexpr int NB = BS / 8;
+  static_assert(NB % 2 == 0 && NB / 2 <= 7, "paired row blocks; warp 7 factors the diagonal blocks");
+  const int g = c.lane >> 2, t = c.lane & 3, qbase = c.lane & ~3;
+  double* dd = c.lbuf();        // 8 x 8 diagonal block (pitch 8) + 8 reciprocals
+  double* rdv = c.lbuf() + 64;
+  bar_sync(kBarCompute, kComputeThreads);  // lbuf / pans reuse
+  if (c.warp == 7) {
+    // factor warp: its own loop, disjoint from the row-block code (register pressure)
 #pragma unroll 1
-  for (int p = 0; p < BS / 8; ++p) {
-    const int c0 = 8 * p;
-    double* pan = pans + (p & 1) * BS * kPanelPitch;
-    frag_to_panel(c, x, p, pan);
+    for (int p = 0; p < NB; ++p) {
+      bar_sync(kBarDiag, 64);  // diagonal block p is in dd
+      if (c.lane == 0) factor_8x8(dd, rdv, info, col0 + 8 * p);
+      bar_sync(kBarCompute, kComputeThreads);  // L_pp published
+      bar_sync(kBarCompute, kComputeThreads);  // panel p published
+    }
     bar_sync(kBarCompute, kComputeThreads);
-    if (tid == 0) {  // 8x8 diagonal block: one thread, all 36 entries in registers
-      double v[8][8];
+    return;
+  }
+  const bool active = c.warp < NB / 2;
+  const int rb0 = c.warp, rb1 = NB - 1 - c.warp;  // the warp's two row blocks
+  double x[NB + 1][2];
+#define RB(mi) ((mi) == 0 ? rb0 : rb1)
+#define SL(mi, cb) ((mi) == 0 ? (cb) : NB - (cb))
+  if (active) {
 #pragma unroll
-      for (int r = 0; r < 8; ++r)
+    for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
-        for (int q = 0; q <= r; ++q) v[r][q] = pan[(c0 + r) * kPanelPitch + q];
+      for (int cb = 0; cb < NB; ++cb) {
+        if (cb > RB(mi)) continue;  // strictly upper blocks: never needed
+        const double2 v =
+            __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t));
+        x[SL(mi, cb)][0] = v.x;
+        x[SL(mi, cb)][1] = v.y;
+      }
+    if (c.warp == 0) {  // hand over the first diagonal block (rb0 = 0, slot 0)
+      *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(x[0][0], x[0][1]);
+      bar_arrive(kBarDiag, 64);
+    }
+  }
+#pragma unroll
+  for (int p = 0; p < NB; ++p) {
+    constexpr int kHalf = NB / 2;
+    const int pm = p < kHalf ? 0 : 1;              // which of its blocks holds row block p
+    const int pw = p < kHalf ? p : NB - 1 - p;     // the warp owning row block p
+    double* pan = c.pans() + (p & 1) * BS * kPanelPitch;
+    bar_sync(kBarCompute, kComputeThreads);  // L_pp and 1/L[j][j] published
+    if (active) {
+      if (c.warp == pw) {
+        const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
+        x[SL(pm, p)][0] = l.x;
+        x[SL(pm, p)][1] = l.y;
+      }
+      // (2) rows below the diagonal block: L[r, panel] = A[r, panel] L_pp^{-T}
 #pragma unroll
       for (int j = 0; j < 8; ++j) {
-        const double d = v[j][j];
-        if (!(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
-        // one rsqrt on the column's dependency chain: L[j][j] = d * d^{-1/2}, scale = d^{-1/2}
-        // (exact for the perfect squares of the integer family; within an ulp otherwise)
-        const double rl = rsqrt(d);
-        v[j][j] = d * rl;
-        rdiag[j] = rl;
+        const double rd = rdv[j];
+        const double l0 = dd[(2 * t) * 8 + j], l1 = dd[(2 * t + 1) * 8 + j];
 #pragma unroll
-        for (int r = j + 1; r < 8; ++r) v[r][j] *= rl;
-#pragma unroll
-        for (int r = j + 1; r < 8; ++r)
-#pragma unroll
-          for (int q = j + 1; q <= r; ++q) v[r][q] = fma(-v[r][j], v[q][j], v[r][q]);
+        for (int mi = 0; mi < 2; ++mi) {
+          if (RB(mi) <= p) continue;  // warp-uniform
+          double* xs = x[SL(mi, p)];
+          const double xj = __shfl_sync(0xffffffffu, xs[j & 1], qbase | (j >> 1)) * rd;
+          if (t == (j >> 1)) xs[j & 1] = xj;
+          if (2 * t > j) xs[0] = fma(-xj, l0, xs[0]);
+          if (2 * t + 1 > j) xs[1] = fma(-xj, l1, xs[1]);
+        }
       }
 #pragma unroll
-      for (int r = 0; r < 8; ++r)
-#pragma unroll
-        for (int q = 0; q <= r; ++q) pan[(c0 + r) * kPanelPitch + q] = v[r][q];
+      for (int mi = 0; mi < 2; ++mi)
+        if (RB(mi) > p)
+          *reinterpret_cast<double2*>(pan + (8 * RB(mi) + g) * kPanelPitch + 2 * t) =
+              make_double2(x[SL(mi, p)][0], x[SL(mi, p)][1]);
     }
-    bar_sync(kBarCompute, kComputeThreads);
-    const int r = c0 + 8 + tid;
-    if (r < BS) {  // rows below the diagonal block: L[r, panel] = A[r, panel] L_dd^{-T}
-      double v[8];
-      double* pr = pan + r * kPanelPitch;
-#pragma unroll
-      for (int j = 0; j < 8; j += 2) {
-        const double2 q = *reinterpret_cast<const double2*>(pr + j);
-        v[j] = q.x;
-        v[j + 1] = q.y;
+    bar_sync(kBarCompute, kComputeThreads);  // panel p published; dd / rdv free
+    if (active && p + 1 < NB) {
+      // (3) rank-8 update of this warp's lower blocks (rb >= cb > p); block (p+1, p+1)
+      // first, handed to the factor warp before the rest
+      const int nm = (p + 1) < kHalf ? 0 : 1;
+      const int nw = (p + 1) < kHalf ? p + 1 : NB - 2 - p;
+      if (c.warp == nw) {
+        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * (p + 1) + g) * kPanelPitch + 2 * t);
+        double* xd = x[SL(nm, p + 1)];
+        dmma884(xd[0], xd[1], -x[SL(nm, p)][0], bv.x);
+        dmma884(xd[0], xd[1], -x[SL(nm, p)][1], bv.y);
+        *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
+        bar_arrive(kBarDiag, 64);
       }
 #pragma unroll
-      for (int j = 0; j < 8; ++j) {
-        v[j] *= rdiag[j];
+      for (int cb = 1; cb < NB; ++cb) {  // constant trip count: fully unrolled, x stays in registers
+        if (cb <= p || cb > rb1) continue;  // warp-uniform (rb1 >= rb0)
+        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * cb + g) * kPanelPitch + 2 * t);
 #pragma unroll
-        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], pan[(c0 + j2) * kPanelPitch + j], v[j2]);
-      }
-#pragma unroll
-      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(pr + j) = make_double2(v[j], v[j + 1]);
-    }
-    bar_sync(kBarCompute, kComputeThreads);
-    panel_to_frag(c, x, p, pan);
-    // rank-8 update of this warp's lower blocks (rb >= cb > p)
-    double a[C::MI][2];
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) {
-      const double* pr = pan + (wm * C::WM + mi * 8 + g) * kPanelPitch;
-      a[mi][0] = -pr[t];
-      a[mi][1] = -pr[t + 4];
-    }
-#pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) {
-      const int cb = wn * C::NI + ni;
-      if (cb <= p) continue;
-      const double* lr = pan + (cb * 8 + g) * kPanelPitch;
-      const double b0 = lr[t], b1 = lr[t + 4];
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) {
-        if (wm * C::MI + mi < cb) continue;
-        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][0], b0);
-        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][1], b1);
+        for (int mi = 0; mi < 2; ++mi) {
+          if (RB(mi) < cb) continue;
+          if (cb == p + 1 && mi == nm && c.warp == nw) continue;  // done above
+          dmma884(x[SL(mi, cb)][0], x[SL(mi, cb)][1], -x[SL(mi, p)][0], bv.x);
+          dmma884(x[SL(mi, cb)][0], x[SL(mi, cb)][1], -x[SL(mi, p)][1], bv.y);
+        }
       }
     }
   }
-  frag_store(c, x, A, lda, true);
+  if (active) {
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb) {
+        if (cb > RB(mi)) continue;
+        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t),
+               make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]));
+      }
+  }
+#undef RB
+#undef SL
   bar_sync(kBarCompute, kComputeThreads);
 }
 
@@ -593,7 +662,8 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
   for (int cb = 0; cb < nbb; ++cb) {
     Acc<BS> acc;
     if (cb > 0) gemm_mainloop(c, c.slot(i, k), slab * BS, c.slot(k, k), cb * BS, 0, cb * BS, acc);
-    solve_block(c, acc, cb > 0, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+    if (cb > 0) acc_sub_global(c, acc, X + cb * BS, c.nb);
+    solve_block(c, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
     // X[:, cb] (generic stores) is read by TMA in the next block: complete the stores
     // at L2 (gpu-scope fence), then order them before async-proxy accesses.
     __threadfence();
@@ -605,16 +675,24 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
 // POTRF_k, inner step b (nested tiled Cholesky of the diagonal tile with block BS):
 //   potf2 of block (b, b)
 template <int BS>
+__device__ __forceinline__ void potf2_job(double* A, int lda, int col0, int* info) {
+  // out of line with plain arguments: the in-block factorization gets its own register
+  // allocation (it needs ~164 registers) instead of sharing one with the GEMM paths
+  Ctx<BS> c{};
+  c.warp = threadIdx.x >> 5;
+  c.lane = threadIdx.x & 31;
+  potf2_block(c, A, lda, col0, info);
+}
+template <int BS>
 __device__ __forceinline__ void sub_potrf_diag(Ctx<BS>& c, int k, int b, int* info) {
   double* A = c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS;
-  potf2_block(c, A, c.nb, k * c.nb + b * BS, info);
+  potf2_job<BS>(A, c.nb, k * c.nb + b * BS, info);
 }
 //   block (r, b), r > b:  X <- X L_bb^{-T}
 template <int BS>
 __device__ __forceinline__ void sub_potrf_panel(Ctx<BS>& c, int k, int b, int r) {
   double* T = c.tile(k, k);
-  Acc<BS> acc;
-  solve_block(c, acc, false, T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
+  solve_block(c, T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
 }
 //   block (r, q), b < q <= r:  A[r, q] -= L[r, b] L[q, b]^T   (K = BS)
 template <int BS>

@@ -11,7 +11,7 @@ __global__ void __launch_bounds__(kThreads, 1) k_bench(double* X, double* L, dou
   auto c = make_ctx<BS>(nullptr, nullptr, ld, 1);
   Acc<BS> acc;
   long long t0 = clock64();
-  for (int r = 0; r < reps; ++r) solve_block(c, acc, false, X, ld, L, ld);
+  for (int r = 0; r < reps; ++r) solve_block(c, X, ld, L, ld);
   long long t1 = clock64();
   for (int r = 0; r < reps; ++r) potf2_block(c, A, ld, 0, info);
   __syncthreads();

@@ -6,33 +6,18 @@ __device__ long long g_ph[64];
 __device__ long long g_last;
 namespace chol {
 template <int BS>
-__device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, Acc<BS>& acc, bool has_acc, double* X, int ldx,
-                                            const double* Ld, int ldl) {
+__device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, double* X, int ldx, const double* Ld, int ldl) {
   using C = Cfg<BS>;
   constexpr int P = C::kPitch, NB = BS / 8;
   const int tid = threadIdx.x, g = c.lane >> 2, t = c.lane & 3;
-  double* lb = c.lbuf;  // L block; column BS holds 1/L[c][c]
+  double* lb = c.lbuf();  // L block; column BS holds 1/L[c][c]
   // every warp must be done with lbuf (previous job / previous column block)
   bar_sync(kBarCompute, kComputeThreads);
-  if (threadIdx.x == 0) { long long _t = clock64(); g_ph[0] += _t - g_last; g_last = _t; }
-  if (has_acc) {  // X -= acc in the GEMM's fragment layout, through global memory (L2)
-    const int wm = c.warp >> 2, wn = c.warp & 3;
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) {
-        double2* px = reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN + ni * 8 +
-                                                 2 * t);
-        double2 v = __ldcg(px);
-        v.x -= acc[mi][ni][0];
-        v.y -= acc[mi][ni][1];
-        __stcg(px, v);
-      }
-  }
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[0] += _t - g_last; g_last = _t; }
   load_block<BS>(lb, Ld, ldl);
   if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
   bar_sync(kBarCompute, kComputeThreads);
-  if (threadIdx.x == 0) { long long _t = clock64(); g_ph[1] += _t - g_last; g_last = _t; }
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[1] += _t - g_last; g_last = _t; }
   if (c.warp < BS / 16) {
     RowX<BS> x;
     const int r0 = 16 * c.warp;
@@ -64,7 +49,8 @@ __device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, Acc<BS>& acc, bo
       }
       // (b) later column blocks: x[:, cb] -= x[:, p] L[cb rows, p cols]^T
 #pragma unroll
-      for (int cb = p + 1; cb < NB; ++cb) {
+      for (int cb = 1; cb < NB; ++cb) {  // constant trip count: fully unrolled, x stays in registers
+        if (cb <= p) continue;
         const double2 bv = *reinterpret_cast<const double2*>(lb + (8 * cb + g) * P + c0 + 2 * t);
 #pragma unroll
         for (int mi = 0; mi < 2; ++mi) {
@@ -81,7 +67,7 @@ __device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, Acc<BS>& acc, bo
                make_double2(x.v[mi][cb][0], x.v[mi][cb][1]));
   }
   bar_sync(kBarCompute, kComputeThreads);  // lbuf free for the next user; X stores issued
-  if (threadIdx.x == 0) { long long _t = clock64(); g_ph[2] += _t - g_last; g_last = _t; }
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[2] += _t - g_last; g_last = _t; }
 }
 
 // Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
@@ -94,97 +80,127 @@ __device__ __forceinline__ void solve_block_T(const Ctx<BS>& c, Acc<BS>& acc, bo
 // stored; the upper halves of diagonal 8x8 blocks are scratch (never read).
 template <int BS>
 __device__ __forceinline__ void potf2_block_T(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
-  using C = Cfg<BS>;
-  const int tid = threadIdx.x, lane = c.lane, wm = c.warp >> 2, wn = c.warp & 3, g = lane >> 2, t = lane & 3;
-  double* pans = c.pans;
-  double* rdiag = c.lbuf;  // 1/L[c][c] of the current panel (8 doubles)
-  Acc<BS> x;
-  frag_load(c, x, A, lda);
-  bar_sync(kBarCompute, kComputeThreads);  // buf / lbuf reuse
-  if (threadIdx.x == 0) { long long _t = clock64(); g_ph[0] += _t - g_last; g_last = _t; }
+  constexpr int NB = BS / 8;
+  static_assert(NB % 2 == 0 && NB / 2 <= 7, "paired row blocks; warp 7 factors the diagonal blocks");
+  const int g = c.lane >> 2, t = c.lane & 3, qbase = c.lane & ~3;
+  double* dd = c.lbuf();        // 8 x 8 diagonal block (pitch 8) + 8 reciprocals
+  double* rdv = c.lbuf() + 64;
+  bar_sync(kBarCompute, kComputeThreads);  // lbuf / pans reuse
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[0] += _t - g_last; g_last = _t; }
+  if (c.warp == 7) {
+    // factor warp: its own loop, disjoint from the row-block code (register pressure)
 #pragma unroll 1
-  for (int p = 0; p < BS / 8; ++p) {
-    const int c0 = 8 * p;
-    double* pan = pans + (p & 1) * BS * kPanelPitch;
-    frag_to_panel(c, x, p, pan);
-    bar_sync(kBarCompute, kComputeThreads);
+    for (int p = 0; p < NB; ++p) {
+      bar_sync(kBarDiag, 64);  // diagonal block p is in dd
+      if (c.lane == 0) factor_8x8(dd, rdv, info, col0 + 8 * p);
+      bar_sync(kBarCompute, kComputeThreads);  // L_pp published
     if (threadIdx.x == 0) { long long _t = clock64(); g_ph[1] += _t - g_last; g_last = _t; }
-    if (tid == 0) {  // 8x8 diagonal block: one thread, all 36 entries in registers
-      double v[8][8];
-#pragma unroll
-      for (int r = 0; r < 8; ++r)
-#pragma unroll
-        for (int q = 0; q <= r; ++q) v[r][q] = pan[(c0 + r) * kPanelPitch + q];
-#pragma unroll
-      for (int j = 0; j < 8; ++j) {
-        const double d = v[j][j];
-        if (!(d > 0.0)) atomicMin(info, col0 + c0 + j + 1);
-        // one rsqrt on the column's dependency chain: L[j][j] = d * d^{-1/2}, scale = d^{-1/2}
-        // (exact for the perfect squares of the integer family; within an ulp otherwise)
-        const double rl = rsqrt(d);
-        v[j][j] = d * rl;
-        rdiag[j] = rl;
-#pragma unroll
-        for (int r = j + 1; r < 8; ++r) v[r][j] *= rl;
-#pragma unroll
-        for (int r = j + 1; r < 8; ++r)
-#pragma unroll
-          for (int q = j + 1; q <= r; ++q) v[r][q] = fma(-v[r][j], v[q][j], v[r][q]);
-      }
-#pragma unroll
-      for (int r = 0; r < 8; ++r)
-#pragma unroll
-        for (int q = 0; q <= r; ++q) pan[(c0 + r) * kPanelPitch + q] = v[r][q];
-    }
-    bar_sync(kBarCompute, kComputeThreads);
+      bar_sync(kBarCompute, kComputeThreads);  // panel p published
     if (threadIdx.x == 0) { long long _t = clock64(); g_ph[2] += _t - g_last; g_last = _t; }
-    const int r = c0 + 8 + tid;
-    if (r < BS) {  // rows below the diagonal block: L[r, panel] = A[r, panel] L_dd^{-T}
-      double v[8];
-      double* pr = pan + r * kPanelPitch;
-#pragma unroll
-      for (int j = 0; j < 8; j += 2) {
-        const double2 q = *reinterpret_cast<const double2*>(pr + j);
-        v[j] = q.x;
-        v[j + 1] = q.y;
-      }
-#pragma unroll
-      for (int j = 0; j < 8; ++j) {
-        v[j] *= rdiag[j];
-#pragma unroll
-        for (int j2 = j + 1; j2 < 8; ++j2) v[j2] = fma(-v[j], pan[(c0 + j2) * kPanelPitch + j], v[j2]);
-      }
-#pragma unroll
-      for (int j = 0; j < 8; j += 2) *reinterpret_cast<double2*>(pr + j) = make_double2(v[j], v[j + 1]);
     }
     bar_sync(kBarCompute, kComputeThreads);
     if (threadIdx.x == 0) { long long _t = clock64(); g_ph[3] += _t - g_last; g_last = _t; }
-    panel_to_frag(c, x, p, pan);
-    // rank-8 update of this warp's lower blocks (rb >= cb > p)
-    double a[C::MI][2];
+    return;
+  }
+  const bool active = c.warp < NB / 2;
+  const int rb0 = c.warp, rb1 = NB - 1 - c.warp;  // the warp's two row blocks
+  double x[NB + 1][2];
+#define RB(mi) ((mi) == 0 ? rb0 : rb1)
+#define SL(mi, cb) ((mi) == 0 ? (cb) : NB - (cb))
+  if (active) {
 #pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) {
-      const double* pr = pan + (wm * C::WM + mi * 8 + g) * kPanelPitch;
-      a[mi][0] = -pr[t];
-      a[mi][1] = -pr[t + 4];
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb) {
+        if (cb > RB(mi)) continue;  // strictly upper blocks: never needed
+        const double2 v =
+            __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t));
+        x[SL(mi, cb)][0] = v.x;
+        x[SL(mi, cb)][1] = v.y;
+      }
+    if (c.warp == 0) {  // hand over the first diagonal block (rb0 = 0, slot 0)
+      *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(x[0][0], x[0][1]);
+      bar_arrive(kBarDiag, 64);
     }
+  }
 #pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) {
-      const int cb = wn * C::NI + ni;
-      if (cb <= p) continue;
-      const double* lr = pan + (cb * 8 + g) * kPanelPitch;
-      const double b0 = lr[t], b1 = lr[t + 4];
+  for (int p = 0; p < NB; ++p) {
+    constexpr int kHalf = NB / 2;
+    const int pm = p < kHalf ? 0 : 1;              // which of its blocks holds row block p
+    const int pw = p < kHalf ? p : NB - 1 - p;     // the warp owning row block p
+    double* pan = c.pans() + (p & 1) * BS * kPanelPitch;
+    bar_sync(kBarCompute, kComputeThreads);  // L_pp and 1/L[j][j] published
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[4] += _t - g_last; g_last = _t; }
+    if (active) {
+      if (c.warp == pw) {
+        const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
+        x[SL(pm, p)][0] = l.x;
+        x[SL(pm, p)][1] = l.y;
+      }
+      // (2) rows below the diagonal block: L[r, panel] = A[r, panel] L_pp^{-T}
 #pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) {
-        if (wm * C::MI + mi < cb) continue;
-        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][0], b0);
-        dmma884(x[mi][ni][0], x[mi][ni][1], a[mi][1], b1);
+      for (int j = 0; j < 8; ++j) {
+        const double rd = rdv[j];
+        const double l0 = dd[(2 * t) * 8 + j], l1 = dd[(2 * t + 1) * 8 + j];
+#pragma unroll
+        for (int mi = 0; mi < 2; ++mi) {
+          if (RB(mi) <= p) continue;  // warp-uniform
+          double* xs = x[SL(mi, p)];
+          const double xj = __shfl_sync(0xffffffffu, xs[j & 1], qbase | (j >> 1)) * rd;
+          if (t == (j >> 1)) xs[j & 1] = xj;
+          if (2 * t > j) xs[0] = fma(-xj, l0, xs[0]);
+          if (2 * t + 1 > j) xs[1] = fma(-xj, l1, xs[1]);
+        }
+      }
+#pragma unroll
+      for (int mi = 0; mi < 2; ++mi)
+        if (RB(mi) > p)
+          *reinterpret_cast<double2*>(pan + (8 * RB(mi) + g) * kPanelPitch + 2 * t) =
+              make_double2(x[SL(mi, p)][0], x[SL(mi, p)][1]);
+    }
+    bar_sync(kBarCompute, kComputeThreads);  // panel p published; dd / rdv free
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[5] += _t - g_last; g_last = _t; }
+    if (active && p + 1 < NB) {
+      // (3) rank-8 update of this warp's lower blocks (rb >= cb > p); block (p+1, p+1)
+      // first, handed to the factor warp before the rest
+      const int nm = (p + 1) < kHalf ? 0 : 1;
+      const int nw = (p + 1) < kHalf ? p + 1 : NB - 2 - p;
+      if (c.warp == nw) {
+        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * (p + 1) + g) * kPanelPitch + 2 * t);
+        double* xd = x[SL(nm, p + 1)];
+        dmma884(xd[0], xd[1], -x[SL(nm, p)][0], bv.x);
+        dmma884(xd[0], xd[1], -x[SL(nm, p)][1], bv.y);
+        *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
+        bar_arrive(kBarDiag, 64);
+      }
+#pragma unroll
+      for (int cb = 1; cb < NB; ++cb) {  // constant trip count: fully unrolled, x stays in registers
+        if (cb <= p || cb > rb1) continue;  // warp-uniform (rb1 >= rb0)
+        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * cb + g) * kPanelPitch + 2 * t);
+#pragma unroll
+        for (int mi = 0; mi < 2; ++mi) {
+          if (RB(mi) < cb) continue;
+          if (cb == p + 1 && mi == nm && c.warp == nw) continue;  // done above
+          dmma884(x[SL(mi, cb)][0], x[SL(mi, cb)][1], -x[SL(mi, p)][0], bv.x);
+          dmma884(x[SL(mi, cb)][0], x[SL(mi, cb)][1], -x[SL(mi, p)][1], bv.y);
+        }
       }
     }
   }
-  frag_store(c, x, A, lda, true);
+  if (active) {
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb) {
+        if (cb > RB(mi)) continue;
+        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t),
+               make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]));
+      }
+  }
+#undef RB
+#undef SL
   bar_sync(kBarCompute, kComputeThreads);
-  if (threadIdx.x == 0) { long long _t = clock64(); g_ph[4] += _t - g_last; g_last = _t; }
+    if (threadIdx.x == 0) { long long _t = clock64(); g_ph[6] += _t - g_last; g_last = _t; }
 }
 
 
