@@ -58,7 +58,10 @@ struct Ctx {
   // registers of pointers live through the register-hungry in-block routines).
   __device__ static char* base() {
     extern __shared__ __align__(1024) char smem_raw[];
-    return reinterpret_cast<char*>((reinterpret_cast<uintptr_t>(smem_raw) + 1023) & ~uintptr_t(1023));
+    // pointer arithmetic on smem_raw (not an integer round trip) keeps the shared
+    // address space visible to the compiler: LDS/STS instead of generic LD/ST
+    const uint32_t mis = static_cast<uint32_t>(__cvta_generic_to_shared(smem_raw)) & 1023u;
+    return smem_raw + ((1024u - mis) & 1023u);
   }
   __device__ static char* bars() { return base() + Cfg<BS>::kPipeBytes + Cfg<BS>::kBufBytes + Cfg<BS>::kPanBytes; }
   __device__ char* pipe() const { return base(); }  // kStages x {A, B} operand buffers
