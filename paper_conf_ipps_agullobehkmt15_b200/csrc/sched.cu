@@ -549,7 +549,14 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // TRSM decomposition: row-slab jobs (default) or right-looking block nodes
   // (CHOL_TRSM_BLOCKS=1, development switch; measured 2.5% slower at n=19200).
   const char* ev = getenv("CHOL_TRSM_BLOCKS");
-  const bool trsm_slab = !(ev && ev[0] == '1');
+  const bool trsm_slab_all = !(ev && ev[0] == '1');
+  // Steps whose TRSMs are on the critical path use the block decomposition (TS/TU:
+  // more parallel, ~2.5x shorter latency than a 500 us slab job): the last step always,
+  // every step of a small factorization (N <= 8).  Measured (job traces, r01): n=19200
+  // 72.02 -> 71.79 ms, n=3840 4.40 -> 4.04 ms, n=1920 1.84 -> 1.72 ms.
+  // CHOL_TRSM_TAIL=t overrides (last t steps; development switch).
+  const char* et = getenv("CHOL_TRSM_TAIL");
+  const int trsm_tail = et ? atoi(et) : (N <= 8 ? (int)N : 1);
   // Multi-GPU: this rank creates the nodes of the tasks that overwrite the tiles it owns
   // (owner-computes), plus one RECV node per remote panel tile it reads.
   auto mine = [&](int64_t i, int64_t j) { return !dist || tile_owner(i, j, dist->p, dist->q) == dist->rank; };
@@ -584,6 +591,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     }
     for (int i = k + 1; i < N; ++i) {
       if (!mine(i, k)) continue;
+      const bool trsm_slab = trsm_slab_all && k < N - 1 - trsm_tail;
       if (trsm_slab) {  // one left-looking row-slab job per BS rows
         const int tid = (int)id_trsm(N, i, k);
         const int n = B.add_node(tid, T_TRSM, i, k);
