@@ -653,25 +653,27 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     build_task_dag(N, E, type_of);
     for (auto& e : E) B.edge(last_node[e.first], first_node[e.second]);
     // Streamed input (chol_factor from host memory): the first task touching a tile
-    // waits for the tile's arrival flag (the copy engine writes it after the tile);
-    // watch order = first-use order = the order the tiles are copied in.
-    std::vector<char> seen((size_t)(N * (N + 1) / 2), 0);
+    // waits for the tile's arrival flag (the copy engine writes it after the tile).
+    // Tiles arrive in row-major tile order (row i: tiles (i,0..i)); the watch list
+    // follows the same order.  Row-major arrival lets each arriving row feed the
+    // trailing updates of every factored column at once (list-scheduling model of
+    // the job DAG, 148 workers, 53.6 GB/s: 72.2 ms vs 73.8 ms for column order and
+    // 70.6 ms for instant arrival at n=19200).
     int order = 0;
     auto first_touch = [&](int64_t task, int64_t i, int64_t j) {
       const int64_t t = tile_index(i, j);
-      if (seen[t]) return;
-      seen[t] = 1;
       B.deps[first_node[task]] += 1;
       watch.push_back(make_int4(first_node[task], 0, (int)t, order++));
     };
-    for (int64_t k = 0; k < N; ++k) {
-      first_touch(id_potrf(N, k), k, k);
-      for (int64_t i = k + 1; i < N; ++i) first_touch(id_trsm(N, i, k), i, k);
-      for (int64_t j = k + 1; j < N; ++j) {
-        first_touch(id_syrk(N, j, k), j, j);
-        for (int64_t i = j + 1; i < N; ++i) first_touch(id_gemm(N, i, j, k), i, j);
+    for (int64_t i = 0; i < N; ++i)
+      for (int64_t j = 0; j <= i; ++j) {
+        if (j == 0)
+          first_touch(i == 0 ? id_potrf(N, 0) : id_trsm(N, i, 0), i, 0);  // POTRF_0 / TRSM_i_0
+        else if (i == j)
+          first_touch(id_syrk(N, j, 0), j, j);  // SYRK_j_0
+        else
+          first_touch(id_gemm(N, i, j, 0), i, j);  // GEMM_i_j_0
       }
-    }
     // Streamed output: every final panel tile is published (host-mapped flags)
     publish.assign(B.deps.size(), -1);
     for (int64_t k = 0; k < N; ++k) {

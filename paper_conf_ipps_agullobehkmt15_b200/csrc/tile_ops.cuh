@@ -521,8 +521,7 @@ __device__ __forceinline__ void factor_8x8(double* dd, double* rdv, int* info, i
 //   (3) after a second barrier every warp applies the rank-8 update to its lower
 //       blocks with FP64 DMMA (A operand = its own solved fragments).
 // A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
-// reading R6).  Only the lower blocks are stored; the upper halves of the diagonal 8x8
-// blocks are never read (stored back as the input values).
+// reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
 template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   constexpr int NB = BS / 8;
@@ -627,13 +626,21 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
     }
   }
   if (active) {
+    // the whole block is written: L on and below the diagonal, zeros above it (the
+    // strictly upper triangle of the factor is zero; written here so a diagonal tile
+    // can be copied out as soon as its POTRF completes)
 #pragma unroll
     for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
       for (int cb = 0; cb < NB; ++cb) {
-        if (cb > RB(mi)) continue;
-        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t),
-               make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]));
+        double2 v = make_double2(0.0, 0.0);
+        if (cb < RB(mi)) {
+          v = make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]);
+        } else if (cb == RB(mi)) {
+          v.x = 2 * t <= g ? x[SL(mi, cb)][0] : 0.0;
+          v.y = 2 * t + 1 <= g ? x[SL(mi, cb)][1] : 0.0;
+        }
+        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t), v);
       }
   }
 #undef RB
@@ -696,6 +703,13 @@ template <int BS>
 __device__ __forceinline__ void sub_potrf_panel(Ctx<BS>& c, int k, int b, int r) {
   double* T = c.tile(k, k);
   solve_block(c, T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
+  // the mirror block (b, r) lies in the strictly upper triangle of L_kk: final as zero
+  // (no task reads it; zeroing it here lets the tile be copied out as soon as it is final)
+  double* U = T + (int64_t)b * BS * c.nb + r * BS;
+  for (int e = threadIdx.x; e < BS * BS / 2; e += kComputeThreads) {
+    const int row = e / (BS / 2), col = 2 * (e % (BS / 2));
+    __stcg(reinterpret_cast<double2*>(U + (int64_t)row * c.nb + col), make_double2(0.0, 0.0));
+  }
 }
 //   block (r, q), b < q <= r:  A[r, q] -= L[r, b] L[q, b]^T   (K = BS)
 template <int BS>
