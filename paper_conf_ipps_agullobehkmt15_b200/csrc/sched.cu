@@ -98,15 +98,96 @@ __device__ __forceinline__ void push_node(const DevSched& d, int node) {
   atomicExch(&d.q_items[d.q_base[q] + slot], node + 1);
 }
 
+// A node is done (its last job completed, or it has no jobs): publish the tile it makes
+// final (multi-GPU / streamed output), release its successors, count it.  Called by a
+// whole warp: lane l releases successors l, l+32, ... concurrently (a POTRF diagonal
+// block or a TRSM exit node has up to ~2N successors; one push costs two dependent L2
+// round trips).  A successor without jobs (the entry / exit node of a block-decomposed
+// TRSM) is done as soon as it is ready, by the whole warp; Depth bounds that recursion
+// (the builder never chains two job-less nodes).
+// Direct handoff: if the calling worker will be idle (can_take), the first ready
+// single-job successor is not queued but returned, and the worker runs it next -- no
+// queue round trips on chains of single-job nodes (the POTRF block DAG's critical path
+// D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1)).  Returns that node or -1 (warp-uniform).
+template <int Depth>
+__device__ int node_done_warp(const DevSched& d, int node, int lane, bool can_take) {
+  __threadfence();
+  if (lane == 0 && d.node_publish) {
+    const int pt = d.node_publish[node];
+    if (pt >= 0) {  // panel tile final: release it to every rank (system scope, NVLink)
+      __threadfence_system();
+      asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(d.my_flags + pt), "r"(d.epoch) : "memory");
+    }
+  }
+  int take = -1;
+  const int beg = d.succ_off[node], end = d.succ_off[node + 1];
+  for (int e0 = beg; e0 < end; e0 += 32) {
+    const int e = e0 + lane;
+    int s = -1, cnt = -1;
+    if (e < end) {
+      s = d.succ[e];
+      if (atomicSub(&d.node_deps[s], 1) == 1) cnt = d.node_job_count[s];
+    }
+    const bool join = Depth > 0 && cnt == 0;
+    const unsigned ms = __ballot_sync(0xffffffffu, can_take && take < 0 && cnt == 1);
+    const int taker = ms ? __ffs(ms) - 1 : -1;
+    if (taker >= 0) {
+      take = __shfl_sync(0xffffffffu, s, taker);
+      if (lane == taker && d.job_trace) d.job_trace[4 * (size_t)d.node_job_begin[s] + 3] = globaltimer_ns() - *d.tr_base;
+    }
+    if (cnt > 0 && lane != taker) push_node(d, s);
+    if constexpr (Depth > 0) {
+      unsigned m = __ballot_sync(0xffffffffu, join);
+      while (m) {
+        const int src = __ffs(m) - 1;
+        m &= m - 1;
+        const int t = node_done_warp<Depth - 1>(d, __shfl_sync(0xffffffffu, s, src), lane, can_take && take < 0);
+        if (take < 0) take = t;
+      }
+    }
+  }
+  if (lane == 0 && atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
+    __threadfence();
+    atomicExch(d.finished, 1);
+  }
+  __syncwarp();
+  return take;
+}
+
+// A node whose dependencies are all satisfied, single thread (init, watcher lanes):
+// queue its jobs, or -- job-less -- release its successors at once.
+__device__ void ready_node(const DevSched& d, int node) {
+  if (d.node_job_count[node] > 0) {
+    push_node(d, node);
+    return;
+  }
+  __threadfence();
+  if (d.node_publish && d.node_publish[node] >= 0) {
+    __threadfence_system();
+    asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(d.my_flags + d.node_publish[node]), "r"(d.epoch) : "memory");
+  }
+  for (int e = d.succ_off[node]; e < d.succ_off[node + 1]; ++e)
+    if (atomicSub(&d.node_deps[d.succ[e]], 1) == 1) push_node(d, d.succ[e]);  // never job-less (builder)
+  if (atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
+    __threadfence();
+    atomicExch(d.finished, 1);
+  }
+}
+
 // One warp pops one job: lanes inspect 32 queues at a time, highest priority first
 // (two passes over the kBuckets buckets of the worker's class); the head node of the
 // best non-empty queue hands out its next job; an exhausted head node is retired by
 // advancing the queue head.  Returns -1 if nothing is ready.
-__device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, int lane) {
+__device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, int lane, uint32_t done_bar,
+                                       uint32_t done_parity) {
   const int cls = (d.policy == 2 && latency_worker) ? kBuckets : 0;  // pinned queues or normal ones
+  bool gave_up = false;
   for (int pass = 0; pass < kBuckets / 32; ++pass) {
     const int q = cls + (kBuckets - 1 - (pass * 32 + lane));
     for (int attempt = 0; attempt < 16; ++attempt) {
+      // the worker's running job finished: return to retire it (its successors may be
+      // on the critical path) instead of racing other workers for queue heads
+      if (done_bar && __any_sync(0xffffffffu, mbar_test_wait(done_bar, done_parity))) return -2;
       const int h = ld_volatile(&d.q_head[q * kQStride]);
       const int t = ld_volatile(&d.q_tail[q * kQStride]);
       const int item = h < t ? ld_volatile(&d.q_items[d.q_base[q] + h]) : 0;
@@ -117,8 +198,12 @@ __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, i
       if (lane == src) {
         const int node = item - 1;
         const int j = atomicAdd(&d.node_next[node], 1);
-        if (j < d.node_job_count[node]) {
+        const int cnt = d.node_job_count[node];
+        if (j < cnt) {
           job = d.node_job_begin[node] + j;
+          // the claimer of a node's last job retires it from the head at once: lazy
+          // retirement by later scanners walks claimed single-job nodes one CAS at a time
+          if (j == cnt - 1) atomicCAS(&d.q_head[q * kQStride], h, h + 1);
         } else {
           atomicCAS(&d.q_head[q * kQStride], h, h + 1);  // node exhausted: retire it
           job = -2;
@@ -126,9 +211,10 @@ __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, i
       }
       job = __shfl_sync(0xffffffffu, job, src);
       if (job >= 0) return job;
+      if (attempt == 15) gave_up = true;
     }
   }
-  return -1;
+  return gave_up ? -2 : -1;
 }
 
 // ------------------------------------------------------------------ warp-specialised worker
@@ -214,7 +300,10 @@ __device__ void producer_loop(Ctx<BS>& c) {
       }
     }
     ++q;
-    *issued = (int)q;
+    // jobs without TMA stages (in-register solves, POTRF diagonal blocks, RECV copies)
+    // never mark themselves issued: their worker claims its next job only when they end,
+    // so a critical job is not captured by a worker busy for another 10-20 us
+    if (!skip && (type == J_UPD || type == J_PUPD || type == J_TU || type == J_TRSM)) *issued = (int)q;
   }
 }
 
@@ -264,7 +353,7 @@ __device__ void watcher_loop(const DevSched& d) {
       if (fire) {
         d.watch_fired[e] = 1;
         __threadfence();
-        if (atomicSub(&d.node_deps[w.x], 1) == 1) push_node(d, w.x);
+        if (atomicSub(&d.node_deps[w.x], 1) == 1) ready_node(d, w.x);
       }
       fired_any |= __any_sync(0xffffffffu, fire);
     }
@@ -311,7 +400,7 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     for (int cb = 0; cb < nbb; ++cb) {
       if (cb > 0) gemm_consume(c, cb * BS / BK, acc);
       if (cb > 0) acc_sub_global(c, acc, X + cb * BS, c.nb);
-      solve_block(c, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+      solve_block_job<BS>(X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
       if (cb + 1 < nbb) {
         // X[:, cb] is read by the producer's TMA for the next column block
         __threadfence();
@@ -327,8 +416,8 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     epi_sub_global(c, acc, c.tile(i, k) + (int64_t)sl * BS * c.nb + c2 * BS, c.nb, false);
   } else if (type == J_TS) {
     const int i = d0.z, k = d1.x, cb = d1.y, sl = d1.z;
-    solve_block(c, c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
-                c.tile(k, k) + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+    solve_block_job<BS>(c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
+                        c.tile(k, k) + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
   } else if (type == J_RECV) {  // copy BS rows of a remote panel tile into the local cache
     const int i = d0.z, j = d0.w, sl = d1.y, owner = d1.z;
     (void)owner;
@@ -368,12 +457,19 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
   }
 }
 
-// ---- scheduler warp
-__device__ __forceinline__ void complete_job(const DevSched& d, const StepParams& sp, int job, uint64_t t0_abs,
-                                             uint64_t t1_abs) {
-  __threadfence();  // the compute warps' stores (acquired through jdone) before the counters
+// ---- scheduler warp (all lanes): job counter, node completion, trace
+__device__ __forceinline__ int complete_job(const DevSched& d, const StepParams& sp, int job, uint64_t t0_abs,
+                                            uint64_t t1_abs, int lane, bool can_take) {
   const int node = d.job_node[job];
-  if (sp.tr_t0 && d.node_paper[node] >= 0) {
+  int last = 0;
+  if (lane == 0) {
+    __threadfence();  // the compute warps' stores (acquired through jdone) before the counters
+    last = atomicSub(&d.node_left[node], 1) == 1;
+  }
+  const int take = __shfl_sync(0xffffffffu, last, 0) ? node_done_warp<1>(d, node, lane, can_take) : -1;
+  // trace records after the release: every job of a task updates the same two words,
+  // and that contention must not delay the successors
+  if (lane == 0 && sp.tr_t0 && d.node_paper[node] >= 0) {
     const uint64_t base = *sp.tr_base;
     const uint64_t t0 = t0_abs - base, t_end = t1_abs - base;
     const int pt = d.node_paper[node];
@@ -385,50 +481,34 @@ __device__ __forceinline__ void complete_job(const DevSched& d, const StepParams
       d.job_trace[4 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
     }
   }
-  if (atomicSub(&d.node_left[node], 1) == 1) {
-    __threadfence();
-    if (d.node_publish) {
-      const int pt = d.node_publish[node];
-      if (pt >= 0) {  // panel tile final: release it to every rank (system scope, NVLink)
-        __threadfence_system();
-        asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(d.my_flags + pt), "r"(d.epoch) : "memory");
-      }
-    }
-    for (int e = d.succ_off[node]; e < d.succ_off[node + 1]; ++e) {
-      const int s = d.succ[e];
-      if (atomicSub(&d.node_deps[s], 1) == 1) push_node(d, s);
-    }
-    if (atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
-      __threadfence();
-      atomicExch(d.finished, 1);
-    }
-  }
+  return take;
 }
-
 template <int BS>
 __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& sp, bool latency_worker) {
   const int lane = c.lane;
   uint32_t q_issue = 0, q_done = 0;
   int pending[2] = {-1, -1};
+  int take = -1;  // single-job successor handed to this worker by its own completion
   unsigned backoff = 32;
   while (true) {
     // 1. retire finished jobs in order
     while (q_done < q_issue) {
       const int e = q_done & 1;
       if (!mbar_try_wait(smem_u32(&c.jdone()[e]), (q_done >> 1) & 1)) break;
-      if (lane == 0) {
-        const int4 tt = c.jdesc()[e * 3 + 2];
-        const uint64_t t0 = (uint64_t)(uint32_t)tt.x | ((uint64_t)(uint32_t)tt.y << 32);
-        const uint64_t t1 = (uint64_t)(uint32_t)tt.z | ((uint64_t)(uint32_t)tt.w << 32);
-        complete_job(d, sp, pending[e], t0, t1);
-      }
-      __syncwarp();
+      const int4 tt = c.jdesc()[e * 3 + 2];
+      const uint64_t t0 = (uint64_t)(uint32_t)tt.x | ((uint64_t)(uint32_t)tt.y << 32);
+      const uint64_t t1 = (uint64_t)(uint32_t)tt.z | ((uint64_t)(uint32_t)tt.w << 32);
+      const int t = complete_job(d, sp, pending[e], t0, t1, lane, take < 0 && q_done + 1 == q_issue);
+      if (t >= 0) take = t;
       ++q_done;
     }
     // 2. claim the next job once the ring has room and the producer is done with the
     //    running job's loads (late claim keeps critical-path hops short)
     if (q_issue - q_done < 2 && (q_issue == q_done || ld_volatile(prod_issued_ptr(c.jdesc())) >= (int)q_issue)) {
-      const int job = try_pop(d, latency_worker, lane);
+      const int job = take >= 0 ? d.node_job_begin[take]
+                                : try_pop(d, latency_worker, lane,
+                                          q_issue > q_done ? smem_u32(&c.jdone()[q_done & 1]) : 0u, (q_done >> 1) & 1);
+      take = -1;
       if (job >= 0) {
         const int e = q_issue & 1;
         if (lane == 0) {
@@ -455,7 +535,7 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
       break;
     }
     __nanosleep(backoff);
-    backoff = backoff < 512 ? backoff * 2 : 512;
+    backoff = backoff < 256 ? backoff * 2 : 256;
   }
 }
 
@@ -480,7 +560,7 @@ __global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__
 }
 
 __global__ void k_sched_init(DevSched d, const int* roots, int nroots) {
-  for (int r = 0; r < nroots; ++r) push_node(d, roots[r]);
+  for (int r = 0; r < nroots; ++r) ready_node(d, roots[r]);
 }
 
 // ------------------------------------------------------------------ host planner
@@ -557,6 +637,18 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // CHOL_TRSM_TAIL=t overrides (last t steps; development switch).
   const char* et = getenv("CHOL_TRSM_TAIL");
   const int trsm_tail = et ? atoi(et) : (N <= 8 ? (int)N : 1);
+  // ... and the TRSMs within trsm_dist tiles of the diagonal at every step (TRSM_{k+1,k}
+  // is on the chain POTRF_k -> TRSM_{k+1,k} -> SYRK_{k+1,k} -> POTRF_{k+1}).
+  // CHOL_TRSM_DIST=d overrides (development switch).
+  const char* etd = getenv("CHOL_TRSM_DIST");
+  const int trsm_dist = etd ? atoi(etd) : 0;
+  // TS/TU decomposition: per-column-step nodes (0, default) or per-row-slab chains of
+  // single-job nodes (1; measured slower under load).  CHOL_TRSM_SLABCHAIN.
+  const char* esc = getenv("CHOL_TRSM_SLABCHAIN");
+  const bool trsm_slabchain = esc && atoi(esc) != 0;
+  // POTRF inner structure: block-level DAG (1) or per-step nodes (0).  CHOL_POTRF_BLOCKDAG.
+  const char* epb = getenv("CHOL_POTRF_BLOCKDAG");
+  const bool potrf_blockdag = epb ? atoi(epb) != 0 : true;
   // Multi-GPU: this rank creates the nodes of the tasks that overwrite the tiles it owns
   // (owner-computes), plus one RECV node per remote panel tile it reads.
   auto mine = [&](int64_t i, int64_t j) { return !dist || tile_owner(i, j, dist->p, dist->q) == dist->rank; };
@@ -565,33 +657,63 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   std::vector<int> first_node(n_tasks(N), -1), last_node(n_tasks(N), -1);
   for (int k = 0; k < N; ++k) {
     const int pid = (int)id_potrf(N, k);
-    int prev = -1;
-    if (mine(k, k)) {
-    for (int b = 0; b < nbb; ++b) {
-      const int dn = B.add_node(pid, T_POTRF, k, k);
-      B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
-      if (prev >= 0) B.edge(prev, dn);
-      if (b == 0) first_node[pid] = dn;
-      prev = dn;
-      const int m = nbb - 1 - b;
-      if (m > 0) {
-        const int pn = B.add_node(pid, T_POTRF, k, k);
-        for (int r = b + 1; r < nbb; ++r)
-          B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
-        B.edge(prev, pn);
-        const int un = B.add_node(pid, T_POTRF, k, k);
-        for (int r = b + 1; r < nbb; ++r)
-          for (int q = b + 1; q <= r; ++q)
-            B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
-        B.edge(pn, un);
-        prev = un;
+    if (mine(k, k) && !potrf_blockdag) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
+      int prev = -1;
+      for (int b = 0; b < nbb; ++b) {
+        const int dn = B.add_node(pid, T_POTRF, k, k);
+        B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+        if (prev >= 0) B.edge(prev, dn);
+        if (b == 0) first_node[pid] = dn;
+        prev = dn;
+        if (b + 1 < nbb) {
+          const int pn = B.add_node(pid, T_POTRF, k, k);
+          for (int r = b + 1; r < nbb; ++r)
+            B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
+          B.edge(prev, pn);
+          const int un = B.add_node(pid, T_POTRF, k, k);
+          for (int r = b + 1; r < nbb; ++r)
+            for (int q = b + 1; q <= r; ++q)
+              B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
+          B.edge(pn, un);
+          prev = un;
+        }
       }
-    }
-    last_node[pid] = prev;
+      last_node[pid] = prev;
+    } else if (mine(k, k)) {
+      // POTRF_k as a block-level DAG over the BS x BS blocks of the diagonal tile
+      // (right-looking nested Cholesky): D(b) = potf2 of block (b,b); P(r,b) = solve of
+      // block (r,b) against L_bb; U(r,q,b) = K=BS update of block (r,q) by blocks (r,b),
+      // (q,b).  One job per node, so the chain D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1)
+      // never waits for a whole column or trailing update of the step.  D(nbb-1) is the
+      // sink (every inner node is its ancestor).
+      std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1);
+      for (int b = 0; b < nbb; ++b) {
+        const int dn = B.add_node(pid, T_POTRF, k, k);
+        B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+        if (lastU[b * nbb + b] >= 0) B.edge(lastU[b * nbb + b], dn);
+        if (b == 0) first_node[pid] = dn;
+        last_node[pid] = dn;
+        for (int r = b + 1; r < nbb; ++r) {
+          const int pn = B.add_node(pid, T_POTRF, k, k);
+          B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
+          B.edge(dn, pn);
+          if (lastU[r * nbb + b] >= 0) B.edge(lastU[r * nbb + b], pn);
+          pan[r] = pn;
+        }
+        for (int r = b + 1; r < nbb; ++r)
+          for (int q = b + 1; q <= r; ++q) {
+            const int un = B.add_node(pid, T_POTRF, k, k);
+            B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
+            B.edge(pan[r], un);
+            if (q != r) B.edge(pan[q], un);
+            if (lastU[r * nbb + q] >= 0) B.edge(lastU[r * nbb + q], un);  // same block, previous step
+            lastU[r * nbb + q] = un;
+          }
+      }
     }
     for (int i = k + 1; i < N; ++i) {
       if (!mine(i, k)) continue;
-      const bool trsm_slab = trsm_slab_all && k < N - 1 - trsm_tail;
+      const bool trsm_slab = trsm_slab_all && k < N - 1 - trsm_tail && i - k > trsm_dist;
       if (trsm_slab) {  // one left-looking row-slab job per BS rows
         const int tid = (int)id_trsm(N, i, k);
         const int n = B.add_node(tid, T_TRSM, i, k);
@@ -600,28 +722,58 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         first_node[tid] = last_node[tid] = n;
         continue;
       }
-      // TRSM_i_k, right-looking over the BS-column blocks c of A_ik (rows independent):
-      //   TS(c): A_ik[:, c] <- A_ik[:, c] L_kk[c,c]^{-T}        (nbb row-block jobs)
-      //   TU(c): A_ik[:, c'] -= A_ik[:, c] L_kk[c',c]^T, c' > c  (nbb x (nbb-1-c) jobs, K = BS)
-      const int tid = (int)id_trsm(N, i, k);
-      int prev_t = -1;
-      for (int cb = 0; cb < nbb; ++cb) {
-        const int ts = B.add_node(tid, T_TRSM, i, k);
-        for (int sl = 0; sl < nbb; ++sl)
-          B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
-        if (prev_t >= 0) B.edge(prev_t, ts);
-        if (cb == 0) first_node[tid] = ts;
-        prev_t = ts;
-        if (cb + 1 < nbb) {
-          const int tu = B.add_node(tid, T_TRSM, i, k);
+      if (!trsm_slabchain) {
+        // TRSM_i_k, right-looking over the BS-column blocks c of A_ik, one node per
+        // column step:  TS(c): A_ik[:, c] <- A_ik[:, c] L_kk[c,c]^{-T}  (nbb row-block jobs)
+        //               TU(c): A_ik[:, c'] -= A_ik[:, c] L_kk[c',c]^T, c' > c  (K = BS)
+        const int tid = (int)id_trsm(N, i, k);
+        int prev_t = -1;
+        for (int cb = 0; cb < nbb; ++cb) {
+          const int ts = B.add_node(tid, T_TRSM, i, k);
           for (int sl = 0; sl < nbb; ++sl)
-            for (int c2 = cb + 1; c2 < nbb; ++c2)
-              B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
-          B.edge(ts, tu);
-          prev_t = tu;
+            B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+          if (prev_t >= 0) B.edge(prev_t, ts);
+          if (cb == 0) first_node[tid] = ts;
+          prev_t = ts;
+          if (cb + 1 < nbb) {
+            const int tu = B.add_node(tid, T_TRSM, i, k);
+            for (int sl = 0; sl < nbb; ++sl)
+              for (int c2 = cb + 1; c2 < nbb; ++c2)
+                B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
+            B.edge(ts, tu);
+            prev_t = tu;
+          }
+        }
+        last_node[tid] = prev_t;
+        continue;
+      }
+      // Alternative (CHOL_TRSM_SLABCHAIN=1): rows are independent (X L^{-T}), so each
+      // BS-row slab sl is its own chain:
+      //   TS(c, sl): A_ik[sl, c] <- A_ik[sl, c] L_kk[c,c]^{-T}
+      //   TU(c, sl, c'): A_ik[sl, c'] -= A_ik[sl, c] L_kk[c',c]^T, c' > c   (K = BS)
+      // one job per node; a job-less entry node fans out to the nbb chains and a
+      // job-less exit node joins them (the task's single first / last node).
+      const int tid = (int)id_trsm(N, i, k);
+      const int entry = B.add_node(tid, T_TRSM, i, k), exit_ = B.add_node(tid, T_TRSM, i, k);
+      first_node[tid] = entry;
+      last_node[tid] = exit_;
+      std::vector<int> lastTU(nbb, -1);
+      for (int sl = 0; sl < nbb; ++sl) {
+        std::fill(lastTU.begin(), lastTU.end(), -1);
+        for (int cb = 0; cb < nbb; ++cb) {
+          const int ts = B.add_node(tid, T_TRSM, i, k);
+          B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+          B.edge(cb == 0 ? entry : lastTU[cb], ts);
+          if (cb + 1 == nbb) B.edge(ts, exit_);
+          for (int c2 = cb + 1; c2 < nbb; ++c2) {
+            const int tu = B.add_node(tid, T_TRSM, i, k);
+            B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
+            B.edge(ts, tu);
+            if (lastTU[c2] >= 0) B.edge(lastTU[c2], tu);
+            lastTU[c2] = tu;
+          }
         }
       }
-      last_node[tid] = prev_t;
     }
     for (int j = k + 1; j < N; ++j) {
       const int sid = (int)id_syrk(N, j, k);

@@ -13,6 +13,8 @@
 // the per-thread register budget at 255 -- a 9th warp caps it at 168.)  Sub-task granularity is a BS x BS block (BS = 96 at
 // nb = 960, so a GEMM task is 100 CTA sub-tasks of 96 x 96 x 960).
 #pragma once
+#include <utility>
+
 #include "dev_common.cuh"
 #include "taskid.h"
 
@@ -522,11 +524,115 @@ __device__ __forceinline__ void factor_8x8(double* dd, double* rdv, int* info, i
 //       blocks with FP64 DMMA (A operand = its own solved fragments).
 // A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
 // reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
+// Per-thread state of potf2_block: the warp's two row blocks rb0 = w, rb1 = NB-1-w; slot
+// SL(mi, cb) of x holds column block cb of row block mi (cb of the first block in slot
+// cb, of the second in slot NB-cb: disjoint since cb <= w < NB-cb).
+template <int BS>
+struct Potf2Regs {
+  static constexpr int NB = BS / 8;
+  double x[NB + 1][2];
+  int rb0, rb1, g, t, qbase;
+  bool active;
+  __device__ __forceinline__ int rb(int mi) const { return mi == 0 ? rb0 : rb1; }
+  __host__ __device__ static constexpr int sl(int mi, int cb) { return mi == 0 ? cb : NB - cb; }
+};
+
+// One 8-column panel P of potf2_block.  P is a template parameter so that every index
+// into x is a compile-time constant (a runtime panel index puts x in local memory:
+// 208-byte stack frame, 3x slower).
+template <int BS, int P>
+__device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, double* dd, double* rdv) {
+  using R = Potf2Regs<BS>;
+  constexpr int NB = R::NB, kHalf = NB / 2;
+  constexpr int pm = P < kHalf ? 0 : 1;           // which of its blocks holds row block P
+  constexpr int pw = P < kHalf ? P : NB - 1 - P;  // the warp owning row block P
+  double* pan = c.pans() + (P & 1) * BS * kPanelPitch;
+  const int g = s.g, t = s.t;
+  bar_sync(kBarCompute, kComputeThreads);  // L_pp and 1/L[j][j] published
+  if (s.active) {
+    if (c.warp == pw) {
+      const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
+      s.x[R::sl(pm, P)][0] = l.x;
+      s.x[R::sl(pm, P)][1] = l.y;
+    }
+    // (2) rows below the diagonal block: L[r, panel] = A[r, panel] L_pp^{-T}
+#pragma unroll
+    for (int j = 0; j < 8; ++j) {
+      const double rd = rdv[j];
+      const double l0 = dd[(2 * t) * 8 + j], l1 = dd[(2 * t + 1) * 8 + j];
+#pragma unroll
+      for (int mi = 0; mi < 2; ++mi) {
+        if (s.rb(mi) <= P) continue;  // warp-uniform
+        double* xs = s.x[R::sl(mi, P)];
+        const double xj = __shfl_sync(0xffffffffu, xs[j & 1], s.qbase | (j >> 1)) * rd;
+        if (t == (j >> 1)) xs[j & 1] = xj;
+        if (2 * t > j) xs[0] = fma(-xj, l0, xs[0]);
+        if (2 * t + 1 > j) xs[1] = fma(-xj, l1, xs[1]);
+      }
+    }
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi)
+      if (s.rb(mi) > P)
+        *reinterpret_cast<double2*>(pan + (8 * s.rb(mi) + g) * kPanelPitch + 2 * t) =
+            make_double2(s.x[R::sl(mi, P)][0], s.x[R::sl(mi, P)][1]);
+  }
+  bar_sync(kBarCompute, kComputeThreads);  // panel p published; dd / rdv free
+  if constexpr (P + 1 < NB) {
+    if (s.active) {
+      // (3) rank-8 update of this warp's lower blocks (rb >= cb > p); block (p+1, p+1)
+      // first, handed to the factor warp before the rest
+      constexpr int nm = (P + 1) < kHalf ? 0 : 1;
+      constexpr int nw = (P + 1) < kHalf ? P + 1 : NB - 2 - P;
+      if (c.warp == nw) {
+        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * (P + 1) + g) * kPanelPitch + 2 * t);
+        double* xd = s.x[R::sl(nm, P + 1)];
+        dmma884(xd[0], xd[1], -s.x[R::sl(nm, P)][0], bv.x);
+        dmma884(xd[0], xd[1], -s.x[R::sl(nm, P)][1], bv.y);
+        *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
+        bar_arrive(kBarDiag, 64);
+      }
+#pragma unroll
+      for (int cb = P + 1; cb < NB; ++cb) {
+        if (cb > s.rb1) continue;  // warp-uniform (rb1 >= rb0)
+        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * cb + g) * kPanelPitch + 2 * t);
+#pragma unroll
+        for (int mi = 0; mi < 2; ++mi) {
+          if (s.rb(mi) < cb) continue;
+          if (cb == P + 1 && mi == nm && c.warp == nw) continue;  // done above
+          dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][0], bv.x);
+          dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][1], bv.y);
+        }
+      }
+    }
+  }
+}
+
+template <int BS, int... P>
+__device__ __forceinline__ void potf2_panels(const Ctx<BS>& c, Potf2Regs<BS>& s, double* dd, double* rdv,
+                                             std::integer_sequence<int, P...>) {
+  (potf2_panel<BS, P>(c, s, dd, rdv), ...);
+}
+
+// Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
+// L196-199), blocked right-looking over 8-column panels p, register resident in a
+// row layout with paired row blocks: warp w < NB/2 owns the 8-row blocks rb = w and
+// rb = NB-1-w (13 of the 78 lower 8x8 blocks each for BS = 96: balanced work, and
+// NB+1 fragment slots per thread instead of 2*NB).  Per panel (potf2_panel):
+//   (1) the owner of the diagonal block updates it first and hands it to the idle
+//       warp 7 (named barrier kBarDiag), which factors it with one thread in
+//       registers (column algorithm of SURVEY §8c, one rsqrt per column) while the
+//       other warps finish their updates (one-panel lookahead);
+//   (2) after a compute barrier every warp solves its rows below against L_pp (quad
+//       shuffles) and publishes them to shared memory;
+//   (3) after a second barrier every warp applies the rank-8 update to its lower
+//       blocks with FP64 DMMA (A operand = its own solved fragments).
+// A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
+// reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
 template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   constexpr int NB = BS / 8;
   static_assert(NB % 2 == 0 && NB / 2 <= 7, "paired row blocks; warp 7 factors the diagonal blocks");
-  const int g = c.lane >> 2, t = c.lane & 3, qbase = c.lane & ~3;
+  using R = Potf2Regs<BS>;
   double* dd = c.lbuf();        // 8 x 8 diagonal block (pitch 8) + 8 reciprocals
   double* rdv = c.lbuf() + 64;
   bar_sync(kBarCompute, kComputeThreads);  // lbuf / pans reuse
@@ -542,90 +648,32 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
     bar_sync(kBarCompute, kComputeThreads);
     return;
   }
-  const bool active = c.warp < NB / 2;
-  const int rb0 = c.warp, rb1 = NB - 1 - c.warp;  // the warp's two row blocks
-  double x[NB + 1][2];
-#define RB(mi) ((mi) == 0 ? rb0 : rb1)
-#define SL(mi, cb) ((mi) == 0 ? (cb) : NB - (cb))
-  if (active) {
+  R s;
+  s.g = c.lane >> 2;
+  s.t = c.lane & 3;
+  s.qbase = c.lane & ~3;
+  s.active = c.warp < NB / 2;
+  s.rb0 = c.warp;
+  s.rb1 = NB - 1 - c.warp;
+  const int g = s.g, t = s.t;
+  if (s.active) {
 #pragma unroll
     for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
       for (int cb = 0; cb < NB; ++cb) {
-        if (cb > RB(mi)) continue;  // strictly upper blocks: never needed
+        if (cb > s.rb(mi)) continue;  // strictly upper blocks: never needed
         const double2 v =
-            __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t));
-        x[SL(mi, cb)][0] = v.x;
-        x[SL(mi, cb)][1] = v.y;
+            __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t));
+        s.x[R::sl(mi, cb)][0] = v.x;
+        s.x[R::sl(mi, cb)][1] = v.y;
       }
     if (c.warp == 0) {  // hand over the first diagonal block (rb0 = 0, slot 0)
-      *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(x[0][0], x[0][1]);
+      *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(s.x[0][0], s.x[0][1]);
       bar_arrive(kBarDiag, 64);
     }
   }
-#pragma unroll
-  for (int p = 0; p < NB; ++p) {
-    constexpr int kHalf = NB / 2;
-    const int pm = p < kHalf ? 0 : 1;              // which of its blocks holds row block p
-    const int pw = p < kHalf ? p : NB - 1 - p;     // the warp owning row block p
-    double* pan = c.pans() + (p & 1) * BS * kPanelPitch;
-    bar_sync(kBarCompute, kComputeThreads);  // L_pp and 1/L[j][j] published
-    if (active) {
-      if (c.warp == pw) {
-        const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
-        x[SL(pm, p)][0] = l.x;
-        x[SL(pm, p)][1] = l.y;
-      }
-      // (2) rows below the diagonal block: L[r, panel] = A[r, panel] L_pp^{-T}
-#pragma unroll
-      for (int j = 0; j < 8; ++j) {
-        const double rd = rdv[j];
-        const double l0 = dd[(2 * t) * 8 + j], l1 = dd[(2 * t + 1) * 8 + j];
-#pragma unroll
-        for (int mi = 0; mi < 2; ++mi) {
-          if (RB(mi) <= p) continue;  // warp-uniform
-          double* xs = x[SL(mi, p)];
-          const double xj = __shfl_sync(0xffffffffu, xs[j & 1], qbase | (j >> 1)) * rd;
-          if (t == (j >> 1)) xs[j & 1] = xj;
-          if (2 * t > j) xs[0] = fma(-xj, l0, xs[0]);
-          if (2 * t + 1 > j) xs[1] = fma(-xj, l1, xs[1]);
-        }
-      }
-#pragma unroll
-      for (int mi = 0; mi < 2; ++mi)
-        if (RB(mi) > p)
-          *reinterpret_cast<double2*>(pan + (8 * RB(mi) + g) * kPanelPitch + 2 * t) =
-              make_double2(x[SL(mi, p)][0], x[SL(mi, p)][1]);
-    }
-    bar_sync(kBarCompute, kComputeThreads);  // panel p published; dd / rdv free
-    if (active && p + 1 < NB) {
-      // (3) rank-8 update of this warp's lower blocks (rb >= cb > p); block (p+1, p+1)
-      // first, handed to the factor warp before the rest
-      const int nm = (p + 1) < kHalf ? 0 : 1;
-      const int nw = (p + 1) < kHalf ? p + 1 : NB - 2 - p;
-      if (c.warp == nw) {
-        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * (p + 1) + g) * kPanelPitch + 2 * t);
-        double* xd = x[SL(nm, p + 1)];
-        dmma884(xd[0], xd[1], -x[SL(nm, p)][0], bv.x);
-        dmma884(xd[0], xd[1], -x[SL(nm, p)][1], bv.y);
-        *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
-        bar_arrive(kBarDiag, 64);
-      }
-#pragma unroll
-      for (int cb = 1; cb < NB; ++cb) {  // constant trip count: fully unrolled, x stays in registers
-        if (cb <= p || cb > rb1) continue;  // warp-uniform (rb1 >= rb0)
-        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * cb + g) * kPanelPitch + 2 * t);
-#pragma unroll
-        for (int mi = 0; mi < 2; ++mi) {
-          if (RB(mi) < cb) continue;
-          if (cb == p + 1 && mi == nm && c.warp == nw) continue;  // done above
-          dmma884(x[SL(mi, cb)][0], x[SL(mi, cb)][1], -x[SL(mi, p)][0], bv.x);
-          dmma884(x[SL(mi, cb)][0], x[SL(mi, cb)][1], -x[SL(mi, p)][1], bv.y);
-        }
-      }
-    }
-  }
-  if (active) {
+  potf2_panels<BS>(c, s, dd, rdv, std::make_integer_sequence<int, NB>{});
+  if (s.active) {
     // the whole block is written: L on and below the diagonal, zeros above it (the
     // strictly upper triangle of the factor is zero; written here so a diagonal tile
     // can be copied out as soon as its POTRF completes)
@@ -634,17 +682,15 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
 #pragma unroll
       for (int cb = 0; cb < NB; ++cb) {
         double2 v = make_double2(0.0, 0.0);
-        if (cb < RB(mi)) {
-          v = make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]);
-        } else if (cb == RB(mi)) {
-          v.x = 2 * t <= g ? x[SL(mi, cb)][0] : 0.0;
-          v.y = 2 * t + 1 <= g ? x[SL(mi, cb)][1] : 0.0;
+        if (cb < s.rb(mi)) {
+          v = make_double2(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1]);
+        } else if (cb == s.rb(mi)) {
+          v.x = 2 * t <= g ? s.x[R::sl(mi, cb)][0] : 0.0;
+          v.y = 2 * t + 1 <= g ? s.x[R::sl(mi, cb)][1] : 0.0;
         }
-        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t), v);
+        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t), v);
       }
   }
-#undef RB
-#undef SL
   bar_sync(kBarCompute, kComputeThreads);
 }
 
@@ -693,6 +739,16 @@ __device__ __forceinline__ void potf2_job(double* A, int lda, int col0, int* inf
   c.lane = threadIdx.x & 31;
   potf2_block(c, A, lda, col0, info);
 }
+// solve_block out of line with plain arguments, for the persistent kernel (three call
+// sites: TRSM slab, TS, POTRF panel): one copy with its own register allocation, so its
+// ~100 live registers do not raise the pressure of the GEMM paths around the call sites.
+template <int BS>
+__device__ __noinline__ void solve_block_job(double* X, int ldx, const double* Ld, int ldl) {
+  Ctx<BS> c{};
+  c.warp = threadIdx.x >> 5;
+  c.lane = threadIdx.x & 31;
+  solve_block(c, X, ldx, Ld, ldl);
+}
 template <int BS>
 __device__ __forceinline__ void sub_potrf_diag(Ctx<BS>& c, int k, int b, int* info) {
   double* A = c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS;
@@ -702,7 +758,7 @@ __device__ __forceinline__ void sub_potrf_diag(Ctx<BS>& c, int k, int b, int* in
 template <int BS>
 __device__ __forceinline__ void sub_potrf_panel(Ctx<BS>& c, int k, int b, int r) {
   double* T = c.tile(k, k);
-  solve_block(c, T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
+  solve_block_job<BS>(T + (int64_t)r * BS * c.nb + b * BS, c.nb, T + (int64_t)b * BS * c.nb + b * BS, c.nb);
   // the mirror block (b, r) lies in the strictly upper triangle of L_kk: final as zero
   // (no task reads it; zeroing it here lets the tile be copied out as soon as it is final)
   double* U = T + (int64_t)b * BS * c.nb + r * BS;

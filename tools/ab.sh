@@ -7,7 +7,7 @@ for lib in variants/*.so; do
   for n in $NS; do
     CHOL_LIB_OVERRIDE=$lib python tools/job_trace.py $n 1 2>/dev/null | python -c "
 import json,sys; d=json.loads(sys.stdin.readline())
-print('$lib', $n, 'factor_ms %.3f util %.3f' % (d['factor_ms'], d['utilisation']), ' '.join('%s %.1f' % (k, d[k]['mean_us']) for k in ['UPD','TRSM','DIAG','PANEL','PUPD'] if k in d))"
+print('$lib', $n, 'factor_ms %.3f util %.3f' % (d['factor_ms'], d['utilisation']), ' '.join('%s %.1f' % (k, d[k]['mean_us']) for k in ['UPD','TRSM','DIAG','PANEL','PUPD','TS','TU'] if k in d))"
   done
 done
 done

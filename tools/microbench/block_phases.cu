@@ -188,13 +188,21 @@ __device__ __forceinline__ void potf2_block_T(const Ctx<BS>& c, double* A, int l
     }
   }
   if (active) {
+    // the whole block is written: L on and below the diagonal, zeros above it (the
+    // strictly upper triangle of the factor is zero; written here so a diagonal tile
+    // can be copied out as soon as its POTRF completes)
 #pragma unroll
     for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
       for (int cb = 0; cb < NB; ++cb) {
-        if (cb > RB(mi)) continue;
-        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t),
-               make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]));
+        double2 v = make_double2(0.0, 0.0);
+        if (cb < RB(mi)) {
+          v = make_double2(x[SL(mi, cb)][0], x[SL(mi, cb)][1]);
+        } else if (cb == RB(mi)) {
+          v.x = 2 * t <= g ? x[SL(mi, cb)][0] : 0.0;
+          v.y = 2 * t + 1 <= g ? x[SL(mi, cb)][1] : 0.0;
+        }
+        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * RB(mi) + g) * lda + 8 * cb + 2 * t), v);
       }
   }
 #undef RB
