@@ -646,9 +646,14 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // single-job nodes (1; measured slower under load).  CHOL_TRSM_SLABCHAIN.
   const char* esc = getenv("CHOL_TRSM_SLABCHAIN");
   const bool trsm_slabchain = esc && atoi(esc) != 0;
-  // POTRF inner structure: block-level DAG (1) or per-step nodes (0).  CHOL_POTRF_BLOCKDAG.
+  // POTRF inner structure: block-level DAG (one job per node: the chain D -> P -> U -> D
+  // never waits for a whole inner step) or per-step nodes (DIAG b, PANEL b, UPDATE b:
+  // 28 nodes per POTRF instead of 220).  The block DAG shortens the POTRF chain
+  // (785 -> 633 us alone, n=9600 15.1 -> 13.3 ms) but its extra nodes cost dispatch
+  // work: 0.3 ms at n=19200, where the area bound dominates (chain/area ~ 141/N^2 at
+  // nb=960).  Default: block DAG while N <= 16.  CHOL_POTRF_BLOCKDAG=0/1 overrides.
   const char* epb = getenv("CHOL_POTRF_BLOCKDAG");
-  const bool potrf_blockdag = epb ? atoi(epb) != 0 : true;
+  const bool potrf_blockdag = epb ? atoi(epb) != 0 : N <= 16;
   // Multi-GPU: this rank creates the nodes of the tasks that overwrite the tiles it owns
   // (owner-computes), plus one RECV node per remote panel tile it reads.
   auto mine = [&](int64_t i, int64_t j) { return !dist || tile_owner(i, j, dist->p, dist->q) == dist->rank; };

@@ -524,6 +524,10 @@ __device__ __forceinline__ void factor_8x8(double* dd, double* rdv, int* info, i
 //       blocks with FP64 DMMA (A operand = its own solved fragments).
 // A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
 // reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
+#ifndef POTF2_STAMP
+#define POTF2_STAMP(id)  // microbenchmark hook (tools/microbench/potf2_phases.cu)
+#endif
+
 // Per-thread state of potf2_block: the warp's two row blocks rb0 = w, rb1 = NB-1-w; slot
 // SL(mi, cb) of x holds column block cb of row block mi (cb of the first block in slot
 // cb, of the second in slot NB-cb: disjoint since cb <= w < NB-cb).
@@ -549,6 +553,7 @@ __device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, 
   double* pan = c.pans() + (P & 1) * BS * kPanelPitch;
   const int g = s.g, t = s.t;
   bar_sync(kBarCompute, kComputeThreads);  // L_pp and 1/L[j][j] published
+  POTF2_STAMP(0);
   if (s.active) {
     if (c.warp == pw) {
       const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
@@ -576,7 +581,9 @@ __device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, 
         *reinterpret_cast<double2*>(pan + (8 * s.rb(mi) + g) * kPanelPitch + 2 * t) =
             make_double2(s.x[R::sl(mi, P)][0], s.x[R::sl(mi, P)][1]);
   }
+  POTF2_STAMP(1);
   bar_sync(kBarCompute, kComputeThreads);  // panel p published; dd / rdv free
+  POTF2_STAMP(2);
   if constexpr (P + 1 < NB) {
     if (s.active) {
       // (3) rank-8 update of this warp's lower blocks (rb >= cb > p); block (p+1, p+1)
@@ -590,6 +597,7 @@ __device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, 
         dmma884(xd[0], xd[1], -s.x[R::sl(nm, P)][1], bv.y);
         *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
         bar_arrive(kBarDiag, 64);
+        POTF2_STAMP(3);
       }
 #pragma unroll
       for (int cb = P + 1; cb < NB; ++cb) {
@@ -603,6 +611,7 @@ __device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, 
           dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][1], bv.y);
         }
       }
+      POTF2_STAMP(4);
     }
   }
 }
@@ -641,7 +650,9 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
 #pragma unroll 1
     for (int p = 0; p < NB; ++p) {
       bar_sync(kBarDiag, 64);  // diagonal block p is in dd
+      POTF2_STAMP(5);
       if (c.lane == 0) factor_8x8(dd, rdv, info, col0 + 8 * p);
+      POTF2_STAMP(6);
       bar_sync(kBarCompute, kComputeThreads);  // L_pp published
       bar_sync(kBarCompute, kComputeThreads);  // panel p published
     }
