@@ -654,15 +654,51 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // nb=960).  Default: block DAG while N <= 16.  CHOL_POTRF_BLOCKDAG=0/1 overrides.
   const char* epb = getenv("CHOL_POTRF_BLOCKDAG");
   const bool potrf_blockdag = epb ? atoi(epb) != 0 : N <= 16;
+  // Hybrid DAG: the steps k >= k0 are built at BS-block granularity across tasks (the
+  // paper's tasks keep their kernels, but a consumer block waits only for the producer
+  // blocks it reads): POTRF as its block DAG, TRSM as per-slab chains (TS/TU), SYRK and
+  // GEMM as one node per BS x BS output block (K = nb), with block-level edges between
+  // them.  Where the run is chain-bound (small N, the last steps of any N) the next
+  // step's POTRF then starts as soon as its first blocks are updated instead of after
+  // the whole SYRK.  A larger block region costs efficiency (K = BS TRSM updates, more
+  // nodes): measured best m (tools/tail_sweep.py, nb = 960) is 4 for N = 4..10 and 2 for
+  // N = 12..24 (n=3840 3.76 -> 2.82 ms, n=9600 13.07 -> 12.18, n=19200 71.82 -> 71.57).
+  // Single GPU only.  CHOL_BLOCK_TAIL=m overrides (m steps).
+  const char* ebt = getenv("CHOL_BLOCK_TAIL");
+  int block_tail = ebt ? atoi(ebt) : (N <= 10 ? 4 : 2);
+  if (dist) block_tail = 0;
+  const int k0 = (int)N - std::max(0, std::min(block_tail, (int)N));
+  // blocked-region TRSM: per-slab TS/TU chains (0) or one left-looking slab job per
+  // slab node (1).  CHOL_TAIL_TRSM.
+  const char* ett = getenv("CHOL_TAIL_TRSM");
+  const bool tail_trsm_slab = ett && atoi(ett) == 1;
   // Multi-GPU: this rank creates the nodes of the tasks that overwrite the tiles it owns
   // (owner-computes), plus one RECV node per remote panel tile it reads.
   auto mine = [&](int64_t i, int64_t j) { return !dist || tile_owner(i, j, dist->p, dist->q) == dist->rank; };
   std::vector<int> publish;  // per node: tile made final (published to other ranks) or -1
   // ---- nodes and jobs, Algorithm 1 order
   std::vector<int> first_node(n_tasks(N), -1), last_node(n_tasks(N), -1);
+  // blocked tasks (k >= k0): per BS x BS block of the tile the task writes, the node that
+  // first touches it (tentry) and the node that leaves it final (tfin); TRSM: the node
+  // that finishes each row slab (tslab)
+  std::vector<std::vector<int>> tentry(n_tasks(N)), tfin(n_tasks(N)), tslab(n_tasks(N));
+  const int nbb2 = nbb * nbb;
+  auto gate_of = [&](int tid, int type, int i, int k) {
+    // job-less node in front of a blocked task's entry nodes: the target of task-level
+    // dependencies (streamed tile arrival at k = 0)
+    const int gate = B.add_node(tid, type, i, k);
+    std::vector<int> seen;
+    for (int e : tentry[tid])
+      if (e >= 0 && std::find(seen.begin(), seen.end(), e) == seen.end()) {
+        B.edge(gate, e);
+        seen.push_back(e);
+      }
+    first_node[tid] = gate;
+  };
   for (int k = 0; k < N; ++k) {
     const int pid = (int)id_potrf(N, k);
-    if (mine(k, k) && !potrf_blockdag) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
+    const bool blk = k >= k0;
+    if (mine(k, k) && !potrf_blockdag && !blk) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
       int prev = -1;
       for (int b = 0; b < nbb; ++b) {
         const int dn = B.add_node(pid, T_POTRF, k, k);
@@ -692,6 +728,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       // never waits for a whole column or trailing update of the step.  D(nbb-1) is the
       // sink (every inner node is its ancestor).
       std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1);
+      if (blk) tentry[pid].assign(nbb2, -1), tfin[pid].assign(nbb2, -1);
       for (int b = 0; b < nbb; ++b) {
         const int dn = B.add_node(pid, T_POTRF, k, k);
         B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
@@ -713,10 +750,63 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
             if (q != r) B.edge(pan[q], un);
             if (lastU[r * nbb + q] >= 0) B.edge(lastU[r * nbb + q], un);  // same block, previous step
             lastU[r * nbb + q] = un;
+            if (blk && b == 0) tentry[pid][r * nbb + q] = un;
           }
+        if (blk) {
+          tfin[pid][b * nbb + b] = dn;
+          if (b == 0) tentry[pid][0] = dn;
+          for (int r = b + 1; r < nbb; ++r) {
+            tfin[pid][r * nbb + b] = pan[r];
+            if (b == 0) tentry[pid][r * nbb] = pan[r];
+          }
+        }
       }
+      if (blk && k == 0) gate_of(pid, T_POTRF, k, k);
     }
-    for (int i = k + 1; i < N; ++i) {
+    for (int i = k + 1; i < N && blk; ++i) {
+      // blocked TRSM_i_k: per row slab sl, TS(c, sl) / TU(c, sl, c') single-job nodes
+      // (or one slab job per node), edges from the POTRF_k blocks each one reads:
+      // TS(c, sl) <- L_kk[c,c] = D(c); TU(c, sl, c') <- L_kk[c',c] = P(c',c)
+      const int tid = (int)id_trsm(N, i, k);
+      tentry[tid].assign(nbb2, -1);
+      tfin[tid].assign(nbb2, -1);
+      tslab[tid].assign(nbb, -1);
+      const int exit_ = B.add_node(tid, T_TRSM, i, k);  // job-less: the tile is final (publish)
+      for (int sl = 0; sl < nbb; ++sl) {
+        if (tail_trsm_slab) {
+          const int sn = B.add_node(tid, T_TRSM, i, k);
+          B.add_job(sn, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
+          B.edge(tfin[pid][(nbb - 1) * nbb + nbb - 1], sn);  // D(nbb-1): all of L_kk
+          for (int c = 0; c < nbb; ++c) tentry[tid][sl * nbb + c] = tfin[tid][sl * nbb + c] = sn;
+          tslab[tid][sl] = sn;
+          B.edge(sn, exit_);
+          continue;
+        }
+        std::vector<int> lastTU(nbb, -1);
+        for (int cb = 0; cb < nbb; ++cb) {
+          const int ts = B.add_node(tid, T_TRSM, i, k);
+          B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+          B.edge(tfin[pid][cb * nbb + cb], ts);
+          if (cb > 0) B.edge(lastTU[cb], ts);
+          else tentry[tid][sl * nbb] = ts;
+          tfin[tid][sl * nbb + cb] = ts;
+          for (int c2 = cb + 1; c2 < nbb; ++c2) {
+            const int tu = B.add_node(tid, T_TRSM, i, k);
+            B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
+            B.edge(ts, tu);
+            B.edge(tfin[pid][c2 * nbb + cb], tu);
+            if (lastTU[c2] >= 0) B.edge(lastTU[c2], tu);
+            else tentry[tid][sl * nbb + c2] = tu;
+            lastTU[c2] = tu;
+          }
+        }
+        tslab[tid][sl] = tfin[tid][sl * nbb + nbb - 1];
+        B.edge(tslab[tid][sl], exit_);
+      }
+      last_node[tid] = exit_;
+      if (k == 0) gate_of(tid, T_TRSM, i, k);
+    }
+    for (int i = k + 1; i < N && !blk; ++i) {
       if (!mine(i, k)) continue;
       const bool trsm_slab = trsm_slab_all && k < N - 1 - trsm_tail && i - k > trsm_dist;
       if (trsm_slab) {  // one left-looking row-slab job per BS rows
@@ -780,7 +870,32 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         }
       }
     }
-    for (int j = k + 1; j < N; ++j) {
+    for (int j = k + 1; j < N && blk; ++j) {
+      // blocked SYRK_j_k / GEMM_i_j_k: one node per output block, K = nb
+      const int sid = (int)id_syrk(N, j, k);
+      tentry[sid].assign(nbb2, -1);
+      for (int bm = 0; bm < nbb; ++bm)
+        for (int bn = 0; bn <= bm; ++bn) {
+          const int n = B.add_node(sid, T_SYRK, j, k);
+          B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
+          tentry[sid][bm * nbb + bn] = n;
+        }
+      tfin[sid] = tentry[sid];
+      if (k == 0) gate_of(sid, T_SYRK, j, k);
+      for (int i = j + 1; i < N; ++i) {
+        const int gid = (int)id_gemm(N, i, j, k);
+        tentry[gid].assign(nbb2, -1);
+        for (int bm = 0; bm < nbb; ++bm)
+          for (int bn = 0; bn < nbb; ++bn) {
+            const int g = B.add_node(gid, T_GEMM, i, k);
+            B.add_job(g, Job{J_UPD, (int16_t)i, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
+            tentry[gid][bm * nbb + bn] = g;
+          }
+        tfin[gid] = tentry[gid];
+        if (k == 0) gate_of(gid, T_GEMM, i, k);
+      }
+    }
+    for (int j = k + 1; j < N && !blk; ++j) {
       const int sid = (int)id_syrk(N, j, k);
       if (mine(j, j)) {
         const int n = B.add_node(sid, T_SYRK, j, k);
@@ -808,7 +923,48 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     std::vector<std::pair<int64_t, int64_t>> E;
     std::vector<int> type_of;
     build_task_dag(N, E, type_of);
-    for (auto& e : E) B.edge(last_node[e.first], first_node[e.second]);
+    // tile written by a task (i, j) -- Algorithm 1 visit order of taskid.h
+    std::vector<int2> wtile(n_tasks(N));
+    for (int64_t k = 0; k < N; ++k) {
+      wtile[id_potrf(N, k)] = make_int2((int)k, (int)k);
+      for (int64_t i = k + 1; i < N; ++i) wtile[id_trsm(N, i, k)] = make_int2((int)i, (int)k);
+      for (int64_t j = k + 1; j < N; ++j) {
+        wtile[id_syrk(N, j, k)] = make_int2((int)j, (int)j);
+        for (int64_t i = j + 1; i < N; ++i) wtile[id_gemm(N, i, j, k)] = make_int2((int)i, (int)j);
+      }
+    }
+    for (auto& e : E) {
+      const int64_t a = e.first, b = e.second;
+      if (tentry[b].empty()) {  // task-level consumer (k < k0)
+        B.edge(last_node[a], first_node[b]);
+        continue;
+      }
+      const int2 tb = wtile[b];
+      const bool diag = tb.x == tb.y;
+      if (tentry[a].empty()) {  // task-level producer of a blocked consumer: every entry waits
+        std::vector<int> seen;
+        for (int x : tentry[b])
+          if (x >= 0 && std::find(seen.begin(), seen.end(), x) == seen.end()) {
+            B.edge(last_node[a], x);
+            seen.push_back(x);
+          }
+        continue;
+      }
+      if (type_of[a] == T_POTRF && type_of[b] == T_TRSM) continue;  // block edges made with the TRSM nodes
+      for (int bm = 0; bm < nbb; ++bm)
+        for (int bn = 0; bn < nbb; ++bn) {
+          if (diag && bn > bm) continue;  // lower blocks of a diagonal tile
+          const int x = tentry[b][bm * nbb + bn];
+          if (x < 0) continue;
+          if (type_of[a] == T_TRSM) {  // L_ik read by SYRK / GEMM: row slabs bm and / or bn
+            const int pi = wtile[a].x;
+            if (pi == tb.x) B.edge(tslab[a][bm], x);
+            if (pi == tb.y && !(pi == tb.x && bm == bn)) B.edge(tslab[a][bn], x);
+          } else {  // the same tile, block by block (SYRK->POTRF, SYRK->SYRK, GEMM->GEMM, GEMM->TRSM)
+            B.edge(tfin[a][bm * nbb + bn], x);
+          }
+        }
+    }
     // Streamed input (chol_factor from host memory): the first task touching a tile
     // waits for the tile's arrival flag (the copy engine writes it after the tile).
     // Tiles arrive in row-major tile order (row i: tiles (i,0..i)); the watch list

@@ -19,9 +19,16 @@ def _lib():
 
 @pytest.mark.parametrize("policy", [0, 1, 2])
 @pytest.mark.parametrize("n,nb", [(1920, 96), (3840, 960), (768, 64)])
-def test_trace_respects_dag(n, nb, policy):
+@pytest.mark.parametrize("block_tail", [0, 2, 99])
+def test_trace_respects_dag(n, nb, policy, block_tail, monkeypatch):
+    """block_tail = m: the last m steps use block-level dependencies between tasks (hybrid
+    DAG): there a task may start once the producer blocks it reads are
+    done, so task-level edges into those steps only guarantee t0(b) >= t0(a) and
+    t1(b) >= t1(a); every other edge is strict (t0(b) >= t1(a))."""
     c = _lib()
     N = n // nb
+    monkeypatch.setenv("CHOL_BLOCK_TAIL", str(block_tail))
+    k0 = N - min(block_tail, N)
     with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=policy, trace=2) as p:
         c.chol_generate(p.h, 3, 0)
         assert c.chol_factor_inplace(p.h) == 0
@@ -46,7 +53,11 @@ def test_trace_respects_dag(n, nb, policy):
     for r in trec:
         assert r["t1_ns"] >= r["t0_ns"]
     for a, b in E:  # task-level direct dependencies: successor starts after predecessor ends
-        assert trec[b]["t0_ns"] >= trec[a]["t1_ns"], (ts[a].name, ts[b].name)
+        if ts[a].k >= k0:  # both in the block-level region
+            assert trec[b]["t0_ns"] >= trec[a]["t0_ns"], (ts[a].name, ts[b].name)
+            assert trec[b]["t1_ns"] >= trec[a]["t1_ns"], (ts[a].name, ts[b].name)
+        else:
+            assert trec[b]["t0_ns"] >= trec[a]["t1_ns"], (ts[a].name, ts[b].name)
     # job level: each job once, no overlap on a worker, busy <= workers * span
     t0 = jt[:, 0].astype(np.int64)
     t1 = jt[:, 1].astype(np.int64)
