@@ -218,6 +218,48 @@ int chol_task_id(int64_t N, int type, int i, int j, int k, int64_t* id);
  * out[4] GEMM-peak bound (n^3/3) / (M 2 nb^3 / T_thr_G), out[5] max(area, cp). */
 int chol_bounds(int64_t n, int64_t nb, int ngpus, const double* T_lat, const double* T_thr, double* out);
 
+/* ---- platform model (host only): the paper's LP bounds over several resource types and
+ * its scheduler simulation (§III-A, §IV-C, §V;
+ * SURVEY §8f NEXT-1).  Times are per task of each type on one processing element of a
+ * class, in seconds; a negative or infinite time means the class cannot run that type. */
+#define CHOL_SIM_MAX_CLASSES 4
+
+/* LP of L349-359 (area bound; mixed != 0 adds the chain constraint of L390-396:
+ *   sum_r n_rP T_rP + (N-1) T*_T + (N-1) T*_S <= l, T* = fastest time over the classes)
+ * over nclasses resource types with workers[r] processing elements and times
+ * time[r*4 + t] (t = POTRF, TRSM, SYRK, GEMM).  The n_rt are relaxed to reals (reading
+ * R10).  *l = optimal makespan bound; n_rt (may be NULL) = optimal task counts per class
+ * and type (row-major nclasses x 4).  Errors: -1 N <= 0; -6 bad arguments or a task type
+ * no class can run. */
+int chol_lp_bound(int64_t N, int nclasses, const int* workers, const double* time, int mixed, double* l,
+                  double* n_rt);
+
+/* Scheduler policies of the simulation (StarPU's, L645-660). */
+enum {
+  CHOL_SIM_DMDA = 0, /* ready tasks (release order) go to the worker with the minimum estimated
+                        completion time; each worker runs its queue in FIFO order */
+  CHOL_SIM_DMDAS = 1 /* the same, ready tasks and worker queues in bottom-level priority order
+                        (longest path to an exit task with each type's fastest time, L655-660) */
+};
+typedef struct {
+  int nclasses;                            /* 1 .. CHOL_SIM_MAX_CLASSES */
+  int workers[CHOL_SIM_MAX_CLASSES];       /* processing elements per class */
+  double time[CHOL_SIM_MAX_CLASSES][4];    /* seconds per task, [class][POTRF, TRSM, SYRK, GEMM] */
+  int policy;                              /* CHOL_SIM_DMDA / CHOL_SIM_DMDAS */
+  int gemm_syrk_class;                     /* static rule (L1000-1007): SYRK/GEMM only on this class; -1 off */
+  int trsm_far_class;                      /* static rule (L1019-1025): TRSM_i_k with i-k >= */
+  int trsm_far_distance;                   /*   trsm_far_distance only on trsm_far_class; -1 off */
+} chol_sim_opts_t;
+
+/* Discrete-event replay of the Algorithm 1 task DAG for N tiles per side on the
+ * platform described by *opts (no data transfers modelled, reading R18).  Ties: events
+ * at equal times are processed together; a task goes to the lowest-numbered worker among
+ * equal completion times; workers are numbered class by class.  *makespan in seconds;
+ * recs (may be NULL; at most cap written, indexed by chol_task_id) receive each task's
+ * class (field gpu), worker, and t0/t1 in ns.  Errors: -1 N <= 0, -4 null pointer,
+ * -6 bad options or a task no class may run. */
+int chol_simulate(int64_t N, const chol_sim_opts_t* opts, double* makespan, chol_task_rec_t* recs, int64_t cap);
+
 #ifdef __cplusplus
 }
 #endif

@@ -37,6 +37,17 @@ class chol_task_rec_t(ctypes.Structure):
                 ("t0_ns", ctypes.c_uint64), ("t1_ns", ctypes.c_uint64)]
 
 
+SIM_MAX_CLASSES = 4
+SIM_DMDA, SIM_DMDAS = 0, 1
+
+
+class chol_sim_opts_t(ctypes.Structure):
+    _fields_ = [("nclasses", ctypes.c_int), ("workers", ctypes.c_int * SIM_MAX_CLASSES),
+                ("time", (ctypes.c_double * 4) * SIM_MAX_CLASSES), ("policy", ctypes.c_int),
+                ("gemm_syrk_class", ctypes.c_int), ("trsm_far_class", ctypes.c_int),
+                ("trsm_far_distance", ctypes.c_int)]
+
+
 def _load():
     if not os.path.exists(LIB_PATH):
         raise ImportError(f"{LIB_PATH} is missing: run __graft_entry__.build() (there is no CPU fallback)")
@@ -74,6 +85,8 @@ def _load():
         "chol_wait": ([P, ctypes.POINTER(i32)], i32),
         "chol_dist_layout": ([i64, i64, i32, i32, i32, ctypes.POINTER(i32), ctypes.POINTER(i32),
                               ctypes.POINTER(ctypes.c_int32), i64], i32),
+        "chol_lp_bound": ([i64, i32, ctypes.POINTER(i32), dp, i32, dp, dp], i32),
+        "chol_simulate": ([i64, ctypes.POINTER(chol_sim_opts_t), dp, ctypes.POINTER(chol_task_rec_t), i64], i32),
     }
     for name, (args, res) in sig.items():
         f = getattr(L, name)
@@ -87,7 +100,8 @@ EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_dest
             "chol_generate", "chol_scatter", "chol_gather", "chol_factor_inplace", "chol_last_times",
             "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
             "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
-            "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout")
+            "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
+            "chol_lp_bound", "chol_simulate")
 
 
 def _ptr(x) -> int:
@@ -238,6 +252,41 @@ def chol_bounds(n: int, nb: int, ngpus: int, T_lat, T_thr) -> dict:
     out = (ctypes.c_double * 6)()
     _check(_lib.chol_bounds(n, nb, ngpus, lat, thr, out), "chol_bounds")
     return dict(zip(BOUND_NAMES, list(out)))
+
+
+def chol_lp_bound(N: int, workers, times, mixed: bool = True):
+    """LP makespan bound over resource classes: workers[r], times[r] =
+    [POTRF, TRSM, SYRK, GEMM] seconds (negative / inf = cannot run).  Returns (l, n_rt)."""
+    R = len(workers)
+    w = (ctypes.c_int * R)(*workers)
+    t = (ctypes.c_double * (4 * R))(*[float(v) for row in times for v in row])
+    l = ctypes.c_double()
+    nrt = (ctypes.c_double * (4 * R))()
+    _check(_lib.chol_lp_bound(N, R, w, t, int(bool(mixed)), ctypes.byref(l), nrt), "chol_lp_bound")
+    return l.value, [list(nrt[4 * r:4 * r + 4]) for r in range(R)]
+
+
+def chol_simulate(N: int, workers, times, policy: int = SIM_DMDAS, gemm_syrk_class: int = -1,
+                  trsm_far_class: int = -1, trsm_far_distance: int = 1, records: bool = False):
+    """Replay of the Algorithm 1 DAG on a platform of resource classes under dmda / dmdas
+    and the paper's static rules (chol_simulate in include/chol.h).  Returns the makespan
+    (seconds) and, with records=True, the per-task records (chol_task_id order)."""
+    o = chol_sim_opts_t()
+    o.nclasses = len(workers)
+    for r, (m, row) in enumerate(zip(workers, times)):
+        o.workers[r] = m
+        for t in range(4):
+            o.time[r][t] = float(row[t])
+    o.policy, o.gemm_syrk_class, o.trsm_far_class, o.trsm_far_distance = policy, gemm_syrk_class, trsm_far_class, \
+        trsm_far_distance
+    mk = ctypes.c_double()
+    nt = N + N * (N - 1) + N * (N - 1) * (N - 2) // 6
+    recs = (chol_task_rec_t * nt)() if records else None
+    _check(_lib.chol_simulate(N, ctypes.byref(o), ctypes.byref(mk), recs, nt if records else 0), "chol_simulate")
+    if not records:
+        return mk.value
+    return mk.value, [{"type": r.type, "cls": r.gpu, "worker": r.worker, "i": r.i, "j": r.j, "k": r.k,
+                       "t0_ns": r.t0_ns, "t1_ns": r.t1_ns} for r in recs]
 
 
 def chol_plan_dist(n: int, nb: int, nranks: int, rank: int, **opts) -> int:
