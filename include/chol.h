@@ -25,6 +25,7 @@
  *   -7  chol_trace before any chol_factor*, or tracing disabled
  *   -8  operation not supported by this build (e.g. ngpus > 1 in one process)
  *   -9  device out of memory while planning
+ *   -10 chol_solve without a successful factorization in the plan
  *   -100 - e   CUDA runtime error e
  *   -200 - e   NCCL error e
  * A non-SPD input is NOT an error status: it is reported through *info.
@@ -186,6 +187,22 @@ int chol_dist_connect(chol_plan_t p, const void* blobs, int64_t stride);
 int chol_get_dist(chol_plan_t p, int* rank, int* nranks, int* grid_p, int* grid_q, int64_t* nowned, int64_t* nslots);
 int chol_factor_async(chol_plan_t p);
 int chol_wait(chol_plan_t p, int* info);
+
+/* Solve A X = B with the factor of the plan's last successful chol_factor* (the tiles
+ * hold L): L Y = B, then L^T X = Y -- the use of A = L L^T (
+ * SURVEY §8f NEXT-2).  B: n x nrhs, ROW-MAJOR with leading dimension ldb >= nrhs, host
+ * or device pointer (on the plan's device), caller-owned; overwritten by X.  The call
+ * is synchronous.  Method: forward and backward sweeps over bs-row blocks (bs = the
+ * plan's block, 96 at nb = 960), each diagonal block applied through its explicit
+ * inverse (computed once per factorization, n x bs doubles of plan workspace); the
+ * rounding therefore differs from plain substitution.  Single-GPU plans
+ * only.  Errors: -4 null / misaligned B or plan, -5 ldb < nrhs, -6 nrhs < 1, -8 a
+ * multi-GPU plan, -9 out of memory, -10 no successful factorization (none yet, or the
+ * last one reported info > 0), -100 - e CUDA errors. */
+int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs);
+/* Timing of the last chol_solve: total (copies in/out included) and the two sweeps
+ * (plus the diagonal-block inverses when they were recomputed), seconds. */
+int chol_last_solve_times(chol_plan_t p, double* total_s, double* sweeps_s);
 
 /* Number of kernel launches the last chol_factor* issued (the persistent scheduler
  * issues 2: queue init + the scheduler kernel). */

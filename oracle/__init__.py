@@ -50,6 +50,8 @@ def lib():
         L.oracle_tile_syrk.restype = None
         L.oracle_tile_gemm.argtypes = [i64, dp, i64, dp, i64, dp, i64]
         L.oracle_tile_gemm.restype = None
+        L.oracle_chol_solve.argtypes = [i64, dp, i64, dp, i64, i64]
+        L.oracle_chol_solve.restype = None
         L.oracle_num_threads.argtypes = [ip]
         L.oracle_num_threads.restype = ip
         _lib = L
@@ -109,6 +111,17 @@ def tile_gemm(Lik: np.ndarray, Ljk: np.ndarray, Aij: np.ndarray) -> np.ndarray:
     nb = C.shape[0]
     lib().oracle_tile_gemm(nb, _p(a), nb, _p(b), nb, _p(C), nb)
     return C
+
+
+def chol_solve(L: np.ndarray, B: np.ndarray) -> np.ndarray:
+    """X with L L^T X = B by forward then backward substitution (NEXT-2, L166-171)."""
+    Lc = np.ascontiguousarray(L, dtype=np.float64)
+    X = np.array(B, dtype=np.float64, order="C", copy=True)
+    if X.ndim == 1:
+        X = X.reshape(-1, 1)
+    n, nrhs = X.shape
+    lib().oracle_chol_solve(n, _p(Lc), n, _p(X), nrhs, nrhs)
+    return X.reshape(B.shape)
 
 
 def num_threads(nthreads: int = 0) -> int:

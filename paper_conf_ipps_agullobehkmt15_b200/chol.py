@@ -86,6 +86,8 @@ def _load():
         "chol_dist_layout": ([i64, i64, i32, i32, i32, ctypes.POINTER(i32), ctypes.POINTER(i32),
                               ctypes.POINTER(ctypes.c_int32), i64], i32),
         "chol_lp_bound": ([i64, i32, ctypes.POINTER(i32), dp, i32, dp, dp], i32),
+        "chol_solve": ([P, vp, i64, i64], i32),
+        "chol_last_solve_times": ([P, dp, dp], i32),
         "chol_simulate": ([i64, ctypes.POINTER(chol_sim_opts_t), dp, ctypes.POINTER(chol_task_rec_t), i64], i32),
     }
     for name, (args, res) in sig.items():
@@ -101,7 +103,7 @@ EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_dest
             "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
             "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
             "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
-            "chol_lp_bound", "chol_simulate")
+            "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times")
 
 
 def _ptr(x) -> int:
@@ -254,6 +256,17 @@ def chol_bounds(n: int, nb: int, ngpus: int, T_lat, T_thr) -> dict:
     return dict(zip(BOUND_NAMES, list(out)))
 
 
+def chol_solve(plan: int, B, ldb: int, nrhs: int) -> None:
+    """A X = B with the plan's factor; B (n x nrhs row-major, host or device) is overwritten."""
+    _check(_lib.chol_solve(plan, _ptr(B), ldb, nrhs), "chol_solve")
+
+
+def chol_last_solve_times(plan: int) -> tuple[float, float]:
+    a, b = ctypes.c_double(), ctypes.c_double()
+    _check(_lib.chol_last_solve_times(plan, ctypes.byref(a), ctypes.byref(b)), "chol_last_solve_times")
+    return a.value, b.value
+
+
 def chol_lp_bound(N: int, workers, times, mixed: bool = True):
     """LP makespan bound over resource classes: workers[r], times[r] =
     [POTRF, TRSM, SYRK, GEMM] seconds (negative / inf = cannot run).  Returns (l, n_rt)."""
@@ -380,6 +393,11 @@ class Plan:
     def factor(self, A, L=None, lda: int | None = None, ldl: int | None = None) -> int:
         L = A if L is None else L
         return chol_factor(self.h, A, lda or self.n, L, ldl or self.n)
+
+    def solve(self, B, ldb: int | None = None) -> None:
+        """A X = B in place (B: n x nrhs row-major, host or device) with this plan's factor."""
+        nrhs = 1 if len(B.shape) == 1 else B.shape[1]
+        chol_solve(self.h, B, ldb or nrhs, nrhs)
 
     def close(self):
         if self.h:

@@ -17,6 +17,7 @@
 #include "dag.h"
 #include "kernels.h"
 #include "sched.h"
+#include "solve.h"
 #include "taskid.h"
 
 using namespace chol;
@@ -59,6 +60,16 @@ struct chol_plan_s {
   int* h_epoch = nullptr;      // pinned source of the 4-byte arrival-flag copies
   cudaStream_t s_in = nullptr, s_out = nullptr;
   bool streamed_run = false;
+  // ---- triangular solves with the factor (chol_solve, solve.cu)
+  int last_info = -1;           // info of the last completed factorization (-1: none)
+  double* d_inv = nullptr;      // diagonal-block inverses + chain matrices (3 n x bs doubles)
+  bool inv_valid = false;
+  double* d_rhs = nullptr;      // padded right-hand sides, n x ldw
+  size_t rhs_cap = 0;           // doubles
+  int* d_solve_ctl = nullptr;   // counters + flags
+  size_t ctl_cap = 0;           // ints
+  double last_solve_s = 0.0, last_sweeps_s = 0.0;
+  cudaEvent_t ev4 = nullptr, ev5 = nullptr;
 };
 
 #define CUDA_TRY(x)                                   \
@@ -102,6 +113,7 @@ extern "C" const char* chol_strerror(int s) {
     case -7: return "no trace available (factor first with opts.trace = 1)";
     case -8: return "not supported by this build";
     case -9: return "device out of memory";
+    case -10: return "no successful factorization in the plan";
   }
   if (s <= -200) return "NCCL error";
   if (s <= -100) return cudaGetErrorString((cudaError_t)(-100 - s));
@@ -122,6 +134,11 @@ extern "C" int chol_destroy(chol_plan_t p) {
   cudaSetDevice(p->device);
   if (p->stream) cudaStreamSynchronize(p->stream);
   for (void* ptr : p->ipc_opened) cudaIpcCloseMemHandle(ptr);
+  cudaFree(p->d_inv);
+  cudaFree(p->d_rhs);
+  cudaFree(p->d_solve_ctl);
+  if (p->ev4) cudaEventDestroy(p->ev4);
+  if (p->ev5) cudaEventDestroy(p->ev5);
   cudaFree(p->d_slot_map);
   cudaFree(p->d_owner_slot);
   cudaFree(p->d_owned_tile);
@@ -587,7 +604,9 @@ static int finish_info(chol_plan_s* p, int* info) {
   CUDA_TRY(cudaEventElapsedTime(&ms, p->ev0, p->ev1));
   p->last_factor_s = ms * 1e-3;
   p->factored = true;
-  if (info) *info = (h == INT_MAX) ? 0 : h;
+  p->last_info = (h == INT_MAX) ? 0 : h;
+  p->inv_valid = false;  // a new factor: the diagonal-block inverses are stale
+  if (info) *info = p->last_info;
   return 0;
 }
 
@@ -733,6 +752,86 @@ extern "C" int chol_last_times(chol_plan_t p, double* factor_s, double* layout_s
   if (!p) return -4;
   if (factor_s) *factor_s = p->last_factor_s;
   if (layout_s) *layout_s = p->last_layout_s;
+  return 0;
+}
+
+// ------------------------------------------------------------------ solve
+// A X = B with the factor of the last successful factorization (solve.cu): the
+// right-hand sides are copied (host or device, any ldb) into a padded device buffer,
+// solved by the forward and backward sweeps, and copied back.
+extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
+  if (!p || !B || (reinterpret_cast<uintptr_t>(B) & 7)) return -4;
+  if (nrhs < 1) return -6;
+  if (ldb < nrhs) return -5;
+  if (p->dist) return -8;
+  if (!p->factored || p->last_info != 0) return -10;
+  cudaSetDevice(p->device);
+  const int64_t n = p->n;
+  const int rc = nrhs <= 8 ? 8 : 32;  // columns per work item (lanes of a row group)
+  const int nchunks = (int)((nrhs + rc - 1) / rc), ldw = rc * nchunks;
+  const int64_t nblocks = n / p->bs;
+  const size_t need = (size_t)n * ldw, ctl = 2 + 2 * (size_t)nblocks * nchunks;
+  if (!p->d_inv) {
+    cudaError_t e = cudaMalloc(&p->d_inv, 3 * (size_t)n * p->bs * sizeof(double));
+    if (e) return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
+  }
+  if (p->rhs_cap < need) {
+    cudaFree(p->d_rhs);
+    p->d_rhs = nullptr;
+    p->rhs_cap = 0;
+    cudaError_t e = cudaMalloc(&p->d_rhs, need * sizeof(double));
+    if (e) return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
+    p->rhs_cap = need;
+  }
+  if (p->ctl_cap < ctl) {
+    cudaFree(p->d_solve_ctl);
+    p->d_solve_ctl = nullptr;
+    p->ctl_cap = 0;
+    cudaError_t e = cudaMalloc(&p->d_solve_ctl, ctl * sizeof(int));
+    if (e) return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
+    p->ctl_cap = ctl;
+  }
+  if (!p->ev4) {
+    CUDA_TRY(cudaEventCreate(&p->ev4));
+    CUDA_TRY(cudaEventCreate(&p->ev5));
+  }
+  CUDA_TRY(cudaEventRecord(p->ev2, p->stream));
+  if (ldw != nrhs) CUDA_TRY(cudaMemsetAsync(p->d_rhs, 0, need * sizeof(double), p->stream));
+  CUDA_TRY(cudaMemcpy2DAsync(p->d_rhs, ldw * 8, B, ldb * 8, nrhs * 8, n, cudaMemcpyDefault, p->stream));
+  SolveArgs a{};
+  a.tiles = p->tiles;
+  a.n = n;
+  a.nb = (int)p->nb;
+  a.sb = p->bs;
+  a.inv = p->d_inv;
+  a.inv_valid = p->inv_valid;
+  a.W = p->d_rhs;
+  a.ldw = ldw;
+  a.nchunks = nchunks;
+  a.rc = rc;
+  a.ctl = p->d_solve_ctl;
+  a.sms = p->sms;
+  int nl = 0;
+  CUDA_TRY(cudaEventRecord(p->ev4, p->stream));
+  CUDA_TRY(solve_run(a, p->stream, &nl));
+  CUDA_TRY(cudaEventRecord(p->ev5, p->stream));
+  p->inv_valid = true;
+  CUDA_TRY(cudaMemcpy2DAsync(B, ldb * 8, p->d_rhs, ldw * 8, nrhs * 8, n, cudaMemcpyDefault, p->stream));
+  CUDA_TRY(cudaEventRecord(p->ev3, p->stream));
+  CUDA_TRY(cudaStreamSynchronize(p->stream));
+  float ms = 0.f, ms2 = 0.f;
+  CUDA_TRY(cudaEventElapsedTime(&ms, p->ev2, p->ev3));
+  CUDA_TRY(cudaEventElapsedTime(&ms2, p->ev4, p->ev5));
+  p->last_solve_s = ms * 1e-3;
+  p->last_sweeps_s = ms2 * 1e-3;
+  p->last_launches = nl;
+  return 0;
+}
+
+extern "C" int chol_last_solve_times(chol_plan_t p, double* total_s, double* sweeps_s) {
+  if (!p) return -4;
+  if (total_s) *total_s = p->last_solve_s;
+  if (sweeps_s) *sweeps_s = p->last_sweeps_s;
   return 0;
 }
 

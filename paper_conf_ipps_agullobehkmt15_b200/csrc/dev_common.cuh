@@ -69,6 +69,14 @@ __device__ __forceinline__ void tma_load_3d(void* dst, const CUtensorMap* map, u
 }
 // Order this thread's generic-proxy accesses before later async-proxy (TMA) ones.
 __device__ __forceinline__ void fence_proxy_async() { asm volatile("fence.proxy.async;" ::: "memory"); }
+// 1-D bulk copy global -> shared through the TMA engine (bytes % 16 == 0, both addresses
+// 16-byte aligned), completing as transaction bytes on the mbarrier
+__device__ __forceinline__ void bulk_load(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(smem_u32(bar))
+      : "memory");
+}
 
 // ---------------------------------------------------------------- shared loads
 // Explicit ld.shared (not a generic LD): the consumer's reads of a TMA stage must be

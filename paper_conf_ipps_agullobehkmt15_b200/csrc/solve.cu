@@ -1,0 +1,296 @@
+// Triangular solves with the factor held in a plan's tile store:
+// A X = B as L Y = B (forward) then L^T X = Y (backward) -- the use of the Cholesky
+// factor (A = L L^T "is used to solve" the SPD system).
+//
+// B200 form.  The right-hand sides live in a padded device buffer W (n x ldw, row-major,
+// ldw = 32 * nchunks); the unknowns are cut into SB-row blocks (SB = the plan's block, 96
+// at nb = 960) and the right-hand sides into chunks of 32 columns (one per lane).  One
+// work item = (block row b, chunk) computes
+//     forward:  Y_b = inv(L_bb) (B_b - sum_{c<b} L_bc Y_c)
+//     backward: X_b = inv(L_bb)^T (Y_b - sum_{c>b} L_cb^T X_c)
+// where inv(L_bb) is the inverse of the SB x SB diagonal block, computed once per
+// factorization (k_diag_inv): the sequential substitution inside a block becomes a small
+// product, so the chain from block to block is one flag hop plus one SB x SB x 32 FMA
+// pass.  Items are claimed in dependency order with an atomic counter by a persistent
+// grid (a CTA only waits on items claimed before its own, so every wait ends); a block's
+// result is published with a release flag, consumers acquire it.  Each CTA stages the
+// L block it needs in shared memory before waiting for the flag, so the HBM read of L
+// (the dominant traffic: the lower triangle once per sweep) overlaps the wavefront.
+// Arithmetic: FP64 FMA (SIMT; on B200 DFMA and DMMA share the 37 TF/s FP64 peak).
+#include <cuda.h>
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "dev_common.cuh"
+#include "solve.h"
+#include "taskid.h"
+
+namespace chol {
+
+constexpr int kSolveThreads = 256;
+
+template <int SB, int RC>
+struct SolveCfg {
+  static constexpr int P = SB + 2;                   // shared pitch (doubles): rows stay 16-byte aligned
+  static constexpr int G = kSolveThreads / RC;       // row groups (thread t: column t % RC, group t / RC)
+  static constexpr int RPT = SB / G;                 // rows per thread
+  static constexpr int kLBytes = SB * P * 8;
+  static constexpr int kSmem = 2 * kLBytes + SB * RC * 8 + 16;  // k_sweep: 2 L buffers + Y block + item
+  static_assert(SB % G == 0, "rows per thread");
+};
+constexpr int kInvPitch = 97;  // k_diag_inv (odd pitch: the column-per-thread walks are conflict-free)
+
+// first element of SB-block (R, C), R >= C, of the factor in the tile store (ld = nb)
+__device__ __forceinline__ const double* lblock(const double* tiles, int nb, int sb, int R, int C) {
+  const int64_t r = (int64_t)R * sb, c = (int64_t)C * sb;
+  const int64_t i = r / nb, j = c / nb;
+  return tiles + tile_index(i, j) * (int64_t)nb * nb + (r - i * nb) * nb + (c - j * nb);
+}
+
+// acc[i] += sum_k Lop[row_i][k] * Ys[k][col]; Lop = Ls (TRANS = false) or Ls^T (TRANS =
+// true: the backward sweep reads L_cb^T and inv(L_bb)^T straight from the untransposed
+// block -- every lane of a row group reads the same element, a shared-memory broadcast)
+template <int SB, int RC, bool TRANS>
+__device__ __forceinline__ void block_fma(const double* Ls, const double* Ys, double (&acc)[SolveCfg<SB, RC>::RPT]) {
+  using C = SolveCfg<SB, RC>;
+  const int col = threadIdx.x % RC, r0 = (threadIdx.x / RC) * C::RPT;
+#pragma unroll 4
+  for (int k = 0; k < SB; ++k) {
+    const double y = Ys[k * RC + col];
+#pragma unroll
+    for (int i = 0; i < C::RPT; ++i) acc[i] = fma(TRANS ? Ls[k * C::P + r0 + i] : Ls[(r0 + i) * C::P + k], y, acc[i]);
+  }
+}
+
+// Per diagonal block b (once per factorization): inv_b = inv(L_bb) -- column j by forward
+// substitution of e_j (thread j) in shared memory -- and the two chain matrices
+// Mf_b = inv_b L_{b,b-1} (forward) and Mb_b = L_{b+1,b} inv_b (backward), all written
+// whole (SB x SB, row-major; zeros above the diagonal of inv_b).  aux = [inv | Mf | Mb],
+// each nblocks x SB x SB.
+template <int SB>
+__global__ void __launch_bounds__(kSolveThreads) k_diag_aux(const double* tiles, int nb, int nblocks, double* aux) {
+  extern __shared__ __align__(16) double sm[];
+  constexpr int P = kInvPitch;
+  double* Ls = sm;
+  double* Zs = sm + SB * P;  // Zs[r][j] = inv_b
+  double* inv = aux;
+  double* Mf = aux + (int64_t)nblocks * SB * SB;
+  double* Mb = Mf + (int64_t)nblocks * SB * SB;
+  for (int b = blockIdx.x; b < nblocks; b += gridDim.x) {
+    __syncthreads();
+    const double* G = lblock(tiles, nb, SB, b, b);
+    for (int e = threadIdx.x; e < SB * SB; e += kSolveThreads)
+      Ls[(e / SB) * P + e % SB] = __ldcg(G + (int64_t)(e / SB) * nb + e % SB);
+    __syncthreads();
+    const int j = threadIdx.x;
+    if (j < SB) {
+      for (int r = 0; r < j; ++r) Zs[r * P + j] = 0.0;
+      Zs[j * P + j] = 1.0 / Ls[j * P + j];
+      for (int r = j + 1; r < SB; ++r) {
+        double s = 0.0;
+        for (int m = j; m < r; ++m) s = fma(Ls[r * P + m], Zs[m * P + j], s);
+        Zs[r * P + j] = -s / Ls[r * P + r];
+      }
+    }
+    __syncthreads();
+    double* out = inv + (int64_t)b * SB * SB;
+    for (int e = threadIdx.x; e < SB * SB; e += kSolveThreads) out[e] = Zs[(e / SB) * P + (e % SB)];
+    // Mf_b = inv_b L_{b,b-1}: Ls <- L_{b,b-1}
+    if (b > 0) {
+      __syncthreads();
+      const double* G1 = lblock(tiles, nb, SB, b, b - 1);
+      for (int e = threadIdx.x; e < SB * SB; e += kSolveThreads)
+        Ls[(e / SB) * P + e % SB] = __ldcg(G1 + (int64_t)(e / SB) * nb + e % SB);
+      __syncthreads();
+      double* o = Mf + (int64_t)b * SB * SB;
+      for (int e = threadIdx.x; e < SB * SB; e += kSolveThreads) {
+        const int r = e / SB, c = e % SB;
+        double s = 0.0;
+        for (int m = 0; m <= r; ++m) s = fma(Zs[r * P + m], Ls[m * P + c], s);
+        o[e] = s;
+      }
+    }
+    // Mb_b = L_{b+1,b} inv_b: Ls <- L_{b+1,b}
+    if (b + 1 < nblocks) {
+      __syncthreads();
+      const double* G2 = lblock(tiles, nb, SB, b + 1, b);
+      for (int e = threadIdx.x; e < SB * SB; e += kSolveThreads)
+        Ls[(e / SB) * P + e % SB] = __ldcg(G2 + (int64_t)(e / SB) * nb + e % SB);
+      __syncthreads();
+      double* o = Mb + (int64_t)b * SB * SB;
+      for (int e = threadIdx.x; e < SB * SB; e += kSolveThreads) {
+        const int r = e / SB, c = e % SB;
+        double s = 0.0;
+        for (int m = c; m < SB; ++m) s = fma(Ls[r * P + m], Zs[m * P + c], s);
+        o[e] = s;
+      }
+    }
+  }
+}
+
+__device__ __forceinline__ void cp_async16(void* dst, const void* src) {
+  asm volatile("cp.async.cg.shared.global [%0], [%1], 16;" ::"r"(smem_u32(dst)), "l"(src) : "memory");
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;" ::: "memory"); }
+template <int N>
+__device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;" ::"n"(N) : "memory"); }
+
+// rows x cols (doubles, cols even) block at G (ld) -> dst (pitch), 16-byte cp.async chunks
+// spread over the CTA: every chunk of the thread in flight at once
+template <int ROWS, int COLS, int PITCH>
+__device__ __forceinline__ void stage_async(double* dst, const double* G, int64_t ld) {
+  constexpr int CH = COLS / 2;
+  for (int e = threadIdx.x; e < ROWS * CH; e += kSolveThreads) {
+    const int r = e / CH, c2 = 2 * (e - r * CH);
+    cp_async16(dst + r * PITCH + c2, G + (int64_t)r * ld + c2);
+  }
+}
+
+// One sweep (forward: FWD = true) over work items (block row b, chunk ch of RC columns):
+//   forward   Y_b = inv_b (B_b - sum_{c<b-1} L_bc Y_c) - Mf_b Y_{b-1}
+//   backward  X_b = inv_b^T (Y_b - sum_{c>b+1} L_cb^T X_c) - Mb_b^T X_{b+1}
+// (Mf_b = inv_b L_{b,b-1}, Mb_b = L_{b+1,b} inv_b, k_diag_aux), so only the last product
+// waits for the previous block row: the chain from block to block is one flag hop, one
+// fetch of the 8- or 32-column block and one SB x SB x RC FMA pass.  Stages: the nc-1
+// older off-diagonal blocks (accumulate), the inverse applied to (rhs - acc), then the
+// chain matrix against the previous block row.  Each stage's SB x SB matrix streams into
+// the other shared buffer (cp.async) while the previous stage computes; the right-hand
+// side block sits in registers from the start of the item.  flags[b * nchunks + ch] =
+// epoch once block b of chunk ch is final in W.
+template <int SB, int RC, bool FWD>
+__global__ void __launch_bounds__(kSolveThreads, 1)
+    k_sweep(const double* tiles, int nb, int nblocks, const double* aux, double* W, int ldw, int nchunks, int* flags,
+            int* counter, int epoch) {
+  using C = SolveCfg<SB, RC>;
+  extern __shared__ __align__(16) double sm[];
+  double* Lb[2] = {sm, sm + SB * C::P};
+  double* Ys = sm + 2 * SB * C::P;
+  int* s_item = reinterpret_cast<int*>(Ys + SB * RC);
+  const int col = threadIdx.x % RC, r0 = (threadIdx.x / RC) * C::RPT;
+  const int total = nblocks * nchunks;
+  const int64_t bsz = (int64_t)SB * SB;
+  const double* inv = aux;
+  const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
+  while (true) {
+    __syncthreads();
+    if (threadIdx.x == 0) *s_item = atomicAdd(counter, 1);
+    __syncthreads();
+    const int item = *s_item;
+    if (item >= total) break;
+    const int ch = item % nchunks;
+    const int b = FWD ? item / nchunks : nblocks - 1 - item / nchunks;
+    const int nc = FWD ? b : nblocks - 1 - b;  // block rows this one depends on
+    const int nold = nc > 0 ? nc - 1 : 0;      // accumulated before the inverse
+    // stage q: q < nold off-diagonal block c(q); q == nold the inverse; q == nold + 1 the chain matrix
+    const int nst = nold + 1 + (nc > 0 ? 1 : 0);
+    auto cof = [&](int q) { return FWD ? q : nblocks - 1 - q; };  // block row consumed by stage q < nold
+    auto stage_L = [&](int q, double* dst) {
+      if (q < nold) {
+        const int c = cof(q);
+        stage_async<SB, SB, C::P>(dst, FWD ? lblock(tiles, nb, SB, b, c) : lblock(tiles, nb, SB, c, b), nb);
+      } else if (q == nold) {
+        stage_async<SB, SB, C::P>(dst, inv + b * bsz, SB);
+      } else {
+        stage_async<SB, SB, C::P>(dst, Mch + b * bsz, SB);
+      }
+      cp_async_commit();
+    };
+    double* Wb = W + (int64_t)b * SB * ldw + ch * RC;
+    double rhs[C::RPT], acc[C::RPT];
+#pragma unroll
+    for (int i = 0; i < C::RPT; ++i) {
+      rhs[i] = __ldcg(Wb + (int64_t)(r0 + i) * ldw + col);
+      acc[i] = 0.0;
+    }
+    stage_L(0, Lb[0]);
+    for (int q = 0; q < nst; ++q) {
+      const int buf = q & 1;
+      if (q != nold) {  // consumes a finished block row: c(q) or the previous row
+        const int c = q < nold ? cof(q) : (FWD ? b - 1 : b + 1);
+        if (threadIdx.x == 0) {
+          const int* f = flags + c * nchunks + ch;
+          int v;
+          do {
+            asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(f) : "memory");
+          } while (v != epoch);
+        }
+        __syncthreads();
+        stage_async<SB, RC, RC>(Ys, W + (int64_t)c * SB * ldw + ch * RC, ldw);
+        cp_async_commit();
+      } else {  // rhs - acc, for the inverse
+#pragma unroll
+        for (int i = 0; i < C::RPT; ++i) {
+          Ys[(r0 + i) * RC + col] = rhs[i] - acc[i];
+          acc[i] = 0.0;
+        }
+        cp_async_commit();  // empty group: keeps the group count uniform
+      }
+      if (q + 1 < nst) {
+        stage_L(q + 1, Lb[buf ^ 1]);  // prefetch the next matrix (its buffer was freed by stage q-1)
+        cp_async_wait<1>();           // everything but that prefetch has landed
+      } else {
+        cp_async_wait<0>();
+      }
+      __syncthreads();
+      if (q == nold + 1) {  // acc = U - M y: negate, accumulate, negate back
+#pragma unroll
+        for (int i = 0; i < C::RPT; ++i) acc[i] = -acc[i];
+        block_fma<SB, RC, !FWD>(Lb[buf], Ys, acc);
+#pragma unroll
+        for (int i = 0; i < C::RPT; ++i) acc[i] = -acc[i];
+      } else {
+        block_fma<SB, RC, !FWD>(Lb[buf], Ys, acc);
+      }
+      __syncthreads();  // Ys and Lb[buf] free
+    }
+#pragma unroll
+    for (int i = 0; i < C::RPT; ++i) __stcg(Wb + (int64_t)(r0 + i) * ldw + col, acc[i]);
+    // the CTA barrier orders every thread's stores before thread 0's release (cumulative),
+    // so one gpu-scope release publishes the whole block
+    __syncthreads();
+    if (threadIdx.x == 0) {
+      int* f = flags + b * nchunks + ch;
+      asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(f), "r"(epoch) : "memory");
+    }
+  }
+}
+
+template <int SB, int RC>
+static cudaError_t solve_sb(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
+  using C = SolveCfg<SB, RC>;
+  const int smem = C::kSmem, smem_inv = 2 * SB * kInvPitch * 8;
+  cudaError_t e;
+  if ((e = cudaFuncSetAttribute(k_diag_aux<SB>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_inv))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep<SB, RC, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep<SB, RC, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  const int nblocks = (int)(a.n / SB);
+  if (!a.inv_valid) {
+    k_diag_aux<SB><<<std::min(nblocks, a.sms), kSolveThreads, smem_inv, s>>>(a.tiles, a.nb, nblocks, a.inv);
+    ++*nlaunch;
+  }
+  int per_sm = 0;
+  if ((e = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sweep<SB, RC, true>, kSolveThreads, smem))) return e;
+  const int total = nblocks * a.nchunks;
+  const int grid = std::min(total, std::max(1, per_sm) * a.sms);
+  if ((e = cudaMemsetAsync(a.ctl, 0, (2 + 2 * (size_t)total) * sizeof(int), s))) return e;
+  int* counters = a.ctl;
+  int* flags = a.ctl + 2;
+  k_sweep<SB, RC, true><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                          flags, counters, 1);
+  k_sweep<SB, RC, false><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                           flags + total, counters + 1, 1);
+  *nlaunch += 2;
+  return cudaGetLastError();
+}
+
+cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
+  const bool narrow = a.rc == 8;
+  switch (a.sb) {
+    case 96: return narrow ? solve_sb<96, 8>(a, s, nlaunch) : solve_sb<96, 32>(a, s, nlaunch);
+    case 64: return narrow ? solve_sb<64, 8>(a, s, nlaunch) : solve_sb<64, 32>(a, s, nlaunch);
+    case 32: return narrow ? solve_sb<32, 8>(a, s, nlaunch) : solve_sb<32, 32>(a, s, nlaunch);
+  }
+  return cudaErrorInvalidValue;
+}
+
+}  // namespace chol

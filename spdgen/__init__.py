@@ -30,7 +30,7 @@ INT_SALT = np.uint64(0xD1B54A32D192ED03)  # separates the integer family's strea
 BW = 3  # bandwidth of L0 in the integer family
 
 __all__ = ["splitmix64", "uniform_spd", "uniform_entries", "integer_L0", "integer_L0_bands", "integer_spd",
-           "make_non_spd", "BW"]
+           "make_non_spd", "BW", "rhs", "integer_rhs_solution"]
 
 
 def splitmix64(x: np.ndarray) -> np.ndarray:
@@ -151,3 +151,26 @@ def make_non_spd(A: np.ndarray, L0: np.ndarray, j0: int, kind: str = "zero") -> 
     d = L0[j0, j0] ** 2 + (1.0 if kind == "neg" else 0.0)
     B[j0, j0] -= d
     return B
+
+
+RHS_SALT = np.uint64(0x5851F42D4C957F2D)
+
+
+def rhs(n: int, nrhs: int, seed: int = 0) -> np.ndarray:
+    """Right-hand sides for the solve: n x nrhs row-major, entries
+    u in [-0.5, 0.5) from splitmix64 of (seed ^ RHS_SALT, row, column)."""
+    i = np.arange(n, dtype=np.uint64)[:, None]
+    j = np.arange(nrhs, dtype=np.uint64)[None, :]
+    with np.errstate(over="ignore"):
+        key = (np.uint64(seed) ^ RHS_SALT) * GOLDEN + i * np.uint64(nrhs) + j
+    return _u01(splitmix64(key)) - 0.5
+
+
+def integer_rhs_solution(n: int, nrhs: int, seed: int = 0) -> np.ndarray:
+    """Small integer solutions X0 in {-2..2} (n x nrhs): with the integer family, B = A X0
+    is an exact integer matrix and the substitutions return X0 exactly."""
+    i = np.arange(n, dtype=np.uint64)[:, None]
+    j = np.arange(nrhs, dtype=np.uint64)[None, :]
+    with np.errstate(over="ignore"):
+        key = (np.uint64(seed) ^ RHS_SALT ^ INT_SALT) * GOLDEN + i * np.uint64(nrhs) + j
+    return ((splitmix64(key) >> np.uint64(61)).astype(np.int64) % 5 - 2).astype(np.float64)
