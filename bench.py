@@ -11,8 +11,11 @@ Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|referenc
        [--n 19200] [--nb 960] [--policy cp|dynamic|static] [--executor sched|host]
        [--logical-ranks R --grid PxQ]
 Under torchrun (N > 1) the N ranks factor ONE matrix together (2D block-cyclic
-owner-computes, panel tiles pulled over NVLink peer memory; strong scaling); rank 0
-prints ONE JSON line.  --logical-ranks R runs the distributed path with R ranks sharing
+owner-computes, panel tiles pulled over NVLink peer memory); rank 0 prints ONE JSON line.
+--scaling weak (default): the matrix order grows with N so that the flops per GPU stay
+fixed, n_N = nb * round(N_1 * N^(1/3)) with N_1 = n / nb tiles at one GPU (n=19200:
+24000, 30720, 38400 at 2, 4, 8 GPUs -- the paper's own axis is the matrix order,
+P:L489); --scaling strong keeps n fixed.  --logical-ranks R runs the distributed path with R ranks sharing
 one GPU (tests the multi-GPU machinery; not a scaling number).
 """
 from __future__ import annotations
@@ -52,6 +55,7 @@ def parse():
     ap.add_argument("--cpu-sample-n", type=int, default=7680)
     ap.add_argument("--grid", default="", help="process grid PxQ (default 1xN; SURVEY §8e prefers p <= q)")
     ap.add_argument("--logical-ranks", type=int, default=0)
+    ap.add_argument("--scaling", choices=["weak", "strong"], default="weak")
     return ap.parse_args()
 
 
@@ -140,6 +144,13 @@ def allmax(ws, x: float) -> float:
     return float(t.item())
 
 
+def workload_n(args, ws: int) -> int:
+    """Matrix order at ws GPUs: fixed (strong) or with fixed flops per GPU (weak)."""
+    if ws <= 1 or args.scaling == "strong":
+        return args.n
+    return args.nb * max(1, round(args.n / args.nb * ws ** (1.0 / 3.0)))
+
+
 # ----------------------------------------------------------------------------- reference arm
 def run_reference(args, ws, rank):
     """The oracle (oracle/chol_oracle.c, plain C + OpenMP, no BLAS) as it stands, on the
@@ -148,7 +159,8 @@ def run_reference(args, ws, rank):
         return
     import oracle
     import spdgen
-    n_s = min(args.n, 3840)
+    n_w = workload_n(args, ws)
+    n_s = min(n_w, 3840)
     A = spdgen.uniform_spd(n_s, args.seed)
     times = []
     for it in range(args.warmup + args.steps):
@@ -165,8 +177,8 @@ def run_reference(args, ws, rank):
     line = {
         "impl": "reference", "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * tot / len(times),
-        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-        "config": {"workload": f"FP64 SPD n={args.n} nb={args.nb} (bounded sample: {sample})", "n": args.n,
+        "higher_is_better": True, "scaling": args.scaling, "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": {"workload": f"FP64 SPD n={n_w} nb={args.nb} (bounded sample: {sample})", "n": n_w,
                    "nb": args.nb},
         "cpu_baseline": {"value": value, "unit": "TFLOP/s", "cores": cores, "kind": "oracle", "sample": sample},
         "e2e": {"value": value, "unit": "TFLOP/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
@@ -239,12 +251,12 @@ def grid_of(args, R):
 
 
 def run_dist(args, ws, rank, local):
-    """Multi-GPU strong scaling: one factorization of A (n x n) on ws ranks."""
+    """Multi-GPU: one factorization of A (n x n, n = workload_n) on ws ranks."""
     import torch
     import torch.distributed as dist
     import paper_conf_ipps_agullobehkmt15_b200 as c
 
-    n, nb = args.n, args.nb
+    n, nb = workload_n(args, ws), args.nb
     flops = n ** 3 / 3.0
     p, q = grid_of(args, ws)
 
@@ -277,9 +289,10 @@ def run_dist(args, ws, rank, local):
     value = flops / t_step / 1e12
     line = {
         "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": ws, "steps": args.steps,
-        "warmup": args.warmup, "ms_per_step": 1e3 * t_step, "higher_is_better": True, "scaling": "strong",
+        "warmup": args.warmup, "ms_per_step": 1e3 * t_step, "higher_is_better": True, "scaling": args.scaling,
         "vs_baseline": None, "dtype": "f64", "data": "synthetic",
         "config": {"workload": f"FP64 SPD n={n} as {n // nb}x{n // nb} tiles of nb={nb}", "n": n, "nb": nb,
+                   "gflop_per_gpu": flops / ws / 1e9,
                    "parallelism": f"2D block-cyclic {p}x{q}, owner-computes, NVLink peer pulls of panel tiles",
                    "policy": args.policy, "tiles_owned_rank0": d["nowned"],
                    "tiles_cached_rank0": d["nslots"] - d["nowned"],
