@@ -651,9 +651,14 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // 28 nodes per POTRF instead of 220).  The block DAG shortens the POTRF chain
   // (785 -> 633 us alone, n=9600 15.1 -> 13.3 ms) but its extra nodes cost dispatch
   // work: 0.3 ms at n=19200, where the area bound dominates (chain/area ~ 141/N^2 at
-  // nb=960).  Default: block DAG while N <= 16.  CHOL_POTRF_BLOCKDAG=0/1 overrides.
+  // nb=960).  Default: block DAG while N <= 16, i.e. N^2 <= 256 tiles per GPU -- a rank
+  // of an R-GPU plan holds ~N^2/R of the area but the whole chain, so the same rule
+  // reads N^2 / R <= 256 there.  CHOL_POTRF_BLOCKDAG=0/1 overrides.
   const char* epb = getenv("CHOL_POTRF_BLOCKDAG");
-  const bool potrf_blockdag = epb ? atoi(epb) != 0 : N <= 16;
+  const int64_t ranks = dist ? std::max(1, dist->nranks) : 1;
+  const bool potrf_blockdag = epb ? atoi(epb) != 0 : N * N <= 256 * ranks;
+  const char* ep0 = getenv("CHOL_POTRF0_BLOCKDAG");
+  const bool potrf0_blockdag = !(ep0 && atoi(ep0) == 0);
   // Hybrid DAG: the steps k >= k0 are built at BS-block granularity across tasks (the
   // paper's tasks keep their kernels, but a consumer block waits only for the producer
   // blocks it reads): POTRF as its block DAG, TRSM as per-slab chains (TS/TU), SYRK and
@@ -698,7 +703,10 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   for (int k = 0; k < N; ++k) {
     const int pid = (int)id_potrf(N, k);
     const bool blk = k >= k0;
-    if (mine(k, k) && !potrf_blockdag && !blk) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
+    // POTRF_0 runs alone on an idle GPU (every other task depends on it): always the
+    // shorter block DAG (CHOL_POTRF0_BLOCKDAG=0 turns this off; development switch)
+    const bool pblock = potrf_blockdag || (k == 0 && potrf0_blockdag);
+    if (mine(k, k) && !pblock && !blk) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
       int prev = -1;
       for (int b = 0; b < nbb; ++b) {
         const int dn = B.add_node(pid, T_POTRF, k, k);
@@ -882,6 +890,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         }
       tfin[sid] = tentry[sid];
       if (k == 0) gate_of(sid, T_SYRK, j, k);
+
       for (int i = j + 1; i < N; ++i) {
         const int gid = (int)id_gemm(N, i, j, k);
         tentry[gid].assign(nbb2, -1);
