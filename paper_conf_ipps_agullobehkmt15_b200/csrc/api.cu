@@ -767,7 +767,9 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   if (!p->factored || p->last_info != 0) return -10;
   cudaSetDevice(p->device);
   const int64_t n = p->n;
-  const int rc = nrhs <= 8 ? 8 : 32;  // columns per work item (lanes of a row group)
+  // columns per work item: 1 (register-streamed matrix-vector sweeps), 8 or 32 (lanes of
+  // a row group, shared-memory staged blocks)
+  const int rc = nrhs == 1 ? 1 : nrhs <= 8 ? 8 : 32;
   const int nchunks = (int)((nrhs + rc - 1) / rc), ldw = rc * nchunks;
   const int64_t nblocks = n / p->bs;
   const size_t need = (size_t)n * ldw, ctl = 2 + 2 * (size_t)nblocks * nchunks;
@@ -811,10 +813,24 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   a.rc = rc;
   a.ctl = p->d_solve_ctl;
   a.sms = p->sms;
+  // development: CHOL_SOLVE_TRACE=<file> writes per-item sweep timestamps (solve.cu)
+  const char* trace_path = getenv("CHOL_SOLVE_TRACE");
+  const size_t ntr = 2 * (size_t)nblocks * nchunks * 6;
+  if (trace_path) CUDA_TRY(cudaMalloc(&a.trace, ntr * sizeof(uint64_t)));
   int nl = 0;
   CUDA_TRY(cudaEventRecord(p->ev4, p->stream));
   CUDA_TRY(solve_run(a, p->stream, &nl));
   CUDA_TRY(cudaEventRecord(p->ev5, p->stream));
+  if (trace_path) {
+    std::vector<uint64_t> h(ntr);
+    CUDA_TRY(cudaMemcpyAsync(h.data(), a.trace, ntr * sizeof(uint64_t), cudaMemcpyDeviceToHost, p->stream));
+    CUDA_TRY(cudaStreamSynchronize(p->stream));
+    cudaFree(a.trace);
+    if (FILE* f = fopen(trace_path, "wb")) {
+      fwrite(h.data(), sizeof(uint64_t), ntr, f);
+      fclose(f);
+    }
+  }
   p->inv_valid = true;
   CUDA_TRY(cudaMemcpy2DAsync(B, ldb * 8, p->d_rhs, ldw * 8, nrhs * 8, n, cudaMemcpyDefault, p->stream));
   CUDA_TRY(cudaEventRecord(p->ev3, p->stream));

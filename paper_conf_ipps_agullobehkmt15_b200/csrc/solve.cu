@@ -160,7 +160,7 @@ __device__ __forceinline__ void stage_async(double* dst, const double* G, int64_
 template <int SB, int RC, bool FWD>
 __global__ void __launch_bounds__(kSolveThreads, 1)
     k_sweep(const double* tiles, int nb, int nblocks, const double* aux, double* W, int ldw, int nchunks, int* flags,
-            int* counter, int epoch) {
+            int* counter, int epoch, uint64_t* trace) {
   using C = SolveCfg<SB, RC>;
   extern __shared__ __align__(16) double sm[];
   double* Lb[2] = {sm, sm + SB * C::P};
@@ -177,6 +177,8 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
     __syncthreads();
     const int item = *s_item;
     if (item >= total) break;
+    uint64_t tr_claim = 0, tr_wait = 0, tr_chain0 = 0, tr_chain1 = 0;
+    if (trace && threadIdx.x == 0) tr_claim = globaltimer_ns();
     const int ch = item % nchunks;
     const int b = FWD ? item / nchunks : nblocks - 1 - item / nchunks;
     const int nc = FWD ? b : nblocks - 1 - b;  // block rows this one depends on
@@ -209,10 +211,16 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
         const int c = q < nold ? cof(q) : (FWD ? b - 1 : b + 1);
         if (threadIdx.x == 0) {
           const int* f = flags + c * nchunks + ch;
+          const uint64_t tw0 = trace ? globaltimer_ns() : 0;
           int v;
           do {
             asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(f) : "memory");
           } while (v != epoch);
+          if (trace) {
+            const uint64_t tw1 = globaltimer_ns();
+            if (q == nold + 1) tr_chain0 = tw0, tr_chain1 = tw1;
+            else tr_wait += tw1 - tw0;
+          }
         }
         __syncthreads();
         stage_async<SB, RC, RC>(Ys, W + (int64_t)c * SB * ldw + ch * RC, ldw);
@@ -251,8 +259,207 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
     if (threadIdx.x == 0) {
       int* f = flags + b * nchunks + ch;
       asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(f), "r"(epoch) : "memory");
+      if (trace) {
+        uint64_t* t = trace + 6 * (int64_t)(item + (FWD ? 0 : total));
+        unsigned smid;
+        asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+        t[0] = tr_claim;
+        t[1] = tr_chain0;
+        t[2] = tr_chain1;
+        t[3] = globaltimer_ns();
+        t[4] = tr_wait;
+        t[5] = ((uint64_t)b << 32) | smid;
+      }
     }
   }
+}
+
+// Single right-hand side (nrhs = 1): register-streamed matrix-vector sweeps, same items,
+// flags and recurrences as k_sweep.  Warp w owns rows [w*RPW, (w+1)*RPW) of every SB x SB
+// matrix it streams and lane l the columns l, l+32, ... (KPL = SB/32), so each warp-load
+// is 256 contiguous bytes.  A matrix element is used once, so it is loaded straight into
+// registers (no shared-memory staging -- staging 73 KB per stage through cp.async or
+// per-row bulk copies capped a CTA at ~17 GB/s, tools/solve_trace.py), the next stage's
+// matrix while the current one is multiplied; each warp walks the stages on its own
+// (its lane 0 acquires the flag of the block row consumed), so CTA barriers only frame
+// the two reductions of an item.
+//   FWD, non-transposed: partial p[i] (warp row i) over the lane's columns, reduced
+//       across lanes;
+//   BWD, transposed (L_cb^T, inv_b^T, Mb_b^T read from the stored blocks): partial p[j]
+//       (column l + 32 j) over the warp's rows, reduced across warps.
+template <int SB, bool FWD>
+__global__ void __launch_bounds__(kSolveThreads, 1)
+    k_sweep_vec(const double* tiles, int nb, int nblocks, const double* aux, double* W, int* flags, int* counter,
+                int epoch, uint64_t* trace) {
+  constexpr int RPW = SB / 8, KPL = SB / 32, NP = FWD ? RPW : KPL, RP = 33;
+  __shared__ double red[FWD ? SB * RP : 8 * SB];
+  __shared__ double xs[SB];
+  __shared__ int s_item;
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, t = threadIdx.x;
+  const int64_t bsz = (int64_t)SB * SB;
+  const double* inv = aux;
+  const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
+  double R0[RPW][KPL], R1[RPW][KPL], p[NP];
+  auto load = [&](double (&R)[RPW][KPL], const double* G, int64_t ld) {
+#pragma unroll
+    for (int i = 0; i < RPW; ++i)
+#pragma unroll
+      for (int j = 0; j < KPL; ++j) R[i][j] = __ldcs(G + (int64_t)(warp * RPW + i) * ld + lane + 32 * j);
+  };
+  // p (+)= sign * Op(R) x with x = block row c of W (c >= 0, after its flag) or xs (c < 0)
+  auto apply = [&](const double (&R)[RPW][KPL], int c, double sign) {
+    const double* xv = xs;
+    if (c >= 0) {
+      if (lane == 0) {
+        const int* f = flags + c;
+        int v;
+        do {
+          asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(f) : "memory");
+        } while (v != epoch);
+      }
+      __syncwarp();
+      xv = W + (int64_t)c * SB;
+    }
+    if (FWD) {
+      double x[KPL];
+#pragma unroll
+      for (int j = 0; j < KPL; ++j) x[j] = sign * (c >= 0 ? __ldcg(xv + lane + 32 * j) : xv[lane + 32 * j]);
+#pragma unroll
+      for (int i = 0; i < RPW; ++i)
+#pragma unroll
+        for (int j = 0; j < KPL; ++j) p[i] = fma(R[i][j], x[j], p[i]);
+    } else {
+      double x[RPW];
+#pragma unroll
+      for (int i = 0; i < RPW; ++i) x[i] = sign * (c >= 0 ? __ldcg(xv + warp * RPW + i) : xv[warp * RPW + i]);
+#pragma unroll
+      for (int i = 0; i < RPW; ++i)
+#pragma unroll
+        for (int j = 0; j < KPL; ++j) p[j] = fma(R[i][j], x[i], p[j]);
+    }
+  };
+  // CTA reduction of the partials: returns the full sum for row/column t (t < SB)
+  auto reduce = [&]() -> double {
+    if (FWD) {
+#pragma unroll
+      for (int i = 0; i < RPW; ++i) red[(warp * RPW + i) * RP + lane] = p[i];
+    } else {
+#pragma unroll
+      for (int j = 0; j < KPL; ++j) red[warp * SB + lane + 32 * j] = p[j];
+    }
+    __syncthreads();
+    double s = 0.0;
+    if (t < SB) {
+      if (FWD) {
+        double s2 = 0.0;
+#pragma unroll
+        for (int l = 0; l < 32; l += 2) {
+          s += red[t * RP + l];
+          s2 += red[t * RP + l + 1];
+        }
+        s += s2;
+      } else {
+#pragma unroll
+        for (int w = 0; w < 8; ++w) s += red[w * SB + t];
+      }
+    }
+    return s;
+  };
+  while (true) {
+    __syncthreads();
+    if (t == 0) s_item = atomicAdd(counter, 1);
+    __syncthreads();
+    const int item = s_item;
+    if (item >= nblocks) break;
+    uint64_t tr_claim = 0, tr_chain0 = 0, tr_chain1 = 0;
+    if (trace && t == 0) tr_claim = globaltimer_ns();
+    const int b = FWD ? item : nblocks - 1 - item;
+    const int nc = FWD ? b : nblocks - 1 - b;
+    const int nold = nc > 0 ? nc - 1 : 0;
+    const int nst = nold + 1 + (nc > 0 ? 1 : 0);
+    auto mat = [&](int q, const double*& G, int64_t& ld) {
+      if (q < nold) {
+        const int c = FWD ? q : nblocks - 1 - q;
+        G = FWD ? lblock(tiles, nb, SB, b, c) : lblock(tiles, nb, SB, c, b);
+        ld = nb;
+      } else {
+        G = (q == nold ? inv : Mch) + b * bsz;
+        ld = SB;
+      }
+    };
+    const double rhs = t < SB ? __ldcg(W + (int64_t)b * SB + t) : 0.0;
+#pragma unroll
+    for (int i = 0; i < NP; ++i) p[i] = 0.0;
+    const double* G;
+    int64_t ld;
+    mat(0, G, ld);
+    load(R0, G, ld);
+    for (int q = 0; q < nst; q += 2) {
+      // stage q in R0 (next into R1), stage q+1 in R1 (next into R0)
+#pragma unroll
+      for (int h = 0; h < 2; ++h) {
+        const int qq = q + h;
+        if (qq >= nst) break;
+        double (&Rc)[RPW][KPL] = h ? R1 : R0;
+        double (&Rn)[RPW][KPL] = h ? R0 : R1;
+        if (qq + 1 < nst) {
+          mat(qq + 1, G, ld);
+          load(Rn, G, ld);
+        }
+        if (qq < nold) {
+          apply(Rc, FWD ? qq : nblocks - 1 - qq, 1.0);
+        } else if (qq == nold) {  // xs = rhs - acc, then p = Op(inv_b) xs
+          const double s = nold > 0 ? reduce() : 0.0;
+          if (t < SB) xs[t] = rhs - s;
+          __syncthreads();
+#pragma unroll
+          for (int i = 0; i < NP; ++i) p[i] = 0.0;
+          apply(Rc, -1, 1.0);
+        } else {  // chain: p -= Op(M_b) x_{b -+ 1}
+          if (trace && t == 0) tr_chain0 = globaltimer_ns();
+          apply(Rc, FWD ? b - 1 : b + 1, -1.0);
+          if (trace && t == 0) tr_chain1 = globaltimer_ns();
+        }
+      }
+    }
+    const double y = reduce();
+    if (t < SB) __stcg(W + (int64_t)b * SB + t, y);
+    __syncthreads();  // every store before the release (cumulative)
+    if (t == 0) {
+      asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(flags + b), "r"(epoch) : "memory");
+      if (trace) {
+        uint64_t* tt = trace + 6 * (int64_t)(item + (FWD ? 0 : nblocks));
+        unsigned smid;
+        asm volatile("mov.u32 %0, %%smid;" : "=r"(smid));
+        tt[0] = tr_claim;
+        tt[1] = tr_chain0;
+        tt[2] = tr_chain1;
+        tt[3] = globaltimer_ns();
+        tt[4] = 0;
+        tt[5] = ((uint64_t)b << 32) | smid;
+      }
+    }
+  }
+}
+
+template <int SB>
+static cudaError_t solve_vec(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
+  const int smem_inv = 2 * SB * kInvPitch * 8;
+  cudaError_t e;
+  if ((e = cudaFuncSetAttribute(k_diag_aux<SB>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_inv))) return e;
+  const int nblocks = (int)(a.n / SB);
+  if (!a.inv_valid) {
+    k_diag_aux<SB><<<std::min(nblocks, a.sms), kSolveThreads, smem_inv, s>>>(a.tiles, a.nb, nblocks, a.inv);
+    ++*nlaunch;
+  }
+  const int grid = std::min(nblocks, a.sms);
+  if ((e = cudaMemsetAsync(a.ctl, 0, (2 + 2 * (size_t)nblocks) * sizeof(int), s))) return e;
+  k_sweep_vec<SB, true><<<grid, kSolveThreads, 0, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ctl + 2, a.ctl, 1,
+                                                        a.trace);
+  k_sweep_vec<SB, false><<<grid, kSolveThreads, 0, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ctl + 2 + nblocks,
+                                                         a.ctl + 1, 1, a.trace);
+  *nlaunch += 2;
+  return cudaGetLastError();
 }
 
 template <int SB, int RC>
@@ -276,14 +483,22 @@ static cudaError_t solve_sb(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   int* counters = a.ctl;
   int* flags = a.ctl + 2;
   k_sweep<SB, RC, true><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
-                                                          flags, counters, 1);
+                                                          flags, counters, 1, a.trace);
   k_sweep<SB, RC, false><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
-                                                           flags + total, counters + 1, 1);
+                                                           flags + total, counters + 1, 1, a.trace);
   *nlaunch += 2;
   return cudaGetLastError();
 }
 
 cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
+  if (a.rc == 1) {
+    switch (a.sb) {
+      case 96: return solve_vec<96>(a, s, nlaunch);
+      case 64: return solve_vec<64>(a, s, nlaunch);
+      case 32: return solve_vec<32>(a, s, nlaunch);
+    }
+    return cudaErrorInvalidValue;
+  }
   const bool narrow = a.rc == 8;
   switch (a.sb) {
     case 96: return narrow ? solve_sb<96, 8>(a, s, nlaunch) : solve_sb<96, 32>(a, s, nlaunch);

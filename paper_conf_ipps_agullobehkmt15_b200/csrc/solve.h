@@ -15,9 +15,10 @@ struct SolveArgs {
   bool inv_valid;       // inverses already computed for this factor
   double* W;            // right-hand sides, n x ldw row-major, overwritten by the solution
   int ldw, nchunks;     // ldw = rc * nchunks
-  int rc;               // right-hand-side columns per work item: 8 (nrhs <= 8) or 32
+  int rc;               // right-hand-side columns per work item: 1 (nrhs = 1), 8 (nrhs <= 8) or 32
   int* ctl;             // 2 + 2 * (n / sb) * nchunks ints of control (counters, flags)
   int sms;
+  uint64_t* trace;      // development: 2 * (n / sb) * nchunks items x 6 u64 (solve.cu), or null
 };
 cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch);
 }  // namespace chol

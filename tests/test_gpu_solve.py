@@ -56,7 +56,7 @@ def test_solve_matches_oracle(n, nb, nrhs):
         assert np.array_equal(dB.cpu().numpy(), X)
 
 
-@pytest.mark.parametrize("nrhs", [32, 70])
+@pytest.mark.parametrize("nrhs", [1, 32, 70])
 def test_solve_padded_ldb_and_repeat(nrhs):
     c = _lib()
     n, nb = 1920, 960
