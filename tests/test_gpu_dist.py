@@ -95,3 +95,50 @@ def test_two_processes_share_gpu_through_ipc():
                        capture_output=True, text=True, timeout=240)
     assert r.returncode == 0, r.stderr[-2000:]
     assert "'infos': [0, 0], 'exact': True" in r.stdout, r.stdout
+
+
+def _run_logical_device(n, nb, p, q, seed, family, policy=1):
+    """run_logical without the host copy: the gathered factor stays on the device."""
+    c = _lib()
+    R = p * q
+    sms = torch.cuda.get_device_properties(0).multi_processor_count
+    plans = [c.DistPlan(n, nb, R, r, grid_p=p, grid_q=q, workers=sms // R, policy=policy) for r in range(R)]
+    c.DistPlan.connect_local(plans)
+    for pl in plans:
+        c.chol_generate(pl.h, seed, family)
+    for pl in plans:
+        c.chol_factor_async(pl.h)
+    infos = [c.chol_wait(pl.h) for pl in plans]
+    out = torch.zeros((n, n), dtype=torch.float64, device="cuda")
+    for pl in plans:
+        c.chol_gather(pl.h, out, n)
+    torch.cuda.synchronize()
+    for pl in plans:
+        pl.close()
+    return out, infos
+
+
+@pytest.mark.parametrize("n,p,q", [(24000, 1, 2), (30720, 2, 2), (38400, 2, 4)])
+def test_dist_bench_sizes_bitwise_equal_single_gpu(n, p, q):
+    """The bench's multi-GPU workloads (weak scaling: n = 24000 / 30720 / 38400 on 1x2 /
+    2x2 / 2x4, nb = 960) as logical ranks: the distributed factor equals the single-plan
+    factor bit for bit (R15), and for the integer family it is L0 exactly (band check)."""
+    c = _lib()
+    nb, seed = 960, 21
+    Ld, infos = _run_logical_device(n, nb, p, q, seed, 1)
+    assert not any(infos), infos
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as pl:
+        c.chol_generate(pl.h, seed, 1)
+        assert c.chol_factor_inplace(pl.h) == 0
+        Ls = torch.empty((n, n), dtype=torch.float64, device="cuda")
+        c.chol_gather(pl.h, Ls, n)
+        torch.cuda.synchronize()
+    assert torch.equal(Ld, Ls)
+    del Ls
+    Lb = torch.from_numpy(spdgen.integer_L0_bands(n, seed).astype(np.float64)).cuda()
+    idx = torch.arange(n, device="cuda")
+    nnz_band = 0
+    for o in range(spdgen.BW + 1):
+        assert torch.equal(Ld[idx[o:], idx[o:] - o], Lb[o, o:]), o
+        nnz_band += int(torch.count_nonzero(Lb[o, o:]))
+    assert int(torch.count_nonzero(Ld)) == nnz_band  # nothing outside the band
