@@ -423,7 +423,7 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     (void)owner;
     recv_slab(c, d, i, j, sl, owner);
   } else if (type == J_DIAG) {
-    sub_potrf_diag(c, d1.x, d1.y, info);
+    sub_potrf_diag(c, d1.x, d1.y, info, d1.z != 0);
   } else if (type == J_PANEL) {
     sub_potrf_panel(c, d1.x, d1.y, d1.z);
   }
@@ -657,6 +657,10 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   const char* epb = getenv("CHOL_POTRF_BLOCKDAG");
   const int64_t ranks = dist ? std::max(1, dist->nranks) : 1;
   const bool potrf_blockdag = epb ? atoi(epb) != 0 : N * N <= 256 * ranks;
+  // POTRF block DAG: the diagonal block's last update fused into its potf2 job
+  // (CHOL_POTRF_FUSE=0 turns it off; development switch)
+  const char* epf = getenv("CHOL_POTRF_FUSE");
+  const bool potrf_fuse = !(epf && atoi(epf) == 0);
   const char* ep0 = getenv("CHOL_POTRF0_BLOCKDAG");
   const bool potrf0_blockdag = !(ep0 && atoi(ep0) == 0);
   // Hybrid DAG: the steps k >= k0 are built at BS-block granularity across tasks (the
@@ -735,12 +739,16 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       // (q,b).  One job per node, so the chain D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1)
       // never waits for a whole column or trailing update of the step.  D(nbb-1) is the
       // sink (every inner node is its ancestor).
-      std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1);
+      // With potrf_fuse the chain's last update U(b,b,b-1) is done by D(b) itself (one job
+      // and one hop less per inner step, same bits: potf2_block).
+      std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1), fusedP(nbb, -1);
       if (blk) tentry[pid].assign(nbb2, -1), tfin[pid].assign(nbb2, -1);
       for (int b = 0; b < nbb; ++b) {
         const int dn = B.add_node(pid, T_POTRF, k, k);
-        B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+        B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)(fusedP[b] >= 0), 0, 0});
         if (lastU[b * nbb + b] >= 0) B.edge(lastU[b * nbb + b], dn);
+        if (fusedP[b] >= 0) B.edge(fusedP[b], dn);
+        if (blk && b == 1 && fusedP[b] >= 0) tentry[pid][b * nbb + b] = dn;  // first touch of block (1,1)
         if (b == 0) first_node[pid] = dn;
         last_node[pid] = dn;
         for (int r = b + 1; r < nbb; ++r) {
@@ -752,6 +760,10 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         }
         for (int r = b + 1; r < nbb; ++r)
           for (int q = b + 1; q <= r; ++q) {
+            if (potrf_fuse && r == b + 1 && q == r) {  // U(b+1,b+1,b): fused into D(b+1)
+              fusedP[r] = pan[r];
+              continue;
+            }
             const int un = B.add_node(pid, T_POTRF, k, k);
             B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
             B.edge(pan[r], un);
