@@ -767,9 +767,10 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   if (!p->factored || p->last_info != 0) return -10;
   cudaSetDevice(p->device);
   const int64_t n = p->n;
-  // columns per work item: 1 (register-streamed matrix-vector sweeps), 8 or 32 (lanes of
-  // a row group, shared-memory staged blocks)
-  const int rc = nrhs == 1 ? 1 : nrhs <= 8 ? 8 : 32;
+  // columns per work item: 1 (register-streamed matrix-vector sweeps), 32 (DMMA sweeps
+  // at block 96 -- also for 2..8 columns: one padded 32-column chunk beats the 8-column
+  // SIMT item), 8 or 32 (SIMT sweeps at blocks 64 / 32)
+  const int rc = nrhs == 1 ? 1 : (nrhs <= 8 && p->bs != 96) ? 8 : 32;
   const int nchunks = (int)((nrhs + rc - 1) / rc), ldw = rc * nchunks;
   const int64_t nblocks = n / p->bs;
   const size_t need = (size_t)n * ldw, ctl = 2 + 2 * (size_t)nblocks * nchunks;

@@ -21,6 +21,8 @@
 #include <cuda_runtime.h>
 #include <stdint.h>
 
+#include <cstdlib>
+
 #include "dev_common.cuh"
 #include "solve.h"
 #include "taskid.h"
@@ -462,6 +464,168 @@ static cudaError_t solve_vec(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   return cudaGetLastError();
 }
 
+// 32-column chunks on the FP64 tensor path: k_sweep's items, stages, flags and
+// recurrences, with each SB x SB x 32 block product on DMMA (m8n8k4) instead of SIMT FMA
+// (the SIMT pass re-reads one shared-memory element per FMA and tops out near 7 TF/s).
+// Warp w owns the 8 x 8 output blocks (R, C), R = 3 (w % 4) + {0,1,2}, C = 2 (w / 4) +
+// {0,1} of the SB = 96 row x 32 column item; thread (g, t) holds elements (8R + g, 8C + 2t,
+// +1) -- the accumulator layout of every DMMA.  The matrix is staged with pitch 100 and
+// the right-hand-side block with pitch 36, so every fragment load of a half-warp hits 16
+// distinct banks (forward: A[g][t] = L[8R+g][k+t]; backward, transposed: L[k+t][8R+g];
+// B[t][g] = Y[k+t][8C+g]).
+template <bool FWD>
+__global__ void __launch_bounds__(kSolveThreads, 1)
+    k_sweep_mma(const double* tiles, int nb, int nblocks, const double* aux, double* W, int ldw, int nchunks,
+                int* flags, int* counter, int epoch) {
+  constexpr int SB = 96, RC = 32, LP = 100, YP = 36;
+  extern __shared__ __align__(16) double sm[];
+  double* Lb[2] = {sm, sm + SB * LP};
+  double* Ys = sm + 2 * SB * LP;
+  int* s_item = reinterpret_cast<int*>(Ys + SB * YP);
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, g = lane >> 2, t = lane & 3;
+  const int R0 = 3 * (warp & 3), C0 = 2 * (warp >> 2);
+  const int total = nblocks * nchunks;
+  const int64_t bsz = (int64_t)SB * SB;
+  const double* inv = aux;
+  const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
+  // acc (+)= Op(Ls) Ys over k = 0..SB-1
+  auto block_mma = [&](const double* Ls, double (&acc)[3][2][2]) {
+#pragma unroll 4
+    for (int k0 = 0; k0 < SB; k0 += 4) {
+      double a[3], bv[2];
+#pragma unroll
+      for (int mi = 0; mi < 3; ++mi)
+        a[mi] = FWD ? Ls[(8 * (R0 + mi) + g) * LP + k0 + t] : Ls[(k0 + t) * LP + 8 * (R0 + mi) + g];
+#pragma unroll
+      for (int ni = 0; ni < 2; ++ni) bv[ni] = Ys[(k0 + t) * YP + 8 * (C0 + ni) + g];
+#pragma unroll
+      for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+        for (int ni = 0; ni < 2; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a[mi], bv[ni]);
+    }
+  };
+  while (true) {
+    __syncthreads();
+    if (threadIdx.x == 0) *s_item = atomicAdd(counter, 1);
+    __syncthreads();
+    const int item = *s_item;
+    if (item >= total) break;
+    const int ch = item % nchunks;
+    const int b = FWD ? item / nchunks : nblocks - 1 - item / nchunks;
+    const int nc = FWD ? b : nblocks - 1 - b;
+    const int nold = nc > 0 ? nc - 1 : 0;
+    const int nst = nold + 1 + (nc > 0 ? 1 : 0);
+    auto cof = [&](int q) { return FWD ? q : nblocks - 1 - q; };
+    auto stage_L = [&](int q, double* dst) {
+      if (q < nold) {
+        const int c = cof(q);
+        stage_async<SB, SB, LP>(dst, FWD ? lblock(tiles, nb, SB, b, c) : lblock(tiles, nb, SB, c, b), nb);
+      } else if (q == nold) {
+        stage_async<SB, SB, LP>(dst, inv + b * bsz, SB);
+      } else {
+        stage_async<SB, SB, LP>(dst, Mch + b * bsz, SB);
+      }
+      cp_async_commit();
+    };
+    double* Wb = W + (int64_t)b * SB * ldw + ch * RC;
+    double rhs[3][2][2], acc[3][2][2];
+#pragma unroll
+    for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < 2; ++ni) {
+        const double2 v = __ldcg(reinterpret_cast<const double2*>(Wb + (int64_t)(8 * (R0 + mi) + g) * ldw +
+                                                                  8 * (C0 + ni) + 2 * t));
+        rhs[mi][ni][0] = v.x;
+        rhs[mi][ni][1] = v.y;
+        acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
+      }
+    stage_L(0, Lb[0]);
+    for (int q = 0; q < nst; ++q) {
+      const int buf = q & 1;
+      if (q != nold) {
+        const int c = q < nold ? cof(q) : (FWD ? b - 1 : b + 1);
+        if (threadIdx.x == 0) {
+          const int* f = flags + c * nchunks + ch;
+          int v;
+          do {
+            asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(f) : "memory");
+          } while (v != epoch);
+        }
+        __syncthreads();
+        stage_async<SB, RC, YP>(Ys, W + (int64_t)c * SB * ldw + ch * RC, ldw);
+        cp_async_commit();
+      } else {  // Ys = rhs - acc, for the inverse; acc restarts
+#pragma unroll
+        for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+          for (int ni = 0; ni < 2; ++ni) {
+            *reinterpret_cast<double2*>(Ys + (8 * (R0 + mi) + g) * YP + 8 * (C0 + ni) + 2 * t) =
+                make_double2(rhs[mi][ni][0] - acc[mi][ni][0], rhs[mi][ni][1] - acc[mi][ni][1]);
+            acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
+          }
+        cp_async_commit();
+      }
+      if (q + 1 < nst) {
+        stage_L(q + 1, Lb[buf ^ 1]);
+        cp_async_wait<1>();
+      } else {
+        cp_async_wait<0>();
+      }
+      __syncthreads();
+      if (q == nold + 1) {  // acc = U - M y
+        double m[3][2][2];
+#pragma unroll
+        for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+          for (int ni = 0; ni < 2; ++ni) m[mi][ni][0] = m[mi][ni][1] = 0.0;
+        block_mma(Lb[buf], m);
+#pragma unroll
+        for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+          for (int ni = 0; ni < 2; ++ni) {
+            acc[mi][ni][0] -= m[mi][ni][0];
+            acc[mi][ni][1] -= m[mi][ni][1];
+          }
+      } else {
+        block_mma(Lb[buf], acc);
+      }
+      __syncthreads();
+    }
+#pragma unroll
+    for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < 2; ++ni)
+        __stcg(reinterpret_cast<double2*>(Wb + (int64_t)(8 * (R0 + mi) + g) * ldw + 8 * (C0 + ni) + 2 * t),
+               make_double2(acc[mi][ni][0], acc[mi][ni][1]));
+    __syncthreads();
+    if (threadIdx.x == 0)
+      asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(flags + b * nchunks + ch), "r"(epoch) : "memory");
+  }
+}
+
+static cudaError_t solve_mma(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
+  constexpr int SB = 96;
+  const int smem = (2 * SB * 100 + SB * 36) * 8 + 16, smem_inv = 2 * SB * kInvPitch * 8;
+  cudaError_t e;
+  if ((e = cudaFuncSetAttribute(k_diag_aux<SB>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_inv))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep_mma<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep_mma<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  const int nblocks = (int)(a.n / SB);
+  if (!a.inv_valid) {
+    k_diag_aux<SB><<<std::min(nblocks, a.sms), kSolveThreads, smem_inv, s>>>(a.tiles, a.nb, nblocks, a.inv);
+    ++*nlaunch;
+  }
+  const int total = nblocks * a.nchunks;
+  const int grid = std::min(total, a.sms);
+  if ((e = cudaMemsetAsync(a.ctl, 0, (2 + 2 * (size_t)total) * sizeof(int), s))) return e;
+  k_sweep_mma<true><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                       a.ctl + 2, a.ctl, 1);
+  k_sweep_mma<false><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                        a.ctl + 2 + total, a.ctl + 1, 1);
+  *nlaunch += 2;
+  return cudaGetLastError();
+}
+
 template <int SB, int RC>
 static cudaError_t solve_sb(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   using C = SolveCfg<SB, RC>;
@@ -499,6 +663,9 @@ cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
     }
     return cudaErrorInvalidValue;
   }
+  // 32-column chunks at SB = 96 on DMMA (CHOL_SOLVE_SIMT=1: the SIMT sweeps; development switch)
+  const char* esimt = getenv("CHOL_SOLVE_SIMT");
+  if (a.rc == 32 && a.sb == 96 && !(esimt && esimt[0] == '1')) return solve_mma(a, s, nlaunch);
   const bool narrow = a.rc == 8;
   switch (a.sb) {
     case 96: return narrow ? solve_sb<96, 8>(a, s, nlaunch) : solve_sb<96, 32>(a, s, nlaunch);

@@ -130,3 +130,24 @@ def test_solve_errors():
         with pytest.raises(c.CholError) as e:
             c.chol_solve(p.h, B, 2, 0)
         assert e.value.status == -6
+
+
+@pytest.mark.parametrize("nrhs", [2, 8, 40])
+def test_solve_dmma_and_simt_sweeps_agree(nrhs, monkeypatch):
+    """Block 96 runs the DMMA sweeps (k_sweep_mma); CHOL_SOLVE_SIMT=1 the SIMT ones
+    (k_sweep): both against the oracle, and against each other within the same bound."""
+    c = _lib()
+    n, nb = 2880, 960
+    p, A, L = _factor(c, n, nb, seed=3)
+    B = spdgen.rhs(n, nrhs, 9)
+    X1 = B.copy()
+    p.solve(X1)
+    _check(A, L, B, X1)
+    p.close()
+    monkeypatch.setenv("CHOL_SOLVE_SIMT", "1")
+    p, _, _ = _factor(c, n, nb, seed=3)
+    X2 = B.copy()
+    p.solve(X2)
+    p.close()
+    _check(A, L, B, X2)
+    assert np.max(np.abs(X1 - X2)) <= 1e-12 * max(1.0, float(np.max(np.abs(X1))))
