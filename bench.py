@@ -180,13 +180,24 @@ def run_reference(args, ws, rank):
         "higher_is_better": True, "scaling": args.scaling, "vs_baseline": None, "dtype": "f64", "data": "synthetic",
         "config": {"workload": f"FP64 SPD n={n_w} nb={args.nb} (bounded sample: {sample})", "n": n_w,
                    "nb": args.nb},
-        "cpu_baseline": {"value": value, "unit": "TFLOP/s", "cores": cores, "kind": "oracle", "sample": sample},
+        "cpu_baseline": {"value": value, "unit": "TFLOP/s", "cores": cores, "kind": "oracle", "sample": sample,
+                         "cpu_model": cpu_model()},
         "e2e": {"value": value, "unit": "TFLOP/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
 
 
 # ----------------------------------------------------------------------------- our arm
+def cpu_model() -> str:
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
 def cpu_baseline(args):
     import oracle
     import spdgen
@@ -197,7 +208,7 @@ def cpu_baseline(args):
     L, info = oracle.chol_tiled(A, args.nb)
     dt = time.perf_counter() - t0
     return {"value": n_s ** 3 / 3.0 / dt / 1e12, "unit": "TFLOP/s", "cores": oracle.num_threads(),
-            "kind": "oracle",
+            "kind": "oracle", "cpu_model": cpu_model(),
             "sample": f"one factorization of a uniform SPD n={n_s} ({n_s // args.nb}x{n_s // args.nb} tiles of "
                       f"nb={args.nb}), {dt:.1f} s"}
 

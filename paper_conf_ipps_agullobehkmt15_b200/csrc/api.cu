@@ -651,10 +651,11 @@ static int factor_streamed(chol_plan_s* p, const double* A, int64_t lda, double*
     CUDA_TRY(cudaMemcpyAsync(p->d_in_flags + t, p->h_epoch, sizeof(int), cudaMemcpyHostToDevice, p->s_in));
     return 0;
   };
-  // row-major tile order (must match the scheduler's watch order, sched.cu)
+  // the scheduler's watch order (sched_arrival_order)
+  std::vector<std::pair<int, int>> arr;
+  sched_arrival_order(p->sched, arr);
   int s = 0;
-  for (int64_t i = 0; i < N && !s; ++i)
-    for (int64_t j = 0; j <= i && !s; ++j) s = copy_in(i, j);
+  for (size_t a = 0; a < arr.size() && !s; ++a) s = copy_in(arr[a].first, arr[a].second);
   if (s) return s;
   // L's strictly upper tiles are zeroed on the host once the input has been read:
   // concurrent with the input copies the memset competes with the copy engine for

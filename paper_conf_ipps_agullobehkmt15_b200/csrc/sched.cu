@@ -566,6 +566,7 @@ __global__ void k_sched_init(DevSched d, const int* roots, int nroots) {
 // ------------------------------------------------------------------ host planner
 struct SchedState {
   int64_t N = 0, nb = 0;
+  int arrival = 0;  // streamed-input tile order (arrival_order)
   int bs = 0, workers = 0, nnodes = 0, njobs = 0, nroots = 0;
   chol_opts_t opts{};
   DevSched d{};
@@ -616,9 +617,26 @@ struct Builder {
 
 }  // namespace
 
+// Streamed-input tile order.  0 (default): row-major, row i = tiles (i, 0..i) -- each
+// arriving row feeds the trailing updates of every factored column at once.  1: column 0
+// first (every TRSM_i_0 can start after N tiles), then the other tiles row-major.
+// CHOL_ARRIVAL=0/1 (development switch, read when the plan is built).
+static void arrival_order(int64_t N, int mode, std::vector<std::pair<int, int>>& tiles) {
+  tiles.clear();
+  if (mode == 1)
+    for (int i = 0; i < N; ++i) tiles.emplace_back(i, 0);
+  for (int i = 0; i < N; ++i)
+    for (int j = mode == 1 ? 1 : 0; j <= i; ++j) tiles.emplace_back(i, j);
+}
+void sched_arrival_order(const SchedState* st, std::vector<std::pair<int, int>>& tiles) {
+  arrival_order(st->N, st->arrival, tiles);
+}
+
 int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts,
                  cudaStream_t s, const DistInfo* dist) {
   auto* st = new SchedState();
+  const char* ear = getenv("CHOL_ARRIVAL");
+  st->arrival = ear ? atoi(ear) : 0;
   st->N = N;
   st->nb = nb;
   st->bs = bs;
@@ -999,15 +1017,17 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       B.deps[first_node[task]] += 1;
       watch.push_back(make_int4(first_node[task], 0, (int)t, order++));
     };
-    for (int64_t i = 0; i < N; ++i)
-      for (int64_t j = 0; j <= i; ++j) {
-        if (j == 0)
-          first_touch(i == 0 ? id_potrf(N, 0) : id_trsm(N, i, 0), i, 0);  // POTRF_0 / TRSM_i_0
-        else if (i == j)
-          first_touch(id_syrk(N, j, 0), j, j);  // SYRK_j_0
-        else
-          first_touch(id_gemm(N, i, j, 0), i, j);  // GEMM_i_j_0
-      }
+    std::vector<std::pair<int, int>> arr;
+    arrival_order(N, st->arrival, arr);
+    for (const auto& ij : arr) {
+      const int64_t i = ij.first, j = ij.second;
+      if (j == 0)
+        first_touch(i == 0 ? id_potrf(N, 0) : id_trsm(N, i, 0), i, 0);  // POTRF_0 / TRSM_i_0
+      else if (i == j)
+        first_touch(id_syrk(N, j, 0), j, j);  // SYRK_j_0
+      else
+        first_touch(id_gemm(N, i, j, 0), i, j);  // GEMM_i_j_0
+    }
     // Streamed output: every final panel tile is published (host-mapped flags)
     publish.assign(B.deps.size(), -1);
     for (int64_t k = 0; k < N; ++k) {

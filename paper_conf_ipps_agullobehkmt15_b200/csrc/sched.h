@@ -3,6 +3,9 @@
 #include <cuda.h>
 #include <cuda_runtime.h>
 
+#include <utility>
+#include <vector>
+
 #include "../../include/chol.h"
 #include "kernels.h"
 
@@ -24,6 +27,9 @@ int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slo
 int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch,
               unsigned epoch = 1);
 int sched_workers(const SchedState* st);
+// Streamed input (chol_factor from host memory): the order in which the tiles are copied
+// in, which the scheduler's watch list follows (fixed when the plan is built).
+void sched_arrival_order(const SchedState* st, std::vector<std::pair<int, int>>& tiles);
 int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* njobs);
 void sched_destroy(SchedState* st);
 }  // namespace chol
