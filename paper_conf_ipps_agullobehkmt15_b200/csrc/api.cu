@@ -774,7 +774,8 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   const int rc = nrhs == 1 ? 1 : (nrhs <= 8 && p->bs != 96) ? 8 : 32;
   const int nchunks = (int)((nrhs + rc - 1) / rc), ldw = rc * nchunks;
   const int64_t nblocks = n / p->bs;
-  const size_t need = (size_t)n * ldw, ctl = 2 + 2 * (size_t)nblocks * nchunks;
+  // one column: + 2 n doubles of chain buffers (forward / backward block results, solve.cu)
+  const size_t need = (size_t)n * ldw + (rc == 1 ? 2 * (size_t)n : 0), ctl = 2 + 2 * (size_t)nblocks * nchunks;
   if (!p->d_inv) {
     cudaError_t e = cudaMalloc(&p->d_inv, 3 * (size_t)n * p->bs * sizeof(double));
     if (e) return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
@@ -800,7 +801,7 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
     CUDA_TRY(cudaEventCreate(&p->ev5));
   }
   CUDA_TRY(cudaEventRecord(p->ev2, p->stream));
-  if (ldw != nrhs) CUDA_TRY(cudaMemsetAsync(p->d_rhs, 0, need * sizeof(double), p->stream));
+  if (ldw != nrhs) CUDA_TRY(cudaMemsetAsync(p->d_rhs, 0, (size_t)n * ldw * sizeof(double), p->stream));
   CUDA_TRY(cudaMemcpy2DAsync(p->d_rhs, ldw * 8, B, ldb * 8, nrhs * 8, n, cudaMemcpyDefault, p->stream));
   SolveArgs a{};
   a.tiles = p->tiles;
@@ -814,6 +815,7 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   a.nchunks = nchunks;
   a.rc = rc;
   a.ctl = p->d_solve_ctl;
+  a.chain = rc == 1 ? p->d_rhs + (size_t)n * ldw : nullptr;
   a.sms = p->sms;
   // development: CHOL_SOLVE_TRACE=<file> writes per-item sweep timestamps (solve.cu)
   const char* trace_path = getenv("CHOL_SOLVE_TRACE");

@@ -257,10 +257,16 @@ __device__ void producer_loop(Ctx<BS>& c) {
     if (job < 0) break;
     fence_proxy_async();  // operands written by generic stores (this or other SMs)
     if (!skip) {
-      if (type == J_UPD || type == J_PUPD || type == J_TU) {
+      const bool fused_diag = type == J_DIAG && d1.z;  // D(b) with U(b,b,b-1) in front
+      if (type == J_UPD || type == J_PUPD || type == J_TU || fused_diag) {
         int64_t ta, tb, tcb;
         int ra, rb, kb, nst, cr, cc;
-        if (type == J_UPD) {  // GEMM/SYRK block (i, j, k, bm, bn)
+        if (fused_diag) {  // the update of block (b, b) by L[b, b-1] (k, b)
+          ta = tb = tcb = c.slot(d1.x, d1.x);
+          ra = rb = cr = cc = d1.y * BS;
+          kb = (d1.y - 1) * BS;
+          nst = BS / BK;
+        } else if (type == J_UPD) {  // GEMM/SYRK block (i, j, k, bm, bn)
           ta = c.slot(d0.z, d1.x); ra = d1.y * BS;
           tb = c.slot(d0.w, d1.x); rb = d1.z * BS;
           kb = 0; nst = c.nb / BK;
@@ -423,7 +429,13 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     (void)owner;
     recv_slab(c, d, i, j, sl, owner);
   } else if (type == J_DIAG) {
-    sub_potrf_diag(c, d1.x, d1.y, info, d1.z != 0);
+    if (d1.z) {  // fused U(b,b,b-1): the K = BS update of the block first, same code as J_PUPD
+      Acc<BS> acc;
+      const int k = d1.x, b = d1.y;
+      gemm_consume(c, BS / BK, acc);
+      epi_sub_global(c, acc, c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS, c.nb, true);
+    }
+    sub_potrf_diag(c, d1.x, d1.y, info);  // its first barrier orders the stores above
   } else if (type == J_PANEL) {
     sub_potrf_panel(c, d1.x, d1.y, d1.z);
   }
@@ -757,8 +769,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       // (q,b).  One job per node, so the chain D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1)
       // never waits for a whole column or trailing update of the step.  D(nbb-1) is the
       // sink (every inner node is its ancestor).
-      // With potrf_fuse the chain's last update U(b,b,b-1) is done by D(b) itself (one job
-      // and one hop less per inner step, same bits: potf2_block).
+      // With potrf_fuse the chain's last update U(b,b,b-1) is done by D(b) itself: the job
+      // runs the J_PUPD code (producer stages, DMMA, epilogue) and then potf2 -- one node
+      // and one hop less per inner step, the same bits.
       std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1), fusedP(nbb, -1);
       if (blk) tentry[pid].assign(nbb2, -1), tfin[pid].assign(nbb2, -1);
       for (int b = 0; b < nbb; ++b) {

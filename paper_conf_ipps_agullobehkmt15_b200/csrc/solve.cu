@@ -276,23 +276,50 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
   }
 }
 
-// Single right-hand side (nrhs = 1): register-streamed matrix-vector sweeps, same items,
-// flags and recurrences as k_sweep.  Warp w owns rows [w*RPW, (w+1)*RPW) of every SB x SB
+// Sentinel of the chain buffers: a signalling NaN (quiet bit clear) -- FP64 arithmetic
+// only ever produces quiet NaNs, so no computed block result can look unpublished.
+constexpr unsigned long long kChainEmpty = 0x7FF57FF57FF57FF5ull;
+// x[i] = sign * p[i * stride] for i < M, once every value is published: all M loads in
+// flight at once (one L2 round trip when the block is there), the batch re-read until none
+// is the sentinel.
+template <int M>
+__device__ __forceinline__ void poll_block(double (&x)[M], const double* p, int stride, double sign) {
+  unsigned long long v[M];
+  bool empty;
+  do {
+#pragma unroll
+    for (int i = 0; i < M; ++i)
+      asm volatile("ld.relaxed.gpu.global.b64 %0, [%1];" : "=l"(v[i]) : "l"(p + i * stride) : "memory");
+    empty = false;
+#pragma unroll
+    for (int i = 0; i < M; ++i) empty |= v[i] == kChainEmpty;
+  } while (empty);
+#pragma unroll
+  for (int i = 0; i < M; ++i) x[i] = sign * __longlong_as_double((long long)v[i]);
+}
+__global__ void k_fill_u64(unsigned long long* p, int64_t n, unsigned long long v) {
+  for (int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; i < n; i += (int64_t)gridDim.x * blockDim.x)
+    p[i] = v;
+}
+
+// Single right-hand side (nrhs = 1): register-streamed matrix-vector sweeps, same items
+// and recurrences as k_sweep; block results are published through a chain buffer whose
+// values double as flags (poll_block) -- no flag round trip, no barrier before publishing.  Warp w owns rows [w*RPW, (w+1)*RPW) of every SB x SB
 // matrix it streams and lane l the columns l, l+32, ... (KPL = SB/32), so each warp-load
 // is 256 contiguous bytes.  A matrix element is used once, so it is loaded straight into
 // registers (no shared-memory staging -- staging 73 KB per stage through cp.async or
 // per-row bulk copies capped a CTA at ~17 GB/s, tools/solve_trace.py), the next stage's
 // matrix while the current one is multiplied; each warp walks the stages on its own
-// (its lane 0 acquires the flag of the block row consumed), so CTA barriers only frame
-// the two reductions of an item.
+// (its lanes poll the values of the block row consumed, poll_block), so CTA barriers only frame the
+// two reductions of an item.
 //   FWD, non-transposed: partial p[i] (warp row i) over the lane's columns, reduced
 //       across lanes;
 //   BWD, transposed (L_cb^T, inv_b^T, Mb_b^T read from the stored blocks): partial p[j]
 //       (column l + 32 j) over the warp's rows, reduced across warps.
 template <int SB, bool FWD>
 __global__ void __launch_bounds__(kSolveThreads, 1)
-    k_sweep_vec(const double* tiles, int nb, int nblocks, const double* aux, double* W, int* flags, int* counter,
-                int epoch, uint64_t* trace) {
+    k_sweep_vec(const double* tiles, int nb, int nblocks, const double* aux, double* W, double* chain, int* counter,
+                uint64_t* trace) {
   constexpr int RPW = SB / 8, KPL = SB / 32, NP = FWD ? RPW : KPL, RP = 33;
   __shared__ double red[FWD ? SB * RP : 8 * SB];
   __shared__ double xs[SB];
@@ -308,32 +335,30 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
 #pragma unroll
       for (int j = 0; j < KPL; ++j) R[i][j] = __ldcs(G + (int64_t)(warp * RPW + i) * ld + lane + 32 * j);
   };
-  // p (+)= sign * Op(R) x with x = block row c of W (c >= 0, after its flag) or xs (c < 0)
+  // p (+)= sign * Op(R) x with x = block row c (c >= 0: polled from the chain buffer, where
+  // each value appears as soon as its producer stores it) or xs (c < 0)
   auto apply = [&](const double (&R)[RPW][KPL], int c, double sign) {
-    const double* xv = xs;
-    if (c >= 0) {
-      if (lane == 0) {
-        const int* f = flags + c;
-        int v;
-        do {
-          asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(f) : "memory");
-        } while (v != epoch);
-      }
-      __syncwarp();
-      xv = W + (int64_t)c * SB;
-    }
+    const double* xv = c >= 0 ? chain + (int64_t)c * SB : xs;
     if (FWD) {
       double x[KPL];
+      if (c >= 0) {
+        poll_block<KPL>(x, xv + lane, 32, sign);
+      } else {
 #pragma unroll
-      for (int j = 0; j < KPL; ++j) x[j] = sign * (c >= 0 ? __ldcg(xv + lane + 32 * j) : xv[lane + 32 * j]);
+        for (int j = 0; j < KPL; ++j) x[j] = sign * xv[lane + 32 * j];
+      }
 #pragma unroll
       for (int i = 0; i < RPW; ++i)
 #pragma unroll
         for (int j = 0; j < KPL; ++j) p[i] = fma(R[i][j], x[j], p[i]);
     } else {
       double x[RPW];
+      if (c >= 0) {
+        poll_block<RPW>(x, xv + warp * RPW, 1, sign);
+      } else {
 #pragma unroll
-      for (int i = 0; i < RPW; ++i) x[i] = sign * (c >= 0 ? __ldcg(xv + warp * RPW + i) : xv[warp * RPW + i]);
+        for (int i = 0; i < RPW; ++i) x[i] = sign * xv[warp * RPW + i];
+      }
 #pragma unroll
       for (int i = 0; i < RPW; ++i)
 #pragma unroll
@@ -425,10 +450,13 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
       }
     }
     const double y = reduce();
-    if (t < SB) __stcg(W + (int64_t)b * SB + t, y);
-    __syncthreads();  // every store before the release (cumulative)
+    if (t < SB) {
+      __stcg(W + (int64_t)b * SB + t, y);
+      // publish: every value is its own flag (8-byte stores are single-copy atomic, and
+      // arithmetic never yields the signalling-NaN sentinel the buffer was filled with)
+      asm volatile("st.relaxed.gpu.global.f64 [%0], %1;" ::"l"(chain + (int64_t)b * SB + t), "d"(y) : "memory");
+    }
     if (t == 0) {
-      asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(flags + b), "r"(epoch) : "memory");
       if (trace) {
         uint64_t* tt = trace + 6 * (int64_t)(item + (FWD ? 0 : nblocks));
         unsigned smid;
@@ -455,12 +483,13 @@ static cudaError_t solve_vec(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
     ++*nlaunch;
   }
   const int grid = std::min(nblocks, a.sms);
-  if ((e = cudaMemsetAsync(a.ctl, 0, (2 + 2 * (size_t)nblocks) * sizeof(int), s))) return e;
-  k_sweep_vec<SB, true><<<grid, kSolveThreads, 0, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ctl + 2, a.ctl, 1,
+  if ((e = cudaMemsetAsync(a.ctl, 0, 2 * sizeof(int), s))) return e;
+  k_fill_u64<<<a.sms, 256, 0, s>>>(reinterpret_cast<unsigned long long*>(a.chain), 2 * a.n, kChainEmpty);
+  k_sweep_vec<SB, true><<<grid, kSolveThreads, 0, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.chain, a.ctl,
                                                         a.trace);
-  k_sweep_vec<SB, false><<<grid, kSolveThreads, 0, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ctl + 2 + nblocks,
-                                                         a.ctl + 1, 1, a.trace);
-  *nlaunch += 2;
+  k_sweep_vec<SB, false><<<grid, kSolveThreads, 0, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.chain + a.n,
+                                                         a.ctl + 1, a.trace);
+  *nlaunch += 3;
   return cudaGetLastError();
 }
 

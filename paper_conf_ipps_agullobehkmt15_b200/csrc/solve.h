@@ -18,6 +18,7 @@ struct SolveArgs {
   int rc;               // right-hand-side columns per work item: 1 (nrhs = 1), 8 (nrhs <= 8) or 32
   int* ctl;             // 2 + 2 * (n / sb) * nchunks ints of control (counters, flags)
   int sms;
+  double* chain;        // nrhs = 1: 2 n doubles (forward / backward block results, polled), or null
   uint64_t* trace;      // development: 2 * (n / sb) * nchunks items x 6 u64 (solve.cu), or null
 };
 cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch);

@@ -637,28 +637,14 @@ __device__ __forceinline__ void potf2_panels(const Ctx<BS>& c, Potf2Regs<BS>& s,
 //       blocks with FP64 DMMA (A operand = its own solved fragments).
 // A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
 // reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
-//
-// Pu != null (POTRF block DAG, chain D(b-1) -> P(b,b-1) -> U(b,b,b-1) -> D(b)): the last
-// update of the block, A -= Pu Pu^T with Pu = L[b, b-1] (BS x BS, ld lda), is fused in
-// front of the factorization -- one job and one hop less on the POTRF chain, and the
-// updated block never goes through global memory.  Pu is staged in the idle TMA ring
-// (pitch kPitch); every 8 x 8 block is accumulated from zero with exactly the DMMA
-// sequence of the K = BS update job (gemm_mainloop: stages of BK = 16, k-slot t <-> k =
-// 16 s + 4 t + 2 h + {0, 1}) and subtracted once, so the result is bit for bit that of
-// U(b,b,b-1) followed by D(b) (reading R15).
 template <int BS>
-__device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info,
-                                            const double* Pu = nullptr) {
+__device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
   constexpr int NB = BS / 8;
   static_assert(NB % 2 == 0 && NB / 2 <= 7, "paired row blocks; warp 7 factors the diagonal blocks");
   using R = Potf2Regs<BS>;
   double* dd = c.lbuf();        // 8 x 8 diagonal block (pitch 8) + 8 reciprocals
   double* rdv = c.lbuf() + 64;
   bar_sync(kBarCompute, kComputeThreads);  // lbuf / pans reuse
-  if (Pu) {
-    load_block<BS>(c.buf(), Pu, lda);
-    bar_sync(kBarCompute, kComputeThreads);
-  }
   if (c.warp == 7) {
     // factor warp: its own loop, disjoint from the row-block code (register pressure)
 #pragma unroll 1
@@ -682,36 +668,6 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
   s.rb1 = NB - 1 - c.warp;
   const int g = s.g, t = s.t;
   if (s.active) {
-    if (Pu) {
-      // acc = Pu[rows of the block] Pu[rows of column block cb]^T, in the x slots
-      constexpr int P = Cfg<BS>::kPitch;
-      const double* ps = c.buf();
-#pragma unroll
-      for (int e = 0; e <= NB; ++e) s.x[e][0] = s.x[e][1] = 0.0;
-#pragma unroll 1
-      for (int k0 = 0; k0 < BS; k0 += BK) {
-#pragma unroll
-        for (int h = 0; h < 2; ++h) {
-          // per 8 x 8 block: DMMA on the .x k-slots, then on the .y ones (the order of
-          // consume_stage); the blocks are independent, so one B fragment at a time
-          const int kk = k0 + 4 * t + 2 * h;
-          double2 af[2];
-#pragma unroll
-          for (int mi = 0; mi < 2; ++mi) af[mi] = *reinterpret_cast<const double2*>(ps + (8 * s.rb(mi) + g) * P + kk);
-#pragma unroll
-          for (int cb = 0; cb < NB; ++cb) {
-            if (cb > s.rb1) continue;  // warp-uniform
-            const double2 bf = *reinterpret_cast<const double2*>(ps + (8 * cb + g) * P + kk);
-#pragma unroll
-            for (int mi = 0; mi < 2; ++mi)
-              if (cb <= s.rb(mi)) {
-                dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], af[mi].x, bf.x);
-                dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], af[mi].y, bf.y);
-              }
-          }
-        }
-      }
-    }
 #pragma unroll
     for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
@@ -719,13 +675,8 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
         if (cb > s.rb(mi)) continue;  // strictly upper blocks: never needed
         const double2 v =
             __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t));
-        if (Pu) {
-          s.x[R::sl(mi, cb)][0] = v.x - s.x[R::sl(mi, cb)][0];
-          s.x[R::sl(mi, cb)][1] = v.y - s.x[R::sl(mi, cb)][1];
-        } else {
-          s.x[R::sl(mi, cb)][0] = v.x;
-          s.x[R::sl(mi, cb)][1] = v.y;
-        }
+        s.x[R::sl(mi, cb)][0] = v.x;
+        s.x[R::sl(mi, cb)][1] = v.y;
       }
     if (c.warp == 0) {  // hand over the first diagonal block (rb0 = 0, slot 0)
       *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(s.x[0][0], s.x[0][1]);
@@ -791,13 +742,13 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
 // POTRF_k, inner step b (nested tiled Cholesky of the diagonal tile with block BS):
 //   potf2 of block (b, b)
 template <int BS>
-__device__ __forceinline__ void potf2_job(double* A, int lda, int col0, int* info, const double* Pu = nullptr) {
+__device__ __forceinline__ void potf2_job(double* A, int lda, int col0, int* info) {
   // out of line with plain arguments: the in-block factorization gets its own register
   // allocation (it needs ~164 registers) instead of sharing one with the GEMM paths
   Ctx<BS> c{};
   c.warp = threadIdx.x >> 5;
   c.lane = threadIdx.x & 31;
-  potf2_block(c, A, lda, col0, info, Pu);
+  potf2_block(c, A, lda, col0, info);
 }
 // solve_block out of line with plain arguments, for the persistent kernel (three call
 // sites: TRSM slab, TS, POTRF panel): one copy with its own register allocation, so its
@@ -809,11 +760,10 @@ __device__ __noinline__ void solve_block_job(double* X, int ldx, const double* L
   c.lane = threadIdx.x & 31;
   solve_block(c, X, ldx, Ld, ldl);
 }
-//   fused (b > 0): A[b, b] -= L[b, b-1] L[b, b-1]^T first (the block DAG's U(b,b,b-1))
 template <int BS>
-__device__ __forceinline__ void sub_potrf_diag(Ctx<BS>& c, int k, int b, int* info, bool fused = false) {
+__device__ __forceinline__ void sub_potrf_diag(Ctx<BS>& c, int k, int b, int* info) {
   double* A = c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS;
-  potf2_job<BS>(A, c.nb, k * c.nb + b * BS, info, fused ? A - BS : nullptr);
+  potf2_job<BS>(A, c.nb, k * c.nb + b * BS, info);
 }
 //   block (r, b), r > b:  X <- X L_bb^{-T}
 template <int BS>
