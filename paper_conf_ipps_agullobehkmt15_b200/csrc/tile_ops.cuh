@@ -220,11 +220,74 @@ __device__ __forceinline__ void zero_acc(Acc<BS>& acc) {
 }
 
 // Consumer side only (warp-specialised kernel: a separate producer issues the stages).
+// Software-pipelined across stages: the fragments of the next stage's first half
+// (k-slots 4t, 4t+1) are loaded -- after its full barrier -- before the DMMAs of this
+// stage's second half, so the shared-memory latency at a stage boundary hides behind
+// ~36 queued DMMAs per warp instead of stalling the pipe (consume_stage paid it every
+// 16 k).  Same DMMA sequence per accumulator as consume_stage (bitwise-identical).
 template <int BS>
 __device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) {
+  using C = Cfg<BS>;
   zero_acc<BS>(acc);
   const uint32_t rt_zero = threadIdx.y;  // 0, unknown to the compiler (see consume_stage)
-  for (int s = 0; s < nst; ++s) consume_stage(c, c.it + s, acc, rt_zero);
+  if (nst <= 0) return;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  const uint32_t base = smem_u32(c.pipe());
+  const uint32_t aoff = (wm * C::WM + g) * 128, boff = C::kOpBytes + (wn * C::WN + g) * 128;
+  const uint32_t ch0 = ((2 * t) ^ g) << 4, ch1 = ((2 * t + 1) ^ g) << 4;  // logical chunks 2t, 2t+1
+  double2 a0[C::MI], b0[C::NI];
+  uint32_t q = c.it;
+  {
+    const uint32_t st = q % kStages;
+    mbar_wait(&c.full()[st], (q / kStages) & 1);
+    const uint32_t sa = base + st * 2 * C::kOpBytes;
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(sa + aoff + mi * 8 * 128 + ch0);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) b0[ni] = lds128(sa + boff + ni * 8 * 128 + ch0);
+  }
+  for (int s = 0; s < nst; ++s, ++q) {
+    const uint32_t st = q % kStages;
+    const uint32_t sa = base + st * 2 * C::kOpBytes;
+    double2 a1[C::MI], b1[C::NI];
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) a1[mi] = lds128(sa + aoff + mi * 8 * 128 + ch1);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) b1[ni] = lds128(sa + boff + ni * 8 * 128 + ch1);
+    uint32_t dep = 0;
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(a0[mi].x) ^ __double2loint(a1[mi].x);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(b0[ni].x) ^ __double2loint(b1[ni].x);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a0[mi].x, b0[ni].x);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a0[mi].y, b0[ni].y);
+    // this stage's loads have all returned (dep): hand the buffer back to the producer
+    __syncwarp();
+    if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty()[st]);
+    if (s + 1 < nst) {  // next stage, first half, while the second half's DMMAs run
+      const uint32_t sn = (q + 1) % kStages;
+      mbar_wait(&c.full()[sn], ((q + 1) / kStages) & 1);
+      const uint32_t san = base + sn * 2 * C::kOpBytes;
+#pragma unroll
+      for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(san + aoff + mi * 8 * 128 + ch0);
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) b0[ni] = lds128(san + boff + ni * 8 * 128 + ch0);
+    }
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a1[mi].x, b1[ni].x);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a1[mi].y, b1[ni].y);
+  }
   c.it += nst;
 }
 
