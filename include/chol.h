@@ -137,6 +137,16 @@ int chol_generate(chol_plan_t p, uint64_t seed, int family);
 int chol_scatter(chol_plan_t p, const double* A, int64_t lda);
 int chol_gather(chol_plan_t p, double* L, int64_t ldl);
 
+/* Host (or device) I/O of the tiles this plan OWNS, packed: `count` nb x nb row-major
+ * tiles back to back, in Algorithm 1 tile order (i ascending, then j <= i ascending),
+ * restricted to the tiles the rank owns (all N(N+1)/2 tiles on a single-GPU plan;
+ * chol_get_dist's nowned on a distributed one) -- the per-rank form of the paper's tile
+ * layout, with no n x n host matrix on any rank.  After a
+ * factorization the diagonal tiles hold L_kk with zeros above the diagonal.
+ * count != the owned-tile count -> -6; null / misaligned pointer -> -4.  Synchronous. */
+int chol_scatter_tiles(chol_plan_t p, const double* tiles, int64_t count);
+int chol_gather_tiles(chol_plan_t p, double* tiles, int64_t count);
+
 /* Factor the tile store in place (no layout conversion); *info as chol_factor. */
 int chol_factor_inplace(chol_plan_t p, int* info);
 

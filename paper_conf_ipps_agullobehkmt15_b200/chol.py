@@ -64,6 +64,8 @@ def _load():
         "chol_generate": ([P, u64, i32], i32),
         "chol_scatter": ([P, vp, i64], i32),
         "chol_gather": ([P, vp, i64], i32),
+        "chol_scatter_tiles": ([P, vp, i64], i32),
+        "chol_gather_tiles": ([P, vp, i64], i32),
         "chol_factor_inplace": ([P, ctypes.POINTER(i32)], i32),
         "chol_last_times": ([P, dp, dp], i32),
         "chol_get_stream": ([P, ctypes.POINTER(vp)], i32),
@@ -103,7 +105,8 @@ EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_dest
             "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
             "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
             "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
-            "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times")
+            "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times", "chol_scatter_tiles",
+            "chol_gather_tiles")
 
 
 def _ptr(x) -> int:
@@ -188,6 +191,15 @@ def chol_scatter(plan: int, A, lda: int) -> None:
 
 def chol_gather(plan: int, L, ldl: int) -> None:
     _check(_lib.chol_gather(plan, _ptr(L), ldl), "chol_gather")
+
+
+def chol_scatter_tiles(plan: int, tiles, count: int) -> None:
+    """The plan's OWNED tiles, packed nb x nb in Algorithm 1 tile order (host or device)."""
+    _check(_lib.chol_scatter_tiles(plan, _ptr(tiles), count), "chol_scatter_tiles")
+
+
+def chol_gather_tiles(plan: int, tiles, count: int) -> None:
+    _check(_lib.chol_gather_tiles(plan, _ptr(tiles), count), "chol_gather_tiles")
 
 
 def chol_last_times(plan: int) -> tuple[float, float]:

@@ -530,6 +530,24 @@ extern "C" int chol_gather(chol_plan_t p, double* L, int64_t ldl) {
   return 0;
 }
 
+// The owned tiles occupy slots 0 .. nowned-1 in tile order (dist_layout; identity on
+// one GPU): one contiguous copy each way.
+static int owned_tiles_copy(chol_plan_t p, void* dst, const void* src, int64_t count) {
+  if (!p || !dst || !src || (reinterpret_cast<uintptr_t>(dst) & 7) || (reinterpret_cast<uintptr_t>(src) & 7))
+    return -4;
+  if (count != (p->dist ? p->nowned : p->ntiles)) return -6;
+  cudaSetDevice(p->device);
+  CUDA_TRY(cudaMemcpyAsync(dst, src, (size_t)count * p->nb * p->nb * sizeof(double), cudaMemcpyDefault, p->stream));
+  CUDA_TRY(cudaStreamSynchronize(p->stream));
+  return 0;
+}
+extern "C" int chol_scatter_tiles(chol_plan_t p, const double* tiles, int64_t count) {
+  return p ? owned_tiles_copy(p, p->tiles, tiles, count) : -4;
+}
+extern "C" int chol_gather_tiles(chol_plan_t p, double* tiles, int64_t count) {
+  return p ? owned_tiles_copy(p, tiles, p->tiles, count) : -4;
+}
+
 extern "C" int chol_generate(chol_plan_t p, uint64_t seed, int family) {
   if (!p) return -4;
   if (family < 0 || family > 1) return -6;

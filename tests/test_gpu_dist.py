@@ -142,3 +142,56 @@ def test_dist_bench_sizes_bitwise_equal_single_gpu(n, p, q):
         assert torch.equal(Ld[idx[o:], idx[o:] - o], Lb[o, o:]), o
         nnz_band += int(torch.count_nonzero(Lb[o, o:]))
     assert int(torch.count_nonzero(Ld)) == nnz_band  # nothing outside the band
+
+
+def _packed_owned(M, nb, owner_ok):
+    """Tiles (i, j), i >= j, in Algorithm 1 tile order, kept where owner_ok(i, j), packed."""
+    N = M.shape[0] // nb
+    return np.concatenate([M[i * nb:(i + 1) * nb, j * nb:(j + 1) * nb].ravel()
+                           for i in range(N) for j in range(i + 1) if owner_ok(i, j)])
+
+
+def test_scatter_gather_tiles_single_and_distributed():
+    """chol_scatter_tiles / chol_gather_tiles: the owned tiles, packed in tile order, in and
+    out of a single-GPU plan and of each rank of a 2x2 distributed plan; the factor equals
+    the oracle's, and a wrong tile count is rejected (-6)."""
+    c = _lib()
+    n, nb, seed = 1920, 96, 17
+    A = spdgen.uniform_spd(n, seed)
+    ref, _ = oracle.chol_tiled(A, nb)
+    N = n // nb
+    # single GPU: every tile is owned
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+        packed = np.ascontiguousarray(_packed_owned(A, nb, lambda i, j: True))
+        ntiles = N * (N + 1) // 2
+        c.chol_scatter_tiles(p.h, packed, ntiles)
+        assert c.chol_factor_inplace(p.h) == 0
+        out = np.empty_like(packed)
+        c.chol_gather_tiles(p.h, out, ntiles)
+        want = _packed_owned(np.tril(ref), nb, lambda i, j: True)
+        assert np.max(np.abs(out - want)) <= 1e-10 * np.max(np.abs(want))
+        with pytest.raises(c.CholError):
+            c.chol_gather_tiles(p.h, out, ntiles - 1)
+    # 2 x 2 logical ranks: each rank streams only its own tiles
+    R, pg, qg = 4, 2, 2
+    sms = torch.cuda.get_device_properties(0).multi_processor_count
+    plans = [c.DistPlan(n, nb, R, r, grid_p=pg, grid_q=qg, workers=sms // R, policy=1) for r in range(R)]
+    c.DistPlan.connect_local(plans)
+    owner = lambda i, j: (i % pg) * qg + (j % qg)  # noqa: E731  (SURVEY §8e)
+    counts = []
+    for r, pl in enumerate(plans):
+        mine = np.ascontiguousarray(_packed_owned(A, nb, lambda i, j: owner(i, j) == r))
+        cnt = mine.size // (nb * nb)
+        assert cnt == c.chol_get_dist(pl.h)["nowned"]
+        counts.append(cnt)
+        c.chol_scatter_tiles(pl.h, mine, cnt)
+    for pl in plans:
+        c.chol_factor_async(pl.h)
+    assert [c.chol_wait(pl.h) for pl in plans] == [0] * R
+    for r, pl in enumerate(plans):
+        out = np.empty(counts[r] * nb * nb)
+        c.chol_gather_tiles(pl.h, out, counts[r])
+        want = _packed_owned(np.tril(ref), nb, lambda i, j: owner(i, j) == r)
+        assert np.max(np.abs(out - want)) <= 1e-10 * np.max(np.abs(ref))
+    for pl in plans:
+        pl.close()
