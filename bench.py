@@ -116,6 +116,12 @@ class ClockSampler:
                 "power_w_max": max(power) if power else None, "samples": len(rows), "reasons": reasons}
 
 
+# Development check of the multi-process path on a one-GPU box: BENCH_SHARED_GPU=1 puts
+# every rank on cuda:0 (CUDA IPC between processes still applies), uses gloo for the
+# host-side collectives and gives each rank SMs / WORLD_SIZE workers.  Not a scaling number.
+SHARED_GPU = os.environ.get("BENCH_SHARED_GPU") == "1"
+
+
 def dist_setup():
     ws = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
@@ -123,8 +129,10 @@ def dist_setup():
     if ws > 1:
         import torch
         import torch.distributed as dist
+        if SHARED_GPU:
+            local = 0
         torch.cuda.set_device(local)
-        dist.init_process_group("nccl")
+        dist.init_process_group("gloo" if SHARED_GPU else "nccl")
     return ws, rank, local
 
 
@@ -139,7 +147,7 @@ def allmax(ws, x: float) -> float:
         return x
     import torch
     import torch.distributed as dist
-    t = torch.tensor([x], dtype=torch.float64, device="cuda")
+    t = torch.tensor([x], dtype=torch.float64, device="cpu" if SHARED_GPU else "cuda")
     dist.all_reduce(t, op=dist.ReduceOp.MAX)
     return float(t.item())
 
@@ -165,14 +173,14 @@ def run_reference(args, ws, rank):
     times = []
     for it in range(args.warmup + args.steps):
         t0 = time.perf_counter()
-        L, info = oracle.chol_tiled(A, args.nb)
+        L, info = oracle.chol_tiled(A, args.nb, host_cores())
         dt = time.perf_counter() - t0
         assert info == 0
         if it >= args.warmup:
             times.append(dt)
     tot = sum(times)
     value = n_s ** 3 / 3.0 / (tot / len(times)) / 1e12
-    cores = oracle.num_threads()
+    cores = oracle.num_threads(host_cores())
     sample = f"uniform SPD n={n_s} ({n_s // args.nb}x{n_s // args.nb} tiles of nb={args.nb}) per step"
     line = {
         "impl": "reference", "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": args.gpus,
@@ -188,6 +196,15 @@ def run_reference(args, ws, rank):
 
 
 # ----------------------------------------------------------------------------- our arm
+def host_cores() -> int:
+    """All host cores this process may run on (torchrun sets OMP_NUM_THREADS=1 per rank;
+    the oracle baseline is stated on the box's cores, so the count is passed explicitly)."""
+    try:
+        return len(os.sched_getaffinity(0))
+    except (AttributeError, OSError):
+        return os.cpu_count() or 1
+
+
 def cpu_model() -> str:
     try:
         for line in open("/proc/cpuinfo"):
@@ -205,9 +222,9 @@ def cpu_baseline(args):
     n_s -= n_s % args.nb
     A = spdgen.uniform_spd(n_s, args.seed)
     t0 = time.perf_counter()
-    L, info = oracle.chol_tiled(A, args.nb)
+    L, info = oracle.chol_tiled(A, args.nb, host_cores())
     dt = time.perf_counter() - t0
-    return {"value": n_s ** 3 / 3.0 / dt / 1e12, "unit": "TFLOP/s", "cores": oracle.num_threads(),
+    return {"value": n_s ** 3 / 3.0 / dt / 1e12, "unit": "TFLOP/s", "cores": oracle.num_threads(host_cores()),
             "kind": "oracle", "cpu_model": cpu_model(),
             "sample": f"one factorization of a uniform SPD n={n_s} ({n_s // args.nb}x{n_s // args.nb} tiles of "
                       f"nb={args.nb}), {dt:.1f} s"}
@@ -276,7 +293,11 @@ def run_dist(args, ws, rank, local):
         dist.all_gather_object(out, blob)
         return out
 
-    plan = c.DistPlan(n, nb, ws, rank, allgather=allgather, grid_p=p, grid_q=q, policy=POLICIES[args.policy])
+    extra = {}
+    if SHARED_GPU:
+        extra["workers"] = torch.cuda.get_device_properties(0).multi_processor_count // ws
+    plan = c.DistPlan(n, nb, ws, rank, allgather=allgather, grid_p=p, grid_q=q, policy=POLICIES[args.policy],
+                      **extra)
     for _ in range(args.warmup):
         c.chol_generate(plan.h, args.seed, 0)
         barrier(ws)
@@ -295,9 +316,40 @@ def run_dist(args, ws, rank, local):
             launches += c.chol_last_launches(plan.h)
     clocks = clk.summary()
     d = c.chol_get_dist(plan.h)
-    plan.close()
     t_step = sum(times) / len(times)
     value = flops / t_step / 1e12
+
+    # end-to-end: each rank streams ITS OWN tiles from pinned host memory through the
+    # C-ABI (chol_scatter_tiles -> chol_factor_inplace -> chol_gather_tiles), copies inside
+    # the timed region, wall time max over ranks; no rank holds the n x n matrix
+    e2e = None
+    if not args.no_e2e:
+        nown, tile_b = d["nowned"], nb * nb * 8
+        ntiles = (n // nb) * (n // nb + 1) // 2
+        try:
+            h_in = torch.empty(nown * nb * nb, dtype=torch.float64, pin_memory=True)
+            h_out = torch.empty(nown * nb * nb, dtype=torch.float64, pin_memory=True)
+            c.chol_generate(plan.h, args.seed, 0)
+            c.chol_gather_tiles(plan.h, h_in, nown)  # this rank's input tiles (untimed)
+            et = []
+            for _ in range(3):
+                barrier(ws)
+                torch.cuda.synchronize()
+                t0 = time.perf_counter()
+                c.chol_scatter_tiles(plan.h, h_in, nown)
+                info = c.chol_factor_inplace(plan.h)
+                c.chol_gather_tiles(plan.h, h_out, nown)
+                dt = time.perf_counter() - t0
+                assert info == 0, info
+                et.append(allmax(ws, dt))
+            t_e = sum(et) / len(et)
+            e2e = {"value": flops / t_e / 1e12, "unit": "TFLOP/s", "h2d_bytes_per_step": ntiles * tile_b,
+                   "d2h_bytes_per_step": ntiles * tile_b, "ms_per_step": 1e3 * t_e,
+                   "path": "per rank: owned tiles pinned host -> chol_scatter_tiles -> chol_factor_inplace -> "
+                           "chol_gather_tiles -> pinned host; bytes summed over ranks"}
+        except Exception as ex:  # report, do not lose the device-timed line
+            e2e = {"unavailable": f"{type(ex).__name__}: {ex}"[:200]}
+    plan.close()
     line = {
         "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": ws, "steps": args.steps,
         "warmup": args.warmup, "ms_per_step": 1e3 * t_step, "higher_is_better": True, "scaling": args.scaling,
@@ -315,6 +367,10 @@ def run_dist(args, ws, rank, local):
                      "peak_source": "measured FP64 DMMA microbenchmark"},
         "clocks": clocks, "gpu_launches": launches,
     }
+    if SHARED_GPU:
+        line["note"] = "BENCH_SHARED_GPU=1: all ranks on cuda:0 (multi-process path check, not a scaling number)"
+    if e2e is not None:
+        line["e2e"] = e2e
     if rank == 0:
         print(json.dumps(line), flush=True)
 
