@@ -69,7 +69,8 @@ typedef struct {
   int trsm_pin_distance; /* STATIC only: TRSM_i_k with i-k <= d are pinned (0 = default 1:
                             the TRSMs on the POTRF-TRSM-SYRK chain) */
   int latency_workers;   /* STATIC only: CTAs reserved for pinned tasks (0 = default 16) */
-  int grid_p, grid_q;    /* 2D block-cyclic process grid (0,0 = 1 x ngpus) */
+  int grid_p, grid_q;    /* 2D block-cyclic process grid (0,0 = the squarest p x q with
+                            p <= q for chol_plan; 1 x nranks for chol_plan_dist) */
   int trace;             /* 1 = record per-task t0/t1 (needed by chol_trace);
                             2 = also per-job (CTA sub-task) records (chol_job_trace) */
   int executor;          /* CHOL_EXEC_* */
@@ -86,11 +87,16 @@ typedef struct {
   uint64_t t1_ns;  /* last sub-task end */
 } chol_task_rec_t;
 
-/* Plan an n x n factorization in nb x nb tiles on ngpus GPUs (the devices
- * 0..ngpus-1 of this process; this build supports ngpus == 1 here and
- * multi-GPU through chol_plan_dist).  Allocates the tile store
- * (N(N+1)/2 tiles, 8*nb*nb bytes each), the task tables and the scheduler
- * state on the device.  *out receives the plan; free it with chol_destroy. */
+/* Plan an n x n factorization in nb x nb tiles on ngpus GPUs, the devices
+ * 0..ngpus-1 of this process.  ngpus == 1: allocates the tile store (N(N+1)/2 tiles,
+ * 8*nb*nb bytes each), the task tables and the scheduler state on the current device.
+ * ngpus > 1: one rank of the 2D block-cyclic plan (chol_plan_dist, grid_p x grid_q,
+ * default the squarest p <= q) per device, connected in-process through peer memory
+ * (NVLink); chol_factor / chol_factor_inplace / chol_generate / chol_scatter /
+ * chol_gather / chol_trace fan out to the ranks (A and L: host pointers or device
+ * pointers, copied by the owners); chol_solve, chol_run_*, chol_job_trace and the
+ * per-rank tile calls return -8.  ngpus > visible devices or grid_p * grid_q != ngpus
+ * -> -3.  *out receives the plan; free it with chol_destroy. */
 int chol_plan(int64_t n, int64_t nb, int ngpus, chol_plan_t* out);
 int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t* opts, chol_plan_t* out);
 

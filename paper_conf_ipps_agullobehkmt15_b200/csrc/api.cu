@@ -70,7 +70,11 @@ struct chol_plan_s {
   size_t ctl_cap = 0;           // ints
   double last_solve_s = 0.0, last_sweeps_s = 0.0;
   cudaEvent_t ev4 = nullptr, ev5 = nullptr;
+  // ---- one process driving ngpus devices (chol_plan with ngpus > 1): one distributed
+  // rank plan per device, connected with plain peer pointers; every call fans out
+  std::vector<chol_plan_s*> subs;
 };
+static bool is_multi(const chol_plan_s* p) { return p && !p->subs.empty(); }
 
 #define CUDA_TRY(x)                                   \
   do {                                                \
@@ -130,6 +134,11 @@ static int pick_block(int64_t nb) {
 // ------------------------------------------------------------------ plan
 extern "C" int chol_destroy(chol_plan_t p) {
   if (!p) return -4;
+  if (is_multi(p)) {
+    for (chol_plan_s* sp : p->subs) chol_destroy(sp);
+    delete p;
+    return 0;
+  }
   if (p->sched) sched_destroy(p->sched);
   cudaSetDevice(p->device);
   if (p->stream) cudaStreamSynchronize(p->stream);
@@ -165,6 +174,8 @@ extern "C" int chol_destroy(chol_plan_t p) {
   return 0;
 }
 
+static int plan_multi(int64_t n, int64_t nb, int ngpus, const chol_opts_t& opts, chol_plan_t* out);
+
 extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t* o, chol_plan_t* out) {
   if (!out) return -4;
   *out = nullptr;
@@ -177,14 +188,23 @@ extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t*
       opts.trace > 2)
     return -6;
   int ndev = 0;
-  if (cudaGetDeviceCount(&ndev) != cudaSuccess) ndev = 0;
-  if (ngpus < 1 || ngpus > ndev) return -3;
+  if (cudaGetDeviceCount(&ndev) != cudaSuccess) {
+    cudaGetLastError();
+    ndev = 0;
+  }
+  // development check on a one-GPU box: CHOL_MULTI_ONE_DEVICE=1 puts every rank of a
+  // multi-device plan on the current device (SMs / ngpus workers each)
+  const char* e1d = getenv("CHOL_MULTI_ONE_DEVICE");
+  const bool one_dev = e1d && e1d[0] == '1' && ndev >= 1;
+  if (ngpus < 1 || (ngpus > ndev && !one_dev)) return -3;
   if (opts.grid_p == 0 && opts.grid_q == 0) {
-    opts.grid_p = 1;
-    opts.grid_q = ngpus;
+    opts.grid_p = 1;  // p <= q, as square as possible
+    for (int c = 1; c * c <= ngpus; ++c)
+      if (ngpus % c == 0) opts.grid_p = c;
+    opts.grid_q = ngpus / opts.grid_p;
   }
   if (opts.grid_p * opts.grid_q != ngpus) return -3;
-  if (ngpus > 1) return -8;  // multi-GPU runs one process per GPU (chol_plan_dist)
+  if (ngpus > 1) return plan_multi(n, nb, ngpus, opts, out);
 
   auto* p = new (std::nothrow) chol_plan_s();
   if (!p) return -9;
@@ -423,8 +443,104 @@ extern "C" int chol_get_dist(chol_plan_t p, int* rank, int* nranks, int* grid_p,
   return 0;
 }
 
+// ------------------------------------------------------------------ one process, ngpus devices
+// chol_plan(n, nb, ngpus > 1) (SURVEY §8b process model): rank r of the 2D block-cyclic
+// plan (chol_plan_dist) lives on device r; the ranks are connected in-process (plain
+// device pointers, cudaDeviceEnablePeerAccess -- NVLink peer memory), and every call
+// below fans out to them.  A, L may be host pointers or device pointers (UVA copies).
+static int factor_launch(chol_plan_s* p);
+static int finish_info(chol_plan_s* p, int* info);
+
+static int plan_multi(int64_t n, int64_t nb, int ngpus, const chol_opts_t& opts, chol_plan_t* out) {
+  int dev0 = 0, ndev = 0;
+  CUDA_TRY(cudaGetDevice(&dev0));
+  CUDA_TRY(cudaGetDeviceCount(&ndev));
+  const char* e1d = getenv("CHOL_MULTI_ONE_DEVICE");
+  const bool one_dev = e1d && e1d[0] == '1';
+  auto* m = new (std::nothrow) chol_plan_s();
+  if (!m) return -9;
+  m->n = n;
+  m->nb = nb;
+  m->N = n / nb;
+  m->ntiles = m->N * (m->N + 1) / 2;
+  m->ntasks = n_tasks(m->N);
+  m->bs = pick_block(nb);
+  m->opts = opts;
+  m->ngpus = m->nranks = ngpus;
+  m->device = dev0;
+  m->p = opts.grid_p;
+  m->q = opts.grid_q;
+  chol_opts_t so = opts;
+  if (one_dev && so.workers == 0) {
+    int sms = 0;
+    cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev0);
+    so.workers = std::max(1, sms / ngpus);
+  }
+  auto fail = [&](int st) {
+    cudaSetDevice(dev0);
+    if (m->subs.empty())
+      delete m;
+    else
+      chol_destroy(m);
+    return st;
+  };
+  for (int r = 0; r < ngpus; ++r) {
+    if (cudaSetDevice(one_dev ? dev0 : r % ndev)) return fail(-3);
+    chol_plan_t sp = nullptr;
+    const int st = chol_plan_dist(n, nb, ngpus, r, &so, &sp);
+    if (st) return fail(st);
+    m->subs.push_back(sp);
+  }
+  constexpr int64_t kStride = 4096;
+  const size_t nr = ngpus > 0 ? (size_t)ngpus : 1;
+  std::vector<char> blobs(nr * (size_t)kStride, 0);
+  for (int r = 0; r < ngpus; ++r) {
+    int64_t len = 0;
+    int st = chol_dist_export(m->subs[r], nullptr, 0, &len);
+    if (st || len > kStride) return fail(st ? st : -8);
+    if ((st = chol_dist_export(m->subs[r], blobs.data() + r * kStride, kStride, &len))) return fail(st);
+  }
+  for (int r = 0; r < ngpus; ++r) {
+    const int st = chol_dist_connect(m->subs[r], blobs.data(), kStride);
+    if (st) return fail(st);
+  }
+  cudaSetDevice(dev0);
+  *out = m;
+  return 0;
+}
+
+static int multi_launch(chol_plan_s* m) {
+  for (chol_plan_s* sp : m->subs) {
+    cudaSetDevice(sp->device);
+    const int st = factor_launch(sp);
+    if (st) return st;
+  }
+  return 0;
+}
+static int multi_finish(chol_plan_s* m, int* info) {
+  int best = 0, launches = 0;
+  double t = 0.0;
+  for (chol_plan_s* sp : m->subs) {
+    cudaSetDevice(sp->device);
+    int i = 0;
+    const int st = finish_info(sp, &i);
+    if (st) return st;
+    if (i && (!best || i < best)) best = i;
+    t = std::max(t, sp->last_factor_s);
+    launches += sp->last_launches;
+  }
+  cudaSetDevice(m->device);
+  m->last_factor_s = t;
+  m->last_launches = launches;
+  m->factored = true;
+  m->last_info = best;
+  if (info) *info = best;
+  return 0;
+}
+
 extern "C" int chol_get_stream(chol_plan_t p, void** stream) {
   if (!p || !stream) return -4;
+  if (is_multi(p)) p = p->subs[0];
   *stream = (void*)p->stream;
   return 0;
 }
@@ -435,7 +551,10 @@ extern "C" int chol_get_info(chol_plan_t p, int64_t* n, int64_t* nb, int* block,
   if (n) *n = p->n;
   if (nb) *nb = p->nb;
   if (block) *block = p->bs;
-  if (workers) *workers = p->sched ? sched_workers(p->sched) : 0;
+  if (workers) {
+    *workers = p->sched ? sched_workers(p->sched) : 0;
+    for (chol_plan_s* sp : p->subs) *workers += sp->sched ? sched_workers(sp->sched) : 0;
+  }
   if (policy) *policy = p->opts.policy;
   if (executor) *executor = p->opts.executor;
   return 0;
@@ -513,6 +632,12 @@ static int gather_impl(chol_plan_s* p, double* L, int64_t ldl) {
 extern "C" int chol_scatter(chol_plan_t p, const double* A, int64_t lda) {
   if (!p || !A || (reinterpret_cast<uintptr_t>(A) & 7)) return -4;
   if (lda < p->n) return -5;
+  if (is_multi(p)) {
+    for (chol_plan_s* sp : p->subs)
+      if (const int st = chol_scatter(sp, A, lda)) return st;
+    cudaSetDevice(p->device);
+    return 0;
+  }
   cudaSetDevice(p->device);
   int st = scatter_impl(p, A, lda);
   if (st) return st;
@@ -523,6 +648,12 @@ extern "C" int chol_scatter(chol_plan_t p, const double* A, int64_t lda) {
 extern "C" int chol_gather(chol_plan_t p, double* L, int64_t ldl) {
   if (!p || !L || (reinterpret_cast<uintptr_t>(L) & 7)) return -4;
   if (ldl < p->n) return -5;
+  if (is_multi(p)) {
+    for (chol_plan_s* sp : p->subs)
+      if (const int st = chol_gather(sp, L, ldl)) return st;
+    cudaSetDevice(p->device);
+    return 0;
+  }
   cudaSetDevice(p->device);
   int st = gather_impl(p, L, ldl);
   if (st) return st;
@@ -542,15 +673,23 @@ static int owned_tiles_copy(chol_plan_t p, void* dst, const void* src, int64_t c
   return 0;
 }
 extern "C" int chol_scatter_tiles(chol_plan_t p, const double* tiles, int64_t count) {
+  if (is_multi(p)) return -8;  // per-rank call: use the rank plans (chol_plan_dist)
   return p ? owned_tiles_copy(p, p->tiles, tiles, count) : -4;
 }
 extern "C" int chol_gather_tiles(chol_plan_t p, double* tiles, int64_t count) {
+  if (is_multi(p)) return -8;
   return p ? owned_tiles_copy(p, tiles, p->tiles, count) : -4;
 }
 
 extern "C" int chol_generate(chol_plan_t p, uint64_t seed, int family) {
   if (!p) return -4;
   if (family < 0 || family > 1) return -6;
+  if (is_multi(p)) {
+    for (chol_plan_s* sp : p->subs)
+      if (const int st = chol_generate(sp, seed, family)) return st;
+    cudaSetDevice(p->device);
+    return 0;
+  }
   cudaSetDevice(p->device);
   CUDA_TRY(launch_generate(p->tiles, p->n, (int)p->nb, (int)p->N, seed, family, p->stream,
                            p->dist ? p->d_owned_tile : nullptr, p->nowned));
@@ -630,18 +769,24 @@ static int finish_info(chol_plan_s* p, int* info) {
 
 extern "C" int chol_factor_async(chol_plan_t p) {
   if (!p) return -4;
+  if (is_multi(p)) return multi_launch(p);
   cudaSetDevice(p->device);
   return factor_launch(p);
 }
 
 extern "C" int chol_wait(chol_plan_t p, int* info) {
   if (!p) return -4;
+  if (is_multi(p)) return multi_finish(p, info);
   cudaSetDevice(p->device);
   return finish_info(p, info);
 }
 
 extern "C" int chol_factor_inplace(chol_plan_t p, int* info) {
   if (!p) return -4;
+  if (is_multi(p)) {
+    const int st = multi_launch(p);
+    return st ? st : multi_finish(p, info);
+  }
   cudaSetDevice(p->device);
   int st = factor_launch(p);
   if (st) return st;
@@ -746,6 +891,15 @@ static int factor_streamed(chol_plan_s* p, const double* A, int64_t lda, double*
 extern "C" int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* L, int64_t ldl, int* info) {
   if (!p || !A || !L || (reinterpret_cast<uintptr_t>(A) & 7) || (reinterpret_cast<uintptr_t>(L) & 7)) return -4;
   if (lda < p->n || ldl < p->n) return -5;
+  if (is_multi(p)) {  // owners pull their tiles of A, factor together, write their tiles of L
+    const auto t0 = std::chrono::steady_clock::now();
+    int st = chol_scatter(p, A, lda);
+    if (!st) st = chol_factor_inplace(p, info);
+    if (!st) st = chol_gather(p, L, ldl);
+    const double tot = std::chrono::duration<double>(std::chrono::steady_clock::now() - t0).count();
+    p->last_layout_s = tot - p->last_factor_s;
+    return st;
+  }
   cudaSetDevice(p->device);
   if (!p->dist && p->sched && !is_device_ptr(A) && !is_device_ptr(L)) return factor_streamed(p, A, lda, L, ldl, info);
   CUDA_TRY(cudaEventRecord(p->ev2, p->stream));
@@ -780,6 +934,7 @@ extern "C" int chol_last_times(chol_plan_t p, double* factor_s, double* layout_s
 // solved by the forward and backward sweeps, and copied back.
 extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   if (!p || !B || (reinterpret_cast<uintptr_t>(B) & 7)) return -4;
+  if (is_multi(p)) return -8;
   if (nrhs < 1) return -6;
   if (ldb < nrhs) return -5;
   if (p->dist) return -8;
@@ -877,6 +1032,59 @@ extern "C" int chol_last_solve_times(chol_plan_t p, double* total_s, double* swe
 extern "C" int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int64_t* nrecs, double* makespan_s) {
   if (!p) return -4;
   if (!p->opts.trace || !p->factored) return -7;
+  if (is_multi(p)) {
+    // every rank records the tasks it ran, relative to its own launch stamp (globaltimer,
+    // one clock per device): shift to absolute, merge by task, emit in Algorithm 1 order
+    const int64_t N = p->N;
+    std::vector<chol_task_rec_t> all(p->ntasks);
+    std::vector<char> have(p->ntasks, 0);
+    std::vector<chol_task_rec_t> part(p->ntasks);
+    uint64_t lo = UINT64_MAX, hi = 0;
+    for (chol_plan_s* sp : p->subs) {
+      int64_t nr = 0;
+      double ms = 0.0;
+      int st = chol_trace(sp, part.data(), (int64_t)part.size(), &nr, &ms);
+      if (st) return st;
+      uint64_t base = 0;
+      cudaSetDevice(sp->device);
+      CUDA_TRY(cudaMemcpy(&base, sp->d_base, sizeof(base), cudaMemcpyDeviceToHost));
+      for (int64_t x = 0; x < nr; ++x) {
+        chol_task_rec_t r = part[x];
+        r.t0_ns += base;
+        r.t1_ns += base;
+        const int64_t id = r.type == T_POTRF ? id_potrf(N, r.k)
+                           : r.type == T_TRSM ? id_trsm(N, r.i, r.k)
+                           : r.type == T_SYRK ? id_syrk(N, r.j, r.k)
+                                              : id_gemm(N, r.i, r.j, r.k);
+        all[id] = r;
+        have[id] = 1;
+        lo = std::min(lo, r.t0_ns);
+        hi = std::max(hi, r.t1_ns);
+      }
+    }
+    cudaSetDevice(p->device);
+    int64_t w = 0;
+    auto emit = [&](int64_t id) {
+      if (!have[id]) return;
+      if (recs && w < cap) {
+        recs[w] = all[id];
+        recs[w].t0_ns -= lo;
+        recs[w].t1_ns -= lo;
+      }
+      ++w;
+    };
+    for (int k = 0; k < N; ++k) {
+      emit(id_potrf(N, k));
+      for (int i = k + 1; i < N; ++i) emit(id_trsm(N, i, k));
+      for (int j = k + 1; j < N; ++j) {
+        emit(id_syrk(N, j, k));
+        for (int i = j + 1; i < N; ++i) emit(id_gemm(N, i, j, k));
+      }
+    }
+    if (nrecs) *nrecs = w;
+    if (makespan_s) *makespan_s = (hi > lo) ? (hi - lo) * 1e-9 : 0.0;
+    return 0;
+  }
   cudaSetDevice(p->device);
   std::vector<uint64_t> t0(p->ntasks), t1(p->ntasks);
   CUDA_TRY(cudaMemcpy(t0.data(), p->d_t0, p->ntasks * 8, cudaMemcpyDeviceToHost));
@@ -920,6 +1128,7 @@ extern "C" int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int
 
 extern "C" int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t* njobs) {
   if (!p) return -4;
+  if (is_multi(p)) return -8;
   if (!p->sched || p->opts.trace != 2 || !p->factored) return -7;
   cudaSetDevice(p->device);
   return sched_job_trace(p->sched, out, cap, njobs);  // 5 u64 per job
@@ -928,6 +1137,7 @@ extern "C" int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t
 // ------------------------------------------------------------------ calibration / single tasks
 extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double* ms) {
   if (!p) return -4;
+  if (is_multi(p)) return -8;
   if (p->dist) return -8;
   const int N = (int)p->N;
   if (type < 0 || type > 3 || reps < 1 || k < 0 || k >= N) return -6;
@@ -965,6 +1175,7 @@ extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int r
 
 extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, double* ms) {
   if (!p) return -4;
+  if (is_multi(p)) return -8;
   if (p->dist) return -8;
   const int N = (int)p->N;
   if (type < 0 || type > 3 || reps < 1 || count < 1) return -6;

@@ -195,3 +195,39 @@ def test_scatter_gather_tiles_single_and_distributed():
         assert np.max(np.abs(out - want)) <= 1e-10 * np.max(np.abs(ref))
     for pl in plans:
         pl.close()
+
+
+@pytest.mark.parametrize("ngpus", [2, 4])
+def test_single_process_multi_device_plan(ngpus, monkeypatch):
+    """chol_plan(n, nb, ngpus > 1): one process drives ngpus ranks (here all on cuda:0 via
+    CHOL_MULTI_ONE_DEVICE=1, SMs / ngpus workers each); device and host pointers; the
+    factor equals the single-plan factor bit for bit (R15); the merged trace holds every
+    task once, from every rank; solve / per-rank calls are rejected (-8)."""
+    monkeypatch.setenv("CHOL_MULTI_ONE_DEVICE", "1")
+    c = _lib()
+    n, nb = 1920, 96
+    N = n // nb
+    A = spdgen.uniform_spd(n, 23)
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p1:
+        d1 = torch.from_numpy(A.copy()).cuda()
+        assert p1.factor(d1) == 0
+        ref = d1.cpu().numpy()
+    with c.Plan(n, nb, ngpus=ngpus, policy=1, trace=1) as p:
+        dA = torch.from_numpy(A.copy()).cuda()
+        assert p.factor(dA) == 0
+        L = dA.cpu().numpy()
+        recs, makespan = c.chol_trace(p.h)
+        Lh = np.full_like(A, np.nan)
+        assert c.chol_factor(p.h, A.copy(), n, Lh, n) == 0
+        with pytest.raises(c.CholError):
+            p.solve(np.ones(n))
+    assert np.array_equal(L, ref)
+    assert np.array_equal(Lh, ref)
+    assert len(recs) == N * (N + 1) * (N + 2) // 6
+    assert {r["gpu"] for r in recs} == set(range(ngpus))
+    assert makespan > 0
+    # non-SPD input: LAPACK info from the owning rank
+    L0 = spdgen.integer_L0(n, 6)
+    B = spdgen.make_non_spd(spdgen.integer_spd(n, 6), L0, 700, "zero")
+    with c.Plan(n, nb, ngpus=ngpus) as p:
+        assert p.factor(torch.from_numpy(B).cuda()) == 701
