@@ -369,6 +369,21 @@ def run_dist(args, ws, rank, local):
     }
     if SHARED_GPU:
         line["note"] = "BENCH_SHARED_GPU=1: all ranks on cuda:0 (multi-process path check, not a scaling number)"
+    if rank == 0 and not args.no_bounds and not SHARED_GPU:
+        # the paper's bounds for M = ws GPUs from one GPU's calibrated task times, plus the
+        # owner-area bound of the block-cyclic grid (SURVEY §8c ext)
+        try:
+            import types
+            a1 = types.SimpleNamespace(n=n, nb=nb, policy=args.policy, seed=args.seed)
+            T_lat, T_thr = calibrate(c, a1, torch.cuda.get_device_properties(local).multi_processor_count)
+            b = c.chol_bounds(n, nb, ws, T_lat, T_thr)
+            b["owner_area"] = c.chol_owner_area(n // nb, p, q, T_thr)[0]
+            line["bounds"] = {"seconds": b, "upper_tflops": {k: flops / v / 1e12 for k, v in b.items() if v > 0},
+                              "makespan_over_mixed": t_step / b["mixed"],
+                              "makespan_over_owner_area": t_step / b["owner_area"],
+                              "calibration": "T_thr / T_lat of one GPU (rank 0, same n), M = n_gpus"}
+        except Exception as ex:
+            line["bounds"] = {"unavailable": f"{type(ex).__name__}: {ex}"[:200]}
     if e2e is not None:
         line["e2e"] = e2e
     if rank == 0:

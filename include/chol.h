@@ -251,6 +251,13 @@ int chol_task_id(int64_t N, int type, int i, int j, int k, int64_t* id);
  * out[4] GEMM-peak bound (n^3/3) / (M 2 nb^3 / T_thr_G), out[5] max(area, cp). */
 int chol_bounds(int64_t n, int64_t nb, int ngpus, const double* T_lat, const double* T_thr, double* out);
 
+/* Owner-area bound (ext; host only): on a p x q 2D block-cyclic grid with
+ * owner-computes every task runs on the owner of the tile it overwrites, so
+ * no schedule beats the busiest rank: *out = max_g sum_{tasks of g} T_thr[type] (seconds,
+ * T_thr as in chol_bounds).  per_rank (may be NULL) receives the p*q sums.  Errors: -1
+ * N <= 0, -3 p or q < 1, -4 null pointer. */
+int chol_owner_area(int64_t N, int p, int q, const double* T_thr, double* out, double* per_rank);
+
 /* ---- platform model (host only): the paper's LP bounds over several resource types and
  * its scheduler simulation (§III-A, §IV-C, §V;
  * SURVEY §8f NEXT-1).  Times are per task of each type on one processing element of a

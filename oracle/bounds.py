@@ -98,3 +98,14 @@ def lp_area_mixed(N: int, T: dict[str, dict[str, float]], M: dict[str, int],
                   bounds=[(0, None)] * nv, method="highs")
     assert sol.status == 0, sol.message
     return float(sol.x[-1])
+
+
+def owner_area(N: int, p: int, q: int, T_thr: dict[str, float]) -> tuple[float, list[float]]:
+    """Owner-area bound (ext): every task of the brute-force task list runs on
+    the owner (i mod p, j mod q) of the tile it writes (owner-computes, L263-274); the
+    busiest rank's summed T_thr bounds any schedule on that grid."""
+    w = [0.0] * (p * q)
+    for t in dag.tasks(N):
+        i, j = t.writes
+        w[(i % p) * q + (j % q)] += T_thr[dag.TYPE_NAMES[t.type]]
+    return max(w), w

@@ -64,6 +64,7 @@ def _load():
         "chol_generate": ([P, u64, i32], i32),
         "chol_scatter": ([P, vp, i64], i32),
         "chol_gather": ([P, vp, i64], i32),
+        "chol_owner_area": ([i64, i32, i32, dp, dp, dp], i32),
         "chol_scatter_tiles": ([P, vp, i64], i32),
         "chol_gather_tiles": ([P, vp, i64], i32),
         "chol_factor_inplace": ([P, ctypes.POINTER(i32)], i32),
@@ -106,7 +107,7 @@ EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_dest
             "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
             "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
             "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times", "chol_scatter_tiles",
-            "chol_gather_tiles")
+            "chol_gather_tiles", "chol_owner_area")
 
 
 def _ptr(x) -> int:
@@ -277,6 +278,16 @@ def chol_last_solve_times(plan: int) -> tuple[float, float]:
     a, b = ctypes.c_double(), ctypes.c_double()
     _check(_lib.chol_last_solve_times(plan, ctypes.byref(a), ctypes.byref(b)), "chol_last_solve_times")
     return a.value, b.value
+
+
+def chol_owner_area(N: int, p: int, q: int, T_thr) -> tuple[float, list]:
+    """Owner-area bound on a p x q block-cyclic grid: (max over ranks, per-rank sums)."""
+    tt = (ctypes.c_double * 4)(*[T_thr[k] for k in ("POTRF", "TRSM", "SYRK", "GEMM")]) \
+        if isinstance(T_thr, dict) else (ctypes.c_double * 4)(*T_thr)
+    out = ctypes.c_double()
+    per = (ctypes.c_double * (p * q))()
+    _check(_lib.chol_owner_area(N, p, q, tt, ctypes.byref(out), per), "chol_owner_area")
+    return out.value, list(per)
 
 
 def chol_lp_bound(N: int, workers, times, mixed: bool = True):

@@ -191,3 +191,25 @@ extern "C" int chol_bounds(int64_t n, int64_t nb, int ngpus, const double* T_lat
   out[5] = std::max(area, cp);
   return 0;
 }
+
+// Owner-area bound (ext): under the fixed 2D block-cyclic owner-computes
+// placement no schedule beats the busiest rank's own work,
+// max_g sum_{tasks owned by g} T_thr(type); the task owner is the owner of the tile it
+// overwrites (POTRF_k -> (k,k), TRSM_i_k -> (i,k), SYRK_j_k -> (j,j), GEMM_i_j_k -> (i,j)).
+extern "C" int chol_owner_area(int64_t N, int p, int q, const double* T_thr, double* out, double* per_rank) {
+  if (N <= 0) return -1;
+  if (p < 1 || q < 1) return -3;
+  if (!T_thr || !out) return -4;
+  std::vector<double> w((size_t)p * q, 0.0);
+  for (int64_t k = 0; k < N; ++k) {
+    w[tile_owner_h(k, k, p, q)] += T_thr[0];
+    for (int64_t i = k + 1; i < N; ++i) w[tile_owner_h(i, k, p, q)] += T_thr[1];
+    for (int64_t j = k + 1; j < N; ++j) {
+      w[tile_owner_h(j, j, p, q)] += T_thr[2];
+      for (int64_t i = j + 1; i < N; ++i) w[tile_owner_h(i, j, p, q)] += T_thr[3];
+    }
+  }
+  *out = *std::max_element(w.begin(), w.end());
+  if (per_rank) std::copy(w.begin(), w.end(), per_rank);
+  return 0;
+}

@@ -70,3 +70,13 @@ def test_bounds_match_oracle(chol):
         ref = obounds.all_bounds(n, nb, dict(zip(keys, T_thr)), dict(zip(keys, T_lat)), M)
         for k in ("area", "chain", "mixed", "critical_path", "gemm_peak"):
             assert abs(got[k] - ref[k]) <= 1e-12 * max(1.0, abs(ref[k])), (k, got[k], ref[k])
+
+
+def test_owner_area_matches_oracle(chol):
+    keys = ["POTRF", "TRSM", "SYRK", "GEMM"]
+    T_thr = [1.2e-4, 1.1e-4, 3.6e-5, 5.7e-5]
+    for N, p, q in [(1, 1, 1), (7, 1, 2), (20, 2, 2), (25, 1, 2), (40, 2, 4), (48, 4, 2), (13, 3, 3)]:
+        mx, per = chol.chol_owner_area(N, p, q, T_thr)
+        rmx, rper = obounds.owner_area(N, p, q, dict(zip(keys, T_thr)))
+        assert abs(mx - rmx) <= 1e-12 * rmx
+        assert all(abs(a - b) <= 1e-12 * max(b, 1e-30) for a, b in zip(per, rper))

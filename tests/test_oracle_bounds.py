@@ -46,3 +46,23 @@ def test_gemm_peak():
     # R_G = 2 nb^3 / T_G; bound = (n^3/3) / (M R_G)
     n, nb = 9600, 960
     assert abs(bounds.gemm_peak(n, nb, 2.0, 1) - (n ** 3 / 3) / (2 * nb ** 3 / 2.0)) < 1e-9
+
+
+def test_owner_area_pins():
+    """Owner-area bound (SURVEY §8c ext): one rank = the area bound; the ranks' sums add up
+    to the total work; with flop weights the max/mean imbalance is SURVEY §8e's table
+    (2x4 / 4x2 / 1x8 at N = 48: 1.035 / 1.095 / 1.013; N = 96: 1.016 / 1.047 / 1.003)."""
+    T = {"POTRF": 0.7, "TRSM": 1.9, "SYRK": 1.3, "GEMM": 2.6}
+    for N in (1, 2, 5, 9):
+        mx, w = bounds.owner_area(N, 1, 1, T)
+        assert mx == pytest.approx(bounds.area(N, T, 1))
+        for p, q in ((1, 2), (2, 2), (2, 3)):
+            mx, w = bounds.owner_area(N, p, q, T)
+            assert sum(w) == pytest.approx(bounds.area(N, T, 1))
+            assert mx >= bounds.area(N, T, p * q) - 1e-12
+    flops = {"POTRF": 1 / 3, "TRSM": 1.0, "SYRK": 1.0, "GEMM": 2.0}
+    want = {(48, 2, 4): 1.035, (48, 4, 2): 1.095, (48, 1, 8): 1.013,
+            (96, 2, 4): 1.016, (96, 4, 2): 1.047, (96, 1, 8): 1.003}
+    for (N, p, q), v in want.items():
+        mx, w = bounds.owner_area(N, p, q, flops)
+        assert round(mx / (sum(w) / len(w)), 3) == v
