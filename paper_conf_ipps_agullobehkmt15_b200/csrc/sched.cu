@@ -17,6 +17,7 @@
 // (the paper's TRSM-distance rule, L1019-1025).
 #include <algorithm>
 #include <climits>
+#include <cstdio>
 #include <cstdlib>
 #include <cstring>
 #include <vector>
@@ -1105,7 +1106,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // L655-660; reading R13) with latency-estimate weights, quantised into kBuckets;
   // POTRF's inner nodes inherit the POTRF priority.
   const int nnodes = (int)B.deps.size();
-  const double w_type[4] = {300.0, 300.0, 80.0, 80.0};
+  double w_type[4] = {300.0, 300.0, 80.0, 80.0};
+  if (const char* ew = getenv("CHOL_PRIO_W"))  // development switch: "p,t,s,g" (us)
+    sscanf(ew, "%lf,%lf,%lf,%lf", &w_type[0], &w_type[1], &w_type[2], &w_type[3]);
   const std::vector<double> bl = bottom_levels(N, w_type);
   const double blmax = *std::max_element(bl.begin(), bl.end()) + 1e-9;
   std::vector<int> node_queue(nnodes, 0);
