@@ -23,11 +23,15 @@
  *   -5  lda / ldl < n
  *   -6  bad options (unknown policy / executor / negative values)
  *   -7  chol_trace before any chol_factor*, or tracing disabled
- *   -8  operation not supported by this build (e.g. ngpus > 1 in one process)
+ *   -8  operation not supported for this plan (e.g. chol_solve on a multi-GPU plan)
  *   -9  device out of memory while planning
  *   -10 chol_solve without a successful factorization in the plan
+ *   -11 watchdog: the persistent scheduler completed no task node for CHOL_WATCHDOG_S
+ *       seconds (env, default 60, 0 = off) -- e.g. a rank of a distributed plan whose
+ *       peer never launched; the run is aborted (the kernel exits) and the factor is
+ *       incomplete
  *   -100 - e   CUDA runtime error e
- *   -200 - e   NCCL error e
+ *   (no NCCL codes: the multi-GPU exchange is peer memory, not NCCL)
  * A non-SPD input is NOT an error status: it is reported through *info.
  *
  * Thread safety: a plan may be used by one host thread at a time.

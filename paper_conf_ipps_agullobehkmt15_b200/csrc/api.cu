@@ -118,6 +118,7 @@ extern "C" const char* chol_strerror(int s) {
     case -8: return "not supported by this build";
     case -9: return "device out of memory";
     case -10: return "no successful factorization in the plan";
+    case -11: return "scheduler made no progress within CHOL_WATCHDOG_S seconds (run aborted)";
   }
   if (s <= -200) return "NCCL error";
   if (s <= -100) return cudaGetErrorString((cudaError_t)(-100 - s));
@@ -753,8 +754,64 @@ static int factor_launch(chol_plan_s* p) {
   return 0;
 }
 
+// Wait for the plan's stream.  With the persistent scheduler, a host watchdog reads the
+// device's completed-node counter every 0.25 s: no progress for CHOL_WATCHDOG_S seconds
+// (default 60, 0 = off) aborts the run (sched_abort: the scheduler warps stop handing out
+// jobs, the kernel exits) and returns -11 -- a stalled scheduler (a rank that never
+// launched, a lost peer flag) is reported instead of hanging the caller.
+static int wait_plan(chol_plan_s* p) {
+  const char* ew = getenv("CHOL_WATCHDOG_S");
+  const double limit = ew ? atof(ew) : 60.0;
+  const int* prog = p->sched ? sched_progress(p->sched) : nullptr;
+  if (!prog || limit <= 0) {
+    CUDA_TRY(cudaStreamSynchronize(p->stream));
+    return 0;
+  }
+  using clk = std::chrono::steady_clock;
+  cudaStream_t ws = nullptr;
+  int* h = nullptr;
+  int last = -1, st = 0;
+  auto t_prog = clk::now(), t_check = clk::now();
+  while (true) {
+    const cudaError_t q = cudaStreamQuery(p->stream);
+    if (q == cudaSuccess) break;
+    if (q != cudaErrorNotReady) {
+      st = -100 - (int)q;
+      break;
+    }
+    const auto now = clk::now();
+    if (std::chrono::duration<double>(now - t_check).count() >= 0.25) {
+      t_check = now;
+      if (!ws) {
+        if (cudaStreamCreateWithFlags(&ws, cudaStreamNonBlocking) || cudaHostAlloc(&h, sizeof(int), 0)) {
+          cudaGetLastError();
+          st = cudaStreamSynchronize(p->stream) ? -100 : 0;  // fall back to a plain wait
+          break;
+        }
+      }
+      cudaMemcpyAsync(h, prog, sizeof(int), cudaMemcpyDeviceToHost, ws);
+      cudaStreamSynchronize(ws);
+      if (*h != last) {
+        last = *h;
+        t_prog = now;
+      } else if (std::chrono::duration<double>(now - t_prog).count() > limit) {
+        sched_abort(p->sched);  // the kernel drains its running jobs and exits
+        cudaStreamSynchronize(p->stream);
+        cudaGetLastError();
+        st = -11;
+        break;
+      }
+    }
+    std::this_thread::yield();
+  }
+  if (ws) cudaStreamDestroy(ws);
+  if (h) cudaFreeHost(h);
+  return st;
+}
+
 static int finish_info(chol_plan_s* p, int* info) {
   int h = 0;
+  if (const int w = wait_plan(p)) return w;
   CUDA_TRY(cudaMemcpyAsync(&h, p->d_info, sizeof(int), cudaMemcpyDeviceToHost, p->stream));
   CUDA_TRY(cudaStreamSynchronize(p->stream));
   float ms = 0.f;

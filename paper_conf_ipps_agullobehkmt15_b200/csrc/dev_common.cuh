@@ -88,11 +88,14 @@ __device__ __forceinline__ double2 lds128(uint32_t addr) {
 }
 
 // ---------------------------------------------------------------- named barriers
+// Non-.aligned forms (barrier.sync / barrier.arrive): the warps meeting at a named barrier
+// execute it at different program points (e.g. potf2's factor warp and its row warps),
+// which bar.sync (= barrier.sync.aligned) does not allow (compute-sanitizer synccheck).
 __device__ __forceinline__ void bar_arrive(uint32_t id, uint32_t nthreads) {
-  asm volatile("bar.arrive %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
+  asm volatile("barrier.arrive %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
 }
 __device__ __forceinline__ void bar_sync(uint32_t id, uint32_t nthreads) {
-  asm volatile("bar.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
+  asm volatile("barrier.sync %0, %1;" ::"r"(id), "r"(nthreads) : "memory");
 }
 
 // ---------------------------------------------------------------- DMMA

@@ -62,6 +62,7 @@ struct DevSched {
   int* q_tail;             // kQueues * kQStride
   int* done_nodes;
   int* finished;
+  const int* abort_flag;   // device word set by the host watchdog (api.cu) to stop a stalled run
   uint64_t* job_trace;     // trace == 2: per job {t0, t1, worker << 32 | smid, t_enqueue}
   const uint64_t* tr_base; // globaltimer at factorization start (trace only)
   int total_nodes;
@@ -344,7 +345,7 @@ __device__ void watcher_loop(const DevSched& d) {
   const int lane = threadIdx.x & 31;
   int w0 = 0;
   unsigned backoff = 64;
-  while (w0 < d.nwatch) {
+  while (w0 < d.nwatch && !ld_volatile(d.abort_flag)) {
     bool fired_any = false;
 #pragma unroll
     for (int h = 0; h < 2; ++h) {
@@ -538,7 +539,7 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
       }
     }
     // 3. done?
-    if (q_done == q_issue && ld_volatile(d.finished)) {
+    if (q_done == q_issue && (ld_volatile(d.finished) || ld_volatile(d.abort_flag))) {
       if (lane == 0) {
         const int e = q_issue & 1;
         c.jdesc()[e * 3] = make_int4(-1, 0, 0, 0);
@@ -592,6 +593,7 @@ struct SchedState {
   int* roots = nullptr;
   int nrecv_jobs = 0;
   uint64_t* job_trace = nullptr;           // device, 4 per job (trace == 2)
+  int* d_abort = nullptr;                  // device abort flag (d.abort_flag), written by sched_abort
   std::vector<int16_t> h_job_type;         // host copies for chol_job_trace
   std::vector<int> h_job_paper;
 };
@@ -1268,6 +1270,16 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   st->workers = opts->workers > 0 ? std::min(opts->workers, sms * per_sm) : sms;
   if (d.latency_workers >= st->workers) d.latency_workers = std::max(1, st->workers / 4);
   (void)s;
+  {
+    // device memory, not host-mapped: the scheduler warps read it whenever they idle
+    cudaError_t ea = cudaMalloc(&st->d_abort, sizeof(int));
+    if (!ea) ea = cudaMemset(st->d_abort, 0, sizeof(int));
+    if (ea) {
+      sched_destroy(st);
+      return -100 - (int)ea;
+    }
+    st->d.abort_flag = st->d_abort;
+  }
   *out = st;
   return 0;
 }
@@ -1286,6 +1298,7 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
               unsigned epoch) {
   st->d.epoch = epoch;
   cudaError_t e;
+  if ((e = cudaMemsetAsync(st->d_abort, 0, sizeof(int), s))) return -100 - (int)e;
   if ((e = cudaMemcpyAsync(st->dev_dynamic, st->dev_pristine, st->pristine_bytes, cudaMemcpyDeviceToDevice, s)))
     return -100 - (int)e;
   if ((e = cudaMemsetAsync(static_cast<char*>(st->dev_dynamic) + st->pristine_bytes, 0,
@@ -1307,6 +1320,17 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
 }
 
 int sched_workers(const SchedState* st) { return st ? st->workers : 0; }
+const int* sched_progress(const SchedState* st) { return st ? st->d.done_nodes : nullptr; }
+void sched_abort(SchedState* st) {
+  // from the host, while the kernel runs: a copy on a stream of its own
+  if (!st || !st->d_abort) return;
+  static const int one = 1;
+  cudaStream_t s = nullptr;
+  if (cudaStreamCreateWithFlags(&s, cudaStreamNonBlocking)) return;
+  cudaMemcpyAsync(st->d_abort, &one, sizeof(int), cudaMemcpyHostToDevice, s);
+  cudaStreamSynchronize(s);
+  cudaStreamDestroy(s);
+}
 
 int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* njobs) {
   if (njobs) *njobs = st->njobs;
@@ -1331,6 +1355,7 @@ void sched_destroy(SchedState* st) {
   cudaFree(st->dev_dynamic);
   cudaFree(st->dev_pristine);
   cudaFree(st->job_trace);
+  cudaFree(st->d_abort);
   delete st;
 }
 

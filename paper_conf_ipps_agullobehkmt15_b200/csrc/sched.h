@@ -27,6 +27,10 @@ int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slo
 int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cudaStream_t s, int* nlaunch,
               unsigned epoch = 1);
 int sched_workers(const SchedState* st);
+// device counter of completed nodes (host watchdog, api.cu)
+const int* sched_progress(const SchedState* st);
+// stop a stalled run: the scheduler warps hand out no further jobs and the kernel exits
+void sched_abort(SchedState* st);
 // Streamed input (chol_factor from host memory): the order in which the tiles are copied
 // in, which the scheduler's watch list follows (fixed when the plan is built).
 void sched_arrival_order(const SchedState* st, std::vector<std::pair<int, int>>& tiles);

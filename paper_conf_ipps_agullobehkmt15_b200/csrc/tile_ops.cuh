@@ -716,6 +716,7 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
       POTF2_STAMP(5);
       if (c.lane == 0) factor_8x8(dd, rdv, info, col0 + 8 * p);
       POTF2_STAMP(6);
+      __syncwarp();  // bar.sync is .aligned: the warp reconverges after lane 0's factor first
       bar_sync(kBarCompute, kComputeThreads);  // L_pp published
       bar_sync(kBarCompute, kComputeThreads);  // panel p published
     }

@@ -231,3 +231,16 @@ def test_single_process_multi_device_plan(ngpus, monkeypatch):
     B = spdgen.make_non_spd(spdgen.integer_spd(n, 6), L0, 700, "zero")
     with c.Plan(n, nb, ngpus=ngpus) as p:
         assert p.factor(torch.from_numpy(B).cuda()) == 701
+
+
+def test_watchdog_reports_a_stalled_scheduler():
+    """SURVEY §5 failure detection: a distributed rank whose peer never launches would spin
+    forever; the host watchdog returns -11 after CHOL_WATCHDOG_S seconds (subprocess: the
+    stalled kernel dies with its process)."""
+    import os
+    import subprocess
+    import sys
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    r = subprocess.run([sys.executable, os.path.join(root, "tools", "watchdog_check.py")], capture_output=True,
+                       text=True, timeout=240)
+    assert "watchdog status -11" in r.stdout, (r.stdout[-1000:], r.stderr[-2000:])
