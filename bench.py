@@ -486,6 +486,10 @@ def run_ours(args, ws, rank, local):
         "roofline": roofline,
         "clocks": clocks,
         "gpu_launches": launches,
+        # the paper reports mean +- std of its runs; the best run beside it
+        "step_ms_stats": {"mean": 1e3 * statistics.mean(times),
+                          "std": 1e3 * (statistics.stdev(times) if len(times) > 1 else 0.0),
+                          "best": 1e3 * min(times), "runs": len(times)},
     }
 
     # end-to-end: the C-ABI with HOST buffers (pinned), copies inside the timed region
