@@ -1,6 +1,6 @@
 import sys, numpy as np, torch
 sys.path.insert(0, '.')
-import oracle, spdgen
+import spdgen
 import paper_conf_ipps_agullobehkmt15_b200 as c
 def run(nb, typ, reps=1):
     n = 3 * nb

@@ -4,7 +4,6 @@ import os, sys
 sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import numpy as np
 import torch
-import oracle
 import spdgen
 import paper_conf_ipps_agullobehkmt15_b200 as c
 
@@ -20,8 +19,8 @@ for n, nb, pol in [(1920, 96, 1), (960, 96, 2), (3840, 960, 0)]:
         p.solve(X)
         X1 = B[:, :1].copy()
         p.solve(X1)
-    ref, _ = oracle.chol_tiled(A, nb)
-    d = oracle.rel_diff(L, ref)
-    print(n, nb, pol, "max_rel", d["max_rel_floored"], flush=True)
-    assert d["max_rel_floored"] <= 1e-10
+    ref = np.linalg.cholesky(A)  # LAPACK; the oracle is test infrastructure only
+    rel = float(np.max(np.abs(L - ref)) / np.max(np.abs(ref)))
+    print(n, nb, pol, "max_rel", rel, flush=True)
+    assert rel <= 1e-10
 print("sanitize run ok")
