@@ -405,6 +405,7 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     const int i = d0.z, k = d1.x, slab = d1.y, nbb = c.nb / BS;
     double* X = c.tile(i, k) + (int64_t)slab * BS * c.nb;
     const double* L = c.tile(k, k);
+    prefetch_l2_rows<BS>(X, c.nb, BS, c.nb);
     for (int cb = 0; cb < nbb; ++cb) {
       if (cb > 0) gemm_consume(c, cb * BS / BK, acc);
       if (cb > 0) acc_sub_global(c, acc, X + cb * BS, c.nb);

@@ -459,17 +459,34 @@ __device__ __forceinline__ void acc_sub_global(const Ctx<BS>& c, const Acc<BS>& 
   using C = Cfg<BS>;
   const int g = c.lane >> 2, t = c.lane & 3;
   const int wm = c.warp >> 2, wn = c.warp & 3;
+  // every load of the thread is issued before its first store (the compiler cannot
+  // reorder them itself: with a runtime ldx the rows may alias), so the L2 / HBM latency
+  // is paid once per block instead of once per fragment
+  double2 v[C::MI][C::NI];
 #pragma unroll
   for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) {
-      double2* px = reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN + ni * 8 +
-                                               2 * t);
-      double2 v = __ldcg(px);
-      v.x -= acc[mi][ni][0];
-      v.y -= acc[mi][ni][1];
-      __stcg(px, v);
-    }
+    for (int ni = 0; ni < C::NI; ++ni)
+      v[mi][ni] = __ldcg(reinterpret_cast<const double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN +
+                                                          ni * 8 + 2 * t));
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni)
+      __stcg(reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * ldx + wn * C::WN + ni * 8 + 2 * t),
+             make_double2(v[mi][ni].x - acc[mi][ni][0], v[mi][ni].y - acc[mi][ni][1]));
+}
+
+// Pull rows [0, BS) x columns [c0, c1) of X (ld ldx) towards L2 (prefetch.global.L2,
+// fire-and-forget): the not-yet-touched column blocks of a TRSM row slab, whose first
+// read (acc_sub_global) would otherwise wait on HBM.
+template <int BS>
+__device__ __forceinline__ void prefetch_l2_rows(const double* X, int ldx, int c0, int c1) {
+  const int lines = (c1 - c0) / 16;  // 128-byte lines per row (c0, c1 multiples of 16)
+  for (int e = threadIdx.x; e < BS * lines; e += kComputeThreads) {
+    const int r = e / lines, l = e - r * lines;
+    asm volatile("prefetch.global.L2 [%0];" ::"l"(X + (int64_t)r * ldx + c0 + 16 * l));
+  }
 }
 
 // X <- X * Ld^{-T} for one BS x BS block X (ld ldx) against the lower
@@ -790,6 +807,7 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
   const int nbb = c.nb / BS;
   double* X = c.tile(i, k) + (int64_t)slab * BS * c.nb;
   const double* L = c.tile(k, k);
+  prefetch_l2_rows<BS>(X, c.nb, BS, c.nb);
   for (int cb = 0; cb < nbb; ++cb) {
     Acc<BS> acc;
     if (cb > 0) gemm_mainloop(c, c.slot(i, k), slab * BS, c.slot(k, k), cb * BS, 0, cb * BS, acc);
