@@ -324,14 +324,22 @@ __device__ __forceinline__ void epi_sub_global(Ctx<BS>& c, const Acc<BS>& acc, d
   mbar_wait(c.cbar(), c.cphase);
   c.cphase ^= 1;
   const uint32_t cs = smem_u32(c.lbuf());
+  // all shared loads first (lds128 is volatile: it would otherwise wait behind each store)
+  double2 cv[C::MI][C::NI];
 #pragma unroll
   for (int mi = 0; mi < C::MI; ++mi)
 #pragma unroll
     for (int ni = 0; ni < C::NI; ++ni) {
       const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
       // box cc/16, row r, logical 16-byte chunk (cc%16)/2, 128B swizzle
-      const uint32_t addr = cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4);
-      double2 v = lds128(addr);
+      cv[mi][ni] = lds128(cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4));
+    }
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
+      double2 v = cv[mi][ni];
       v.x -= acc[mi][ni][0];
       v.y -= acc[mi][ni][1];
       double2* p = reinterpret_cast<double2*>(Cblk + (int64_t)r * ldc + cc);
