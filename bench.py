@@ -35,7 +35,7 @@ sys.path.insert(0, ROOT)
 
 METRIC = "Cholesky FP64 TFLOP/s (n^3/3 / t)"
 FP64_PEAK_TFLOPS = 37.1  # measured DMMA peak, profiles/r01/fp64_peak_microbench.jsonl
-POLICIES = {"dynamic": 0, "cp": 1, "static": 2}
+POLICIES = {"cp": 0, "dynamic": 1, "static": 2}  # CHOL_POLICY_* (include/chol.h)
 
 
 def parse():

@@ -13,7 +13,7 @@ import os
 _HERE = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.environ.get("CHOL_LIB_OVERRIDE") or os.path.join(_HERE, "libchol_b200.so")  # override: A/B experiments only
 
-POLICY_DYNAMIC, POLICY_CP_PRIORITY, POLICY_STATIC = 0, 1, 2
+POLICY_CP_PRIORITY, POLICY_DYNAMIC, POLICY_STATIC = 0, 1, 2  # zero-initialised opts = CP_PRIORITY
 EXEC_SCHEDULER, EXEC_HOST = 0, 1
 POTRF, TRSM, SYRK, GEMM = 0, 1, 2, 3
 TYPE_NAMES = ("POTRF", "TRSM", "SYRK", "GEMM")

@@ -75,6 +75,7 @@ struct chol_plan_s {
   std::vector<chol_plan_s*> subs;
 };
 static bool is_multi(const chol_plan_s* p) { return p && !p->subs.empty(); }
+static void invalidate_factor(chol_plan_s* p);
 
 #define CUDA_TRY(x)                                   \
   do {                                                \
@@ -511,6 +512,7 @@ static int plan_multi(int64_t n, int64_t nb, int ngpus, const chol_opts_t& opts,
 }
 
 static int multi_launch(chol_plan_s* m) {
+  invalidate_factor(m);
   for (chol_plan_s* sp : m->subs) {
     cudaSetDevice(sp->device);
     const int st = factor_launch(sp);
@@ -518,19 +520,32 @@ static int multi_launch(chol_plan_s* m) {
   }
   return 0;
 }
+// On the first failing rank the others are aborted (they would spin on its publish flags
+// forever), every rank is still waited for, and the first error is returned.
 static int multi_finish(chol_plan_s* m, int* info) {
-  int best = 0, launches = 0;
+  int best = 0, launches = 0, first_err = 0;
   double t = 0.0;
   for (chol_plan_s* sp : m->subs) {
     cudaSetDevice(sp->device);
     int i = 0;
     const int st = finish_info(sp, &i);
-    if (st) return st;
+    if (st) {
+      if (!first_err) {
+        first_err = st;
+        for (chol_plan_s* o : m->subs)
+          if (o != sp && o->sched) {
+            cudaSetDevice(o->device);
+            sched_abort(o->sched);
+          }
+      }
+      continue;
+    }
     if (i && (!best || i < best)) best = i;
     t = std::max(t, sp->last_factor_s);
     launches += sp->last_launches;
   }
   cudaSetDevice(m->device);
+  if (first_err) return first_err;
   m->last_factor_s = t;
   m->last_launches = launches;
   m->factored = true;
@@ -640,6 +655,7 @@ extern "C" int chol_scatter(chol_plan_t p, const double* A, int64_t lda) {
     return 0;
   }
   cudaSetDevice(p->device);
+  invalidate_factor(p);
   int st = scatter_impl(p, A, lda);
   if (st) return st;
   CUDA_TRY(cudaStreamSynchronize(p->stream));
@@ -675,6 +691,7 @@ static int owned_tiles_copy(chol_plan_t p, void* dst, const void* src, int64_t c
 }
 extern "C" int chol_scatter_tiles(chol_plan_t p, const double* tiles, int64_t count) {
   if (is_multi(p)) return -8;  // per-rank call: use the rank plans (chol_plan_dist)
+  if (p) invalidate_factor(p);
   return p ? owned_tiles_copy(p, p->tiles, tiles, count) : -4;
 }
 extern "C" int chol_gather_tiles(chol_plan_t p, double* tiles, int64_t count) {
@@ -685,6 +702,7 @@ extern "C" int chol_gather_tiles(chol_plan_t p, double* tiles, int64_t count) {
 extern "C" int chol_generate(chol_plan_t p, uint64_t seed, int family) {
   if (!p) return -4;
   if (family < 0 || family > 1) return -6;
+  invalidate_factor(p);
   if (is_multi(p)) {
     for (chol_plan_s* sp : p->subs)
       if (const int st = chol_generate(sp, seed, family)) return st;
@@ -730,7 +748,19 @@ static int run_host_sequenced(chol_plan_s* p, int* nlaunch) {
   return 0;
 }
 
+// Every call that writes the tile store first forgets the previous factor: chol_solve
+// then refuses (-10) until a factorization completes with info = 0, and the cached
+// diagonal-block inverses are recomputed (a failed, aborted or overwritten factor is
+// never used).
+static void invalidate_factor(chol_plan_s* p) {
+  p->factored = false;
+  p->last_info = -1;
+  p->inv_valid = false;
+  for (chol_plan_s* sp : p->subs) invalidate_factor(sp);
+}
+
 static int factor_launch(chol_plan_s* p) {
+  invalidate_factor(p);
   CUDA_TRY(launch_init_info(p->d_info, p->stream));
   if (p->opts.trace) {
     CUDA_TRY(cudaMemsetAsync(p->d_t0, 0xff, p->ntasks * sizeof(uint64_t), p->stream));
@@ -754,59 +784,72 @@ static int factor_launch(chol_plan_s* p) {
   return 0;
 }
 
-// Wait for the plan's stream.  With the persistent scheduler, a host watchdog reads the
-// device's completed-node counter every 0.25 s: no progress for CHOL_WATCHDOG_S seconds
+// Host watchdog over the persistent scheduler (wait_plan, factor_streamed): it reads the
+// device's completed-node counter every 0.25 s; no progress for CHOL_WATCHDOG_S seconds
 // (default 60, 0 = off) aborts the run (sched_abort: the scheduler warps stop handing out
-// jobs, the kernel exits) and returns -11 -- a stalled scheduler (a rank that never
+// jobs, the kernel exits) and reports -11 -- a stalled scheduler (a rank that never
 // launched, a lost peer flag) is reported instead of hanging the caller.
+namespace {
+struct Watchdog {
+  using clk = std::chrono::steady_clock;
+  chol_plan_s* p;
+  double limit = 60.0;
+  const int* prog = nullptr;
+  cudaStream_t ws = nullptr;
+  int* h = nullptr;
+  int last = -1;
+  clk::time_point t_prog = clk::now(), t_check = clk::now();
+  explicit Watchdog(chol_plan_s* plan) : p(plan) {
+    const char* ew = getenv("CHOL_WATCHDOG_S");
+    if (ew) limit = atof(ew);
+    prog = p->sched ? sched_progress(p->sched) : nullptr;
+    if (prog && limit > 0 &&
+        (cudaStreamCreateWithFlags(&ws, cudaStreamNonBlocking) || cudaHostAlloc(&h, sizeof(int), 0))) {
+      cudaGetLastError();
+      prog = nullptr;  // no watchdog: plain waits
+    }
+  }
+  ~Watchdog() {
+    if (ws) cudaStreamDestroy(ws);
+    if (h) cudaFreeHost(h);
+  }
+  bool enabled() const { return prog && limit > 0; }
+  // 0 while the scheduler makes progress (or between checks); -11 once a stalled run was aborted
+  int check() {
+    if (!enabled()) return 0;
+    const auto now = clk::now();
+    if (std::chrono::duration<double>(now - t_check).count() < 0.25) return 0;
+    t_check = now;
+    cudaMemcpyAsync(h, prog, sizeof(int), cudaMemcpyDeviceToHost, ws);
+    cudaStreamSynchronize(ws);
+    if (*h != last) {
+      last = *h;
+      t_prog = now;
+      return 0;
+    }
+    if (std::chrono::duration<double>(now - t_prog).count() <= limit) return 0;
+    sched_abort(p->sched);  // the kernel drains its running jobs and exits
+    cudaStreamSynchronize(p->stream);
+    cudaGetLastError();
+    return -11;
+  }
+};
+}  // namespace
+
+// Wait for the plan's stream under the watchdog.
 static int wait_plan(chol_plan_s* p) {
-  const char* ew = getenv("CHOL_WATCHDOG_S");
-  const double limit = ew ? atof(ew) : 60.0;
-  const int* prog = p->sched ? sched_progress(p->sched) : nullptr;
-  if (!prog || limit <= 0) {
+  Watchdog wd(p);
+  if (!wd.enabled()) {
     CUDA_TRY(cudaStreamSynchronize(p->stream));
     return 0;
   }
-  using clk = std::chrono::steady_clock;
-  cudaStream_t ws = nullptr;
-  int* h = nullptr;
-  int last = -1, st = 0;
-  auto t_prog = clk::now(), t_check = clk::now();
   while (true) {
     const cudaError_t q = cudaStreamQuery(p->stream);
-    if (q == cudaSuccess) break;
-    if (q != cudaErrorNotReady) {
-      st = -100 - (int)q;
-      break;
-    }
-    const auto now = clk::now();
-    if (std::chrono::duration<double>(now - t_check).count() >= 0.25) {
-      t_check = now;
-      if (!ws) {
-        if (cudaStreamCreateWithFlags(&ws, cudaStreamNonBlocking) || cudaHostAlloc(&h, sizeof(int), 0)) {
-          cudaGetLastError();
-          st = cudaStreamSynchronize(p->stream) ? -100 : 0;  // fall back to a plain wait
-          break;
-        }
-      }
-      cudaMemcpyAsync(h, prog, sizeof(int), cudaMemcpyDeviceToHost, ws);
-      cudaStreamSynchronize(ws);
-      if (*h != last) {
-        last = *h;
-        t_prog = now;
-      } else if (std::chrono::duration<double>(now - t_prog).count() > limit) {
-        sched_abort(p->sched);  // the kernel drains its running jobs and exits
-        cudaStreamSynchronize(p->stream);
-        cudaGetLastError();
-        st = -11;
-        break;
-      }
-    }
+    if (q == cudaSuccess) return 0;
+    if (q != cudaErrorNotReady) return -100 - (int)q;
+    if (const int w = wd.check()) return w;
     std::this_thread::yield();
   }
-  if (ws) cudaStreamDestroy(ws);
-  if (h) cudaFreeHost(h);
-  return st;
 }
 
 static int finish_info(chol_plan_s* p, int* info) {
@@ -864,6 +907,9 @@ static int factor_streamed(chol_plan_s* p, const double* A, int64_t lda, double*
   *p->h_epoch = (int)p->epoch;
   CUDA_TRY(cudaStreamWaitEvent(p->s_in, p->ev2, 0));
   CUDA_TRY(cudaStreamWaitEvent(p->s_out, p->ev2, 0));
+  // from here on every exit path waits for the copy streams (they read A / write L, the
+  // caller's memory) and joins the zeroing thread before returning
+  int rc = 0;
   auto copy_in = [&](int64_t i, int64_t j) -> int {
     const int64_t t = tile_index(i, j);
     CUDA_TRY(cudaMemcpy2DAsync(p->tiles + t * nb * nb, nb * 8, A + i * nb * lda + j * nb, lda * 8, nb * 8, nb,
@@ -874,16 +920,26 @@ static int factor_streamed(chol_plan_s* p, const double* A, int64_t lda, double*
   // the scheduler's watch order (sched_arrival_order)
   std::vector<std::pair<int, int>> arr;
   sched_arrival_order(p->sched, arr);
-  int s = 0;
-  for (size_t a = 0; a < arr.size() && !s; ++a) s = copy_in(arr[a].first, arr[a].second);
-  if (s) return s;
+  for (size_t a = 0; a < arr.size() && !rc; ++a) rc = copy_in(arr[a].first, arr[a].second);
+  if (rc) {  // the kernel waits for arrivals that will never come: stop it
+    sched_abort(p->sched);
+    cudaStreamSynchronize(p->stream);
+    cudaStreamSynchronize(p->s_in);
+    cudaGetLastError();
+    return rc;
+  }
   // L's strictly upper tiles are zeroed on the host once the input has been read:
   // concurrent with the input copies the memset competes with the copy engine for
   // host DRAM bandwidth (measured: arrivals ~2x slower, e2e 90 -> 80 ms at n=19200)
-  std::thread zero_upper([=] {
+  struct Joiner {
+    std::thread t;
+    ~Joiner() {
+      if (t.joinable()) t.join();
+    }
+  } zero_upper{std::thread([=] {
     cudaStreamSynchronize(p->s_in);
     host_zero_upper_tiles(L, ldl, n, nb);
-  });
+  })};
   // stream out every tile as it becomes final: L_kk (the POTRF leaves the strictly
   // upper triangle of diagonal tiles zeroed), then L_ik, in publication order
   std::vector<int64_t> pending;
@@ -895,50 +951,65 @@ static int factor_streamed(chol_plan_s* p, const double* A, int64_t lda, double*
       row_of[tile_index(i, j)] = (int)i;
       col_of[tile_index(i, j)] = (int)j;
     }
+  auto copy_out = [&](int64_t t) {
+    const int64_t i = row_of[t], j = col_of[t];
+    const cudaError_t e = cudaMemcpy2DAsync(L + i * nb * ldl + j * nb, ldl * 8, p->tiles + t * nb * nb, nb * 8,
+                                            nb * 8, nb, cudaMemcpyDefault, p->s_out);
+    if (e && !rc) rc = -100 - (int)e;
+  };
+  Watchdog wd(p);
   const volatile int* outf = p->h_out_flags;
   size_t head = 0;
-  int rc = 0;
   while (head < pending.size() && !rc) {
     bool progressed = false;
     for (size_t w = head; w < pending.size() && w < head + 256; ++w) {
       const int64_t t = pending[w];
       if (t < 0 || outf[t] != (int)p->epoch) continue;
-      const int64_t i = row_of[t], j = col_of[t];
-      const cudaError_t e = cudaMemcpy2DAsync(L + i * nb * ldl + j * nb, ldl * 8, p->tiles + t * nb * nb, nb * 8,
-                                              nb * 8, nb, cudaMemcpyDefault, p->s_out);
-      if (e) rc = -100 - (int)e;
+      copy_out(t);
       pending[w] = -1;
       progressed = true;
     }
     while (head < pending.size() && pending[head] < 0) ++head;
     if (!progressed) {
-      if (cudaStreamQuery(p->stream) == cudaSuccess) {  // kernel done: take the rest
+      const cudaError_t q = cudaStreamQuery(p->stream);
+      if (q == cudaSuccess) {  // kernel done: take the rest
         for (size_t w = head; w < pending.size(); ++w)
           if (pending[w] >= 0) {
-            const int64_t t = pending[w], i = row_of[t], j = col_of[t];
-            cudaMemcpy2DAsync(L + i * nb * ldl + j * nb, ldl * 8, p->tiles + t * nb * nb, nb * 8, nb * 8, nb,
-                              cudaMemcpyDefault, p->s_out);
+            copy_out(pending[w]);
             pending[w] = -1;
           }
         head = pending.size();
+      } else if (q != cudaErrorNotReady) {  // a fault: the query fails from now on
+        rc = -100 - (int)q;
+      } else if (const int w = wd.check()) {  // stalled: aborted, report -11
+        rc = w;
       } else {
         std::this_thread::yield();
       }
     }
   }
-  // ev3 after the last output copy: the timed span covers the exposed transfers
-  cudaEvent_t out_done;
-  CUDA_TRY(cudaEventCreateWithFlags(&out_done, cudaEventDisableTiming));
-  CUDA_TRY(cudaEventRecord(out_done, p->s_out));
-  CUDA_TRY(cudaStreamWaitEvent(p->stream, out_done, 0));
-  cudaEventDestroy(out_done);
-  CUDA_TRY(cudaEventRecord(p->ev3, p->stream));
-  const int st2 = finish_info(p, info);
-  CUDA_TRY(cudaStreamSynchronize(p->s_in));
-  CUDA_TRY(cudaStreamSynchronize(p->s_out));
-  zero_upper.join();
-  if (rc) return rc;
+  int st2 = 0;
+  if (!rc) {
+    // ev3 after the last output copy: the timed span covers the exposed transfers
+    cudaEvent_t out_done;
+    cudaError_t e = cudaEventCreateWithFlags(&out_done, cudaEventDisableTiming);
+    if (!e) e = cudaEventRecord(out_done, p->s_out);
+    if (!e) e = cudaStreamWaitEvent(p->stream, out_done, 0);
+    if (out_done) cudaEventDestroy(out_done);
+    if (!e) e = cudaEventRecord(p->ev3, p->stream);
+    if (e) rc = -100 - (int)e;
+    st2 = rc ? 0 : finish_info(p, info);
+  }
+  const cudaError_t e_in = cudaStreamSynchronize(p->s_in);
+  const cudaError_t e_out = cudaStreamSynchronize(p->s_out);
+  zero_upper.t.join();
+  if (rc) {
+    p->factored = false;
+    return rc;
+  }
   if (st2) return st2;
+  if (e_in) return -100 - (int)e_in;
+  if (e_out) return -100 - (int)e_out;
   float tot = 0.f;
   CUDA_TRY(cudaEventElapsedTime(&tot, p->ev2, p->ev3));
   p->last_layout_s = tot * 1e-3 - p->last_factor_s;  // exposed (non-overlapped) transfer time
@@ -1202,6 +1273,7 @@ extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int r
   if (type == T_SYRK && !(j > k && j < N)) return -6;
   if (type == T_GEMM && !(i > j && j > k && i < N)) return -6;
   cudaSetDevice(p->device);
+  invalidate_factor(p);
   StepParams sp = base_params(p);
   sp.tr_t0 = sp.tr_t1 = nullptr;
   sp.tr_base = nullptr;
@@ -1241,6 +1313,7 @@ extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, doub
   const int maxc = type == T_POTRF ? N : type == T_GEMM ? (N - 1) * (N - 2) / 2 : N - 1;
   if (count > maxc) return -6;
   cudaSetDevice(p->device);
+  invalidate_factor(p);
   StepParams sp = base_params(p);
   sp.tr_t0 = sp.tr_t1 = nullptr;
   sp.tr_base = nullptr;

@@ -194,10 +194,10 @@ __global__ void k_generate(double* tiles, int64_t n, int nb, int N, uint64_t see
 }
 
 // ------------------------------------------------------------------ launchers
+// cudaFuncSetAttribute acts on the current device's context: set it on every call (a
+// plan on another device, or another thread, must not find it skipped); it is cheap.
 template <int BS>
-static cudaError_t set_attrs_once() {
-  static bool done = false;
-  if (done) return cudaSuccess;
+static cudaError_t set_attrs() {
   const int bytes = Cfg<BS>::kSmemBytes;
   cudaError_t e;
   if ((e = cudaFuncSetAttribute(k_potrf_diag<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
@@ -205,7 +205,6 @@ static cudaError_t set_attrs_once() {
   if ((e = cudaFuncSetAttribute(k_potrf_update<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
   if ((e = cudaFuncSetAttribute(k_trsm<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
   if ((e = cudaFuncSetAttribute(k_update<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
-  done = true;
   return cudaSuccess;
 }
 
@@ -251,7 +250,7 @@ static int launch_update_t(const CUtensorMap& map, StepParams p, int ntask, cuda
   }
 
 cudaError_t prepare_kernels(int bs) {
-#define PREP(B) return set_attrs_once<B>()
+#define PREP(B) return set_attrs<B>()
   CHOL_DISPATCH(bs, PREP)
 #undef PREP
   return cudaSuccess;

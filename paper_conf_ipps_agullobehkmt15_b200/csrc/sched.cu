@@ -529,7 +529,11 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
         if (lane == 0) {
           __threadfence();  // acquire: the job's inputs were published before it was enqueued
           const Job jb = d.jobs[job];
-          write_desc(&c.jdesc()[e * 3], job, jb, ld_volatile(sp.info) != INT_MAX);
+          // after a non-positive pivot in tile column kf = (info-1)/nb only the jobs of
+          // steps >= kf are skipped: every job of an earlier step (TRSM_i_k, the updates
+          // of step k < kf) still runs, so columns < kf*nb of L are final (chol.h, info)
+          const int inf = ld_volatile(sp.info);
+          write_desc(&c.jdesc()[e * 3], job, jb, inf != INT_MAX && jb.k >= (inf - 1) / sp.nb);
           mbar_arrive(&c.jfull()[e]);
         }
         __syncwarp();

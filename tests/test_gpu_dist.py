@@ -17,7 +17,7 @@ def _lib():
     return c
 
 
-def run_logical(n, nb, p, q, seed=0, family=0, A=None, policy=1):
+def run_logical(n, nb, p, q, seed=0, family=0, A=None, policy=0):  # 0 = CHOL_POLICY_CP_PRIORITY
     c = _lib()
     R = p * q
     sms = torch.cuda.get_device_properties(0).multi_processor_count
@@ -69,7 +69,7 @@ def test_dist_bitwise_equals_single_gpu():
     n, nb = 1920, 96
     A = spdgen.uniform_spd(n, seed=11)
     L2, _ = run_logical(n, nb, 2, 2, A=A)
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
         dA = torch.from_numpy(A.copy()).cuda()
         assert p.factor(dA) == 0
         L1 = dA.cpu().numpy()
@@ -97,7 +97,7 @@ def test_two_processes_share_gpu_through_ipc():
     assert "'infos': [0, 0], 'exact': True" in r.stdout, r.stdout
 
 
-def _run_logical_device(n, nb, p, q, seed, family, policy=1):
+def _run_logical_device(n, nb, p, q, seed, family, policy=0):  # 0 = CHOL_POLICY_CP_PRIORITY
     """run_logical without the host copy: the gathered factor stays on the device."""
     c = _lib()
     R = p * q
@@ -161,7 +161,7 @@ def test_scatter_gather_tiles_single_and_distributed():
     ref, _ = oracle.chol_tiled(A, nb)
     N = n // nb
     # single GPU: every tile is owned
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
         packed = np.ascontiguousarray(_packed_owned(A, nb, lambda i, j: True))
         ntiles = N * (N + 1) // 2
         c.chol_scatter_tiles(p.h, packed, ntiles)
@@ -175,7 +175,7 @@ def test_scatter_gather_tiles_single_and_distributed():
     # 2 x 2 logical ranks: each rank streams only its own tiles
     R, pg, qg = 4, 2, 2
     sms = torch.cuda.get_device_properties(0).multi_processor_count
-    plans = [c.DistPlan(n, nb, R, r, grid_p=pg, grid_q=qg, workers=sms // R, policy=1) for r in range(R)]
+    plans = [c.DistPlan(n, nb, R, r, grid_p=pg, grid_q=qg, workers=sms // R, policy=c.POLICY_CP_PRIORITY) for r in range(R)]
     c.DistPlan.connect_local(plans)
     owner = lambda i, j: (i % pg) * qg + (j % qg)  # noqa: E731
     counts = []
@@ -208,11 +208,11 @@ def test_single_process_multi_device_plan(ngpus, monkeypatch):
     n, nb = 1920, 96
     N = n // nb
     A = spdgen.uniform_spd(n, 23)
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p1:
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p1:
         d1 = torch.from_numpy(A.copy()).cuda()
         assert p1.factor(d1) == 0
         ref = d1.cpu().numpy()
-    with c.Plan(n, nb, ngpus=ngpus, policy=1, trace=1) as p:
+    with c.Plan(n, nb, ngpus=ngpus, policy=c.POLICY_CP_PRIORITY, trace=1) as p:
         dA = torch.from_numpy(A.copy()).cuda()
         assert p.factor(dA) == 0
         L = dA.cpu().numpy()

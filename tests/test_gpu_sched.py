@@ -110,3 +110,37 @@ def test_repeated_factorizations_reuse_plan():
             res.append(out.cpu().numpy())
     assert np.array_equal(res[0], spdgen.integer_L0(n, 9))
     assert all(np.array_equal(res[0], r) for r in res[1:])
+
+
+@pytest.mark.parametrize("policy", [0, 1, 2])
+@pytest.mark.parametrize("n,nb,j0", [(1920, 96, 1000), (7680, 960, 3 * 960 + 37)])
+def test_non_spd_leading_columns_are_final(policy, n, nb, j0):
+    """chol.h: with info = j, columns < nb*floor((j-1)/nb) of L are valid.  The scheduler
+    skips only the jobs of steps >= the failing tile column, so every TRSM_i_k and update
+    of an earlier step still runs.  Integer family: those columns are exactly L0's
+    (device pointers and the streamed host-pointer path)."""
+    c = _lib()
+    L0 = spdgen.integer_L0(n, 5)
+    A = spdgen.make_non_spd(spdgen.integer_spd(n, 5), L0, j0, "zero")
+    cols = (j0 // nb) * nb
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=policy) as p:
+        dA = torch.from_numpy(A).cuda()
+        assert p.factor(dA) == j0 + 1
+        L = dA.cpu().numpy()
+        assert np.array_equal(L[:, :cols], L0[:, :cols])
+        Lh = np.full_like(A, np.nan)
+        assert c.chol_factor(p.h, A, n, Lh, n) == j0 + 1  # host buffers: streamed in / out
+        assert np.array_equal(Lh[:, :cols], L0[:, :cols])
+
+
+def test_non_spd_leading_columns_final_task_level_path():
+    """The same contract on the bench's task-level path (N = 17 > 16: per-step POTRF nodes,
+    J_TRSM row-slab jobs), failing at a tile boundary deep in the factorization."""
+    c = _lib()
+    n, nb, j0 = 16320, 960, 12 * 960
+    L0 = spdgen.integer_L0(n, 6)
+    A = spdgen.make_non_spd(spdgen.integer_spd(n, 6), L0, j0, "neg")
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
+        dA = torch.from_numpy(A).cuda()
+        assert p.factor(dA) == j0 + 1
+        assert torch.equal(dA[:, :j0].cpu(), torch.from_numpy(np.ascontiguousarray(L0[:, :j0])))

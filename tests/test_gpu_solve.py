@@ -151,3 +151,38 @@ def test_solve_dmma_and_simt_sweeps_agree(nrhs, monkeypatch):
     p.close()
     _check(A, L, B, X2)
     assert np.max(np.abs(X1 - X2)) <= 1e-12 * max(1.0, float(np.max(np.abs(X1))))
+
+
+def test_solve_refuses_a_factor_that_was_overwritten_or_failed():
+    """Every call that writes the tile store (generate, scatter, run_batch / run_task, a
+    factorization that fails) invalidates the factor: chol_solve returns -10 instead of
+    solving with stale data or stale cached inverses."""
+    c = _lib()
+    n, nb = 1920, 960
+    B = torch.from_numpy(spdgen.rhs(n, 3, 1)).cuda()
+    with c.Plan(n, nb) as p:
+
+        def expect_stale():
+            with pytest.raises(c.CholError) as e:
+                p.solve(B.clone())
+            assert e.value.status == -10
+
+        def refactor():
+            c.chol_generate(p.h, 3, 0)
+            assert c.chol_factor_inplace(p.h) == 0
+            p.solve(B.clone())  # fine again
+
+        refactor()
+        c.chol_generate(p.h, 4, 0)
+        expect_stale()
+        refactor()
+        c.chol_scatter(p.h, torch.from_numpy(spdgen.uniform_spd(n, 5)).cuda(), n)
+        expect_stale()
+        refactor()
+        c.chol_run_batch(p.h, c.GEMM if n // nb > 2 else c.SYRK, 1)
+        expect_stale()
+        refactor()
+        L0 = spdgen.integer_L0(n, 2)
+        bad = torch.from_numpy(spdgen.make_non_spd(spdgen.integer_spd(n, 2), L0, 1000)).cuda()
+        assert p.factor(bad) == 1001
+        expect_stale()

@@ -22,9 +22,9 @@ def run(**opts):
     return {"opts": opts, "ms": round(t * 1e3, 3), "tflops": round(n ** 3 / 3 / t / 1e12, 3)}
 
 
-out = [run(policy=0), run(policy=1)]
+out = [run(policy=c.POLICY_DYNAMIC), run(policy=c.POLICY_CP_PRIORITY)]
 for lw in (8, 16, 32):
     for d in (1, 2, 4, 8, N - 1):
-        out.append(run(policy=2, trsm_pin_distance=d, latency_workers=lw))
+        out.append(run(policy=c.POLICY_STATIC, trsm_pin_distance=d, latency_workers=lw))
 for o in out:
     print(json.dumps({"n": n, **o}))

@@ -3,7 +3,7 @@ import sys, os, json
 sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import paper_conf_ipps_agullobehkmt15_b200 as c
 n = int(sys.argv[1]) if len(sys.argv) > 1 else 19200
-pol = int(sys.argv[2]) if len(sys.argv) > 2 else 1
+pol = int(sys.argv[2]) if len(sys.argv) > 2 else 0  # 0 = CP_PRIORITY
 nb = 960
 with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=pol, trace=1) as p:
     for rep in range(2):

@@ -14,7 +14,7 @@ d = torch.empty((nt, nb, nb), dtype=torch.float64, device="cuda")
 s = rt.cudaStreamCreateWithFlags(rt.cudaStreamNonBlocking)[1]
 evs = [rt.cudaEventCreate()[1] for _ in range(nt + 1)]
 res = {}
-with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
     c.chol_generate(p.h, 0, 0)
     for load in (False, True):
         torch.cuda.synchronize()

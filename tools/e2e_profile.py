@@ -11,7 +11,7 @@ nb = 960
 N = n // nb
 A_h = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
 L_h = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
-with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1, trace=2) as p:
+with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY, trace=2) as p:
     c.chol_generate(p.h, 0, 0)
     c.chol_gather(p.h, A_h, n)
     walls = []

@@ -18,7 +18,7 @@ for n in Ns:
         env = dict(kv.split("=") for kv in s.split()) if s else {}
         old = {k: os.environ.get(k) for k in env}
         os.environ.update(env)
-        with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+        with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
             ts = []
             for r in range(7):
                 c.chol_generate(p.h, 0, 0)

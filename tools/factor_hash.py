@@ -9,7 +9,7 @@ import torch
 import paper_conf_ipps_agullobehkmt15_b200 as c
 
 for n in [int(x) for x in sys.argv[1].split(",")]:
-    with c.Plan(n, 960, executor=c.EXEC_SCHEDULER, policy=1) as p:
+    with c.Plan(n, 960, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
         c.chol_generate(p.h, 0, 0)
         assert c.chol_factor_inplace(p.h) == 0
         L = torch.empty(n, n, dtype=torch.float64, device="cuda")

@@ -6,7 +6,7 @@ import numpy as np
 import paper_conf_ipps_agullobehkmt15_b200 as c
 
 n = int(sys.argv[1]) if len(sys.argv) > 1 else 19200
-pol = int(sys.argv[2]) if len(sys.argv) > 2 else 1
+pol = int(sys.argv[2]) if len(sys.argv) > 2 else 0  # 0 = CP_PRIORITY
 binus = float(sys.argv[3]) if len(sys.argv) > 3 else 250.0
 nb = 960
 JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU", "RECV"]

@@ -5,7 +5,7 @@ sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
 import paper_conf_ipps_agullobehkmt15_b200 as c
 n = int(sys.argv[1])
 for nb in [int(x) for x in sys.argv[2].split(",")]:
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
         ts = []
         for r in range(4):
             c.chol_generate(p.h, 0, 0)

@@ -16,7 +16,7 @@ nb = int(sys.argv[1]) if len(sys.argv) > 1 else 960
 reps = int(sys.argv[2]) if len(sys.argv) > 2 else 5
 bs = 96 if nb % 96 == 0 else (64 if nb % 64 == 0 else 32)
 nbb = nb // bs
-with c.Plan(nb, nb, executor=c.EXEC_SCHEDULER, policy=1, trace=2) as p:
+with c.Plan(nb, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY, trace=2) as p:
     best = None
     for rep in range(reps):
         c.chol_generate(p.h, 0, 0)

@@ -23,7 +23,7 @@ def run(**opts):
             "ms": round(t * 1e3, 3), "tflops": round(n ** 3 / 3 / t / 1e12, 3)}
 
 
-print(json.dumps(run(policy=1)), flush=True)
+print(json.dumps(run(policy=c.POLICY_CP_PRIORITY)), flush=True)
 for lw in lws:
     for d in ds:
-        print(json.dumps(run(policy=2, trsm_pin_distance=d, latency_workers=lw)), flush=True)
+        print(json.dumps(run(policy=c.POLICY_STATIC, trsm_pin_distance=d, latency_workers=lw)), flush=True)

@@ -9,7 +9,7 @@ Ns = [int(x) for x in sys.argv[1].split(",")] if len(sys.argv) > 1 else [10, 12,
 nb = 960
 for N in Ns:
     n = N * nb
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
         ts = []
         for r in range(4):
             c.chol_generate(p.h, 0, 0)

@@ -13,7 +13,7 @@ for N in Ns:
         if m > N:
             continue
         os.environ["CHOL_BLOCK_TAIL"] = str(m)
-        with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=1) as p:
+        with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY) as p:
             ts = []
             for r in range(4):
                 c.chol_generate(p.h, 0, 0)

@@ -20,7 +20,7 @@ def worker(rank, world, port, n, nb, q):
         dist.all_gather_object(out, b)
         return out
 
-    plan = c.DistPlan(n, nb, world, rank, allgather=allgather, grid_p=1, grid_q=world, workers=74, policy=1)
+    plan = c.DistPlan(n, nb, world, rank, allgather=allgather, grid_p=1, grid_q=world, workers=74, policy=c.POLICY_CP_PRIORITY)
     c.chol_generate(plan.h, 2, 1)
     dist.barrier()
     t0 = time.time()
