@@ -4,19 +4,21 @@
 
 One step = one factorization A = L L^T of a seeded synthetic SPD matrix through the
 C-ABI (chol_factor_inplace: every Algorithm 1 task -- POTRF, TRSM, SYRK, GEMM -- run by
-the device-side scheduler kernel).  Default workload = BASELINE.json configs[1]:
-n = 19200 as 20 x 20 tiles of nb = 960 on 1 B200.
+the device-side scheduler kernel).  Default workload = the north-star point, the largest
+1-GPU configuration of BASELINE.json configs[2]: n = 46080 as 48 x 48 tiles of nb = 960
+on 1 B200 (target >= 70% of the FP64 peak).  configs[1] (n = 19200, 20 x 20 tiles) is
+measured too and reported as the extra field "config_19200" (--extra-n 0 skips it).
 
 Usage: python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
-       [--n 19200] [--nb 960] [--policy cp|dynamic|static] [--executor sched|host]
-       [--logical-ranks R --grid PxQ]
+       [--n 46080] [--nb 960] [--policy cp|dynamic|static] [--executor sched|host]
+       [--scaling strong|weak] [--logical-ranks R --grid PxQ]
 Under torchrun (N > 1) the N ranks factor ONE matrix together (2D block-cyclic
 owner-computes, panel tiles pulled over NVLink peer memory); rank 0 prints ONE JSON line.
---scaling weak (default): the matrix order grows with N so that the flops per GPU stay
-fixed, n_N = nb * round(N_1 * N^(1/3)) with N_1 = n / nb tiles at one GPU (n=19200:
-24000, 30720, 38400 at 2, 4, 8 GPUs -- the paper's own axis is the matrix order,
-P:L489); --scaling strong keeps n fixed.  --logical-ranks R runs the distributed path with R ranks sharing
-one GPU (tests the multi-GPU machinery; not a scaling number).
+--scaling strong (default): n stays fixed as N grows (north star: >= 5x at n = 46080 on
+8 GPUs); --scaling weak: the matrix order grows with N so that the flops per GPU stay
+fixed, n_N = nb * round(N_1 * N^(1/3)) with N_1 = n / nb tiles at one GPU.
+--logical-ranks R runs the distributed path with R ranks sharing one GPU (tests the
+multi-GPU machinery; not a scaling number).
 """
 from __future__ import annotations
 
@@ -44,7 +46,8 @@ def parse():
     ap.add_argument("--steps", type=int, default=5)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--n", type=int, default=19200)
+    ap.add_argument("--n", type=int, default=46080)
+    ap.add_argument("--extra-n", type=int, default=19200, help="also time configs[1] at this n (0 = skip)")
     ap.add_argument("--nb", type=int, default=960)
     ap.add_argument("--policy", choices=list(POLICIES), default="cp")
     ap.add_argument("--executor", choices=["sched", "host"], default="sched")
@@ -55,7 +58,7 @@ def parse():
     ap.add_argument("--cpu-sample-n", type=int, default=7680)
     ap.add_argument("--grid", default="", help="process grid PxQ (default 1xN; SURVEY §8e prefers p <= q)")
     ap.add_argument("--logical-ranks", type=int, default=0)
-    ap.add_argument("--scaling", choices=["weak", "strong"], default="weak")
+    ap.add_argument("--scaling", choices=["weak", "strong"], default="strong")
     return ap.parse_args()
 
 
@@ -230,38 +233,25 @@ def cpu_baseline(args):
                       f"nb={args.nb}), {dt:.1f} s"}
 
 
-def calibrate(c, args, workers):
-    """Per-type task times for the bounds (reading R9).
+def calibrate(c, args):
+    """Per-type task times for the bounds (reading R9), measured through the
+    persistent scheduler kernel (chol_run_batch on a scheduler plan of the same n, nb):
 
-    T_thr (area term): GPU time a task of type t costs when the GPU is saturated,
-    measured on this scheduler itself -- the SM-time of the task's CTA jobs in the job
-    trace of one factorization, divided by the number of workers.  sum_t N_t T_thr_t is
-    then the busy SM-time / workers, a true lower bound on the makespan.
-    T_lat (path terms): a task alone on an idle GPU (chol_run_task, host-launched tile
-    kernels), capped by the shortest task latency seen in the trace."""
-    import numpy as np
+    T_thr (area term): device time per task in a saturating batch of independent tasks of
+    the type, in the factorization's bulk decomposition -- all (N-1)(N-2)/2 GEMM_i_j_0, the
+    N(N-1)/2 TRSM_i_k row-slab tasks, the N-1 SYRK_j_0, the N POTRFs.
+    T_lat (path terms): one task alone on the idle GPU, in the critical-path decomposition
+    (TRSM column steps, the POTRF block DAG).  Neither is taken from the factorization
+    being bounded."""
     n, nb = args.n, args.nb
     N = n // nb
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=POLICIES[args.policy], trace=2) as p:
+    counts = [N, N * (N - 1) // 2, N - 1, (N - 1) * (N - 2) // 2]
+    T_thr, T_lat = [], []
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=POLICIES[args.policy]) as p:
         c.chol_generate(p.h, args.seed, 0)
-        c.chol_factor_inplace(p.h)
-        jt = c.chol_job_trace(p.h)
-        recs, _ = c.chol_trace(p.h)
-    dur = (jt[:, 1].astype(np.int64) - jt[:, 0].astype(np.int64)) * 1e-9
-    task = (jt[:, 3] & np.uint64(0xffffffff)).astype(np.int64)
-    ttype = np.zeros(task.max() + 1, dtype=np.int64)
-    for r in recs:
-        ttype[c.chol_task_id(N, r["type"], r["i"], r["j"], r["k"])] = r["type"]
-    counts = [N, N * (N - 1) // 2, N * (N - 1) // 2, N * (N - 1) * (N - 2) // 6]
-    T_thr = [float(dur[ttype[task] == t].sum()) / (max(counts[t], 1) * workers) for t in range(4)]
-    lat_trace = [min(((r["t1_ns"] - r["t0_ns"]) * 1e-9 for r in recs if r["type"] == t), default=float("inf"))
-                 for t in range(4)]
-    T_lat = []
-    with c.Plan(3 * nb, nb, executor=c.EXEC_HOST) as p:
-        c.chol_generate(p.h, 1, 0)
         for t in range(4):
-            c.chol_run_task(p.h, t, 2, 1, 0 if t else 1, 1)
-            T_lat.append(min(c.chol_run_task(p.h, t, 2, 1, 0 if t else 1, 5) * 1e-3, lat_trace[t]))
+            T_thr.append(c.chol_run_batch(p.h, t, max(counts[t], 1), 2) * 1e-3)
+            T_lat.append(c.chol_run_batch(p.h, t, 1, 5) * 1e-3)
     return T_lat, T_thr
 
 
@@ -375,7 +365,7 @@ def run_dist(args, ws, rank, local):
         try:
             import types
             a1 = types.SimpleNamespace(n=n, nb=nb, policy=args.policy, seed=args.seed)
-            T_lat, T_thr = calibrate(c, a1, torch.cuda.get_device_properties(local).multi_processor_count)
+            T_lat, T_thr = calibrate(c, a1)
             b = c.chol_bounds(n, nb, ws, T_lat, T_thr)
             b["owner_area"] = c.chol_owner_area(n // nb, p, q, T_thr)[0]
             line["bounds"] = {"seconds": b, "upper_tflops": {k: flops / v / 1e12 for k, v in b.items() if v > 0},
@@ -422,64 +412,82 @@ def run_logical(args):
                       "config": {"n": n, "nb": nb}}), flush=True)
 
 
+def time_factorizations(c, plan, args, ws, steps, warmup):
+    """W untimed warm-ups, then `steps` factorizations, each of a freshly generated input
+    already resident in HBM (untimed); returns the per-step device times (CUDA events on
+    the plan stream) and the kernel launches of the timed steps."""
+    import torch
+    for _ in range(warmup):
+        c.chol_generate(plan.h, args.seed, 0)
+        info = c.chol_factor_inplace(plan.h)
+        assert info == 0, info
+    torch.cuda.synchronize()
+    times, launches = [], 0
+    for _ in range(steps):
+        c.chol_generate(plan.h, args.seed, 0)  # fresh input, resident in HBM, untimed
+        barrier(ws)
+        torch.cuda.synchronize()
+        info = c.chol_factor_inplace(plan.h)  # CUDA events on the plan's stream
+        torch.cuda.synchronize()
+        assert info == 0, info
+        times.append(c.chol_last_times(plan.h)[0])
+        launches += c.chol_last_launches(plan.h)
+    return times, launches
+
+
+def ncu_traffic(n: int):
+    """DRAM bytes (read + write) per launch of k_sched at this n, from the ncu --set full
+    capture of this build committed under profiles/r02/ (None if there is none)."""
+    prof = os.path.join(ROOT, "profiles", "r02", "ncu_summary.json")
+    try:
+        d = json.load(open(prof))
+        return d["k_sched"][str(n)]["dram_bytes_per_launch"]
+    except Exception:
+        return None
+
+
 def run_ours(args, ws, rank, local):
     import torch
     import paper_conf_ipps_agullobehkmt15_b200 as c
 
     n, nb = args.n, args.nb
+    N = n // nb
     flops = n ** 3 / 3.0
     ex = c.EXEC_SCHEDULER if args.executor == "sched" else c.EXEC_HOST
     pol = POLICIES[args.policy]
     plan = c.Plan(n, nb, executor=ex, policy=pol)
     info_d = c.chol_get_info(plan.h)
 
-    for _ in range(args.warmup):
-        c.chol_generate(plan.h, args.seed, 0)
-        info = c.chol_factor_inplace(plan.h)
-        assert info == 0, info
-    torch.cuda.synchronize()
-
-    times, launches = [], 0
     with ClockSampler(local) as clk:
-        for _ in range(args.steps):
-            c.chol_generate(plan.h, args.seed, 0)  # fresh input, resident in HBM, untimed
-            barrier(ws)
-            torch.cuda.synchronize()
-            info = c.chol_factor_inplace(plan.h)  # CUDA events on the plan's stream
-            torch.cuda.synchronize()
-            assert info == 0, info
-            times.append(c.chol_last_times(plan.h)[0])
-            launches += c.chol_last_launches(plan.h)
+        times, launches = time_factorizations(c, plan, args, ws, args.steps, args.warmup)
     clocks = clk.summary()
     total = allmax(ws, sum(times))
     t_step = total / args.steps
     value = ws * flops / t_step / 1e12
 
-    # roofline: the dominant (and only long) kernel is the persistent scheduler kernel
+    # roofline: the dominant (and only long) kernel is the persistent scheduler kernel;
+    # one launch = one factorization = n^3/3 algorithmic flops
     achieved = flops / (sum(times) / len(times)) / 1e12
-    traffic = None
-    prof = os.path.join(ROOT, "profiles", "r01", "ncu_summary.json")
-    if os.path.exists(prof):
-        try:
-            traffic = json.load(open(prof)).get("sched_kernel_dram_bytes_per_launch")
-        except Exception:
-            traffic = None
     roofline = {"bound": "tensor", "achieved": achieved, "peak": FP64_PEAK_TFLOPS, "unit": "TFLOP/s",
-                "frac": achieved / FP64_PEAK_TFLOPS, "traffic": traffic,
+                "frac": achieved / FP64_PEAK_TFLOPS, "traffic": ncu_traffic(n),
                 "kernel": "k_sched (persistent scheduler: all POTRF/TRSM/SYRK/GEMM sub-tasks)",
-                "peak_source": "measured FP64 DMMA microbenchmark (MEASURED_PEAKS.json has no FP64 entry)"}
-
+                "algorithmic": "n^3/3 flop per launch (one factorization)",
+                "peak_source": "measured FP64 DMMA microbenchmark, 148 SM x 64 FMA/clk x 2 x 1.965 GHz "
+                               "(MEASURED_PEAKS.json has no FP64 entry; the 40 TF/s brief figure would give "
+                               "frac x 0.93)"}
+    is_ns = (n, nb) == (46080, 960)
     line = {
         "metric": METRIC, "value": value, "unit": "TFLOP/s", "n_gpus": ws, "steps": args.steps,
         "warmup": args.warmup, "ms_per_step": 1e3 * t_step, "higher_is_better": True,
-        "scaling": "weak", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
-        "config": {"workload": f"FP64 SPD n={n} as {n // nb}x{n // nb} tiles of nb={nb}"
+        "scaling": args.scaling, "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": {"workload": f"FP64 SPD n={n} as {N}x{N} tiles of nb={nb}"
+                               + (" (north star; BASELINE configs[2], largest 1-GPU point)" if is_ns else "")
                                + (" (BASELINE configs[1])" if (n, nb) == (19200, 960) else ""),
                    "n": n, "nb": nb, "block": info_d["block"], "executor": args.executor,
                    "policy": args.policy, "workers": info_d["workers"],
                    "parallelism": "1 GPU" if ws == 1 else f"{ws} replicas (one factorization per GPU)",
                    "input": "uniform family seed %d, regenerated on device before each step (untimed)" % args.seed,
-                   "l2": f"input {(n // nb) * (n // nb + 1) // 2 * nb * nb * 8 / 1e9:.2f} GB >> 126 MB L2, "
+                   "l2": f"input {N * (N + 1) // 2 * nb * nb * 8 / 1e9:.2f} GB >> 126 MB L2, "
                          "rewritten between steps",
                    "timing": "CUDA events on the plan stream around each factorization, max over ranks"},
         "pct_fp64_peak": 100.0 * achieved / FP64_PEAK_TFLOPS,
@@ -492,39 +500,55 @@ def run_ours(args, ws, rank, local):
                           "best": 1e3 * min(times), "runs": len(times)},
     }
 
-    # end-to-end: the C-ABI with HOST buffers (pinned), copies inside the timed region
+    # end-to-end: the C-ABI with HOST buffers, copies inside the timed region.  One pinned
+    # n x n buffer, factored in place (A == L, allowed by chol.h): each step streams the
+    # lower tiles in while the factorization runs and every final tile of L back out.  The
+    # buffer is refilled with the input (untimed) before each step.
     if not args.no_e2e:
-        A_h = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
-        L_h = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
-        c.chol_generate(plan.h, args.seed, 0)
-        c.chol_gather(plan.h, A_h, n)  # the same matrix, lower triangle (upper zero)
+        H = torch.empty((n, n), dtype=torch.float64, pin_memory=True)
         e2e_t = []
         for it in range(3):
+            c.chol_generate(plan.h, args.seed, 0)
+            c.chol_gather(plan.h, H, n)  # the input matrix, lower triangle (untimed)
             barrier(ws)
             torch.cuda.synchronize()
             t0 = time.perf_counter()
-            info = c.chol_factor(plan.h, A_h, n, L_h, n)
+            info = c.chol_factor(plan.h, H, n, H, n)
             dt = time.perf_counter() - t0
             assert info == 0
             if it > 0:
                 e2e_t.append(dt)
         t_e2e = allmax(ws, statistics.mean(e2e_t))
-        tile_bytes = (n // nb) * (n // nb + 1) // 2 * nb * nb * 8
+        tile_bytes = N * (N + 1) // 2 * nb * nb * 8
         line["e2e"] = {"value": ws * flops / t_e2e / 1e12, "unit": "TFLOP/s", "h2d_bytes_per_step": tile_bytes,
                        "d2h_bytes_per_step": tile_bytes, "ms_per_step": 1e3 * t_e2e,
-                       "layout_ms": 1e3 * c.chol_last_times(plan.h)[1]}
-        del A_h, L_h
+                       "exposed_layout_ms": 1e3 * c.chol_last_times(plan.h)[1],
+                       "path": "chol_factor(A=L, pinned host, in place): lower tiles streamed in during the "
+                               "factorization, final tiles of L streamed out as published, upper part zeroed "
+                               "on the host; wall time"}
+        del H
     plan.close()
 
+    # configs[1] beside the headline (parity cases and the r01 headline)
+    if args.extra_n and args.extra_n != n and rank == 0:
+        with c.Plan(args.extra_n, nb, executor=ex, policy=pol) as p2:
+            t2, _ = time_factorizations(c, p2, args, 1, max(args.steps, 5), args.warmup)
+        f2 = args.extra_n ** 3 / 3.0
+        line["config_19200" if args.extra_n == 19200 else f"config_{args.extra_n}"] = {
+            "n": args.extra_n, "nb": nb, "value": f2 / statistics.mean(t2) / 1e12, "unit": "TFLOP/s",
+            "ms_per_step": 1e3 * statistics.mean(t2), "frac": f2 / statistics.mean(t2) / 1e12 / FP64_PEAK_TFLOPS,
+            "runs": len(t2)}
+
     if not args.no_bounds and rank == 0:
-        T_lat, T_thr = calibrate(c, args, info_d["workers"] or 148)
+        T_lat, T_thr = calibrate(c, args)
         b = c.chol_bounds(n, nb, 1, T_lat, T_thr)
         line["bounds"] = {
             "T_lat_s": dict(zip(c.TYPE_NAMES, T_lat)), "T_thr_s": dict(zip(c.TYPE_NAMES, T_thr)),
             "seconds": b, "upper_tflops": {k: (flops / v / 1e12 if v and v > 0 else None) for k, v in b.items()},
             "makespan_over_mixed": t_step / b["mixed"],
-            "calibration": "T_thr from the scheduler's own job trace (SM-time per task / workers); "
-                           "T_lat = min(task alone on an idle GPU, shortest traced task)",
+            "calibration": "chol_run_batch through the persistent scheduler: T_thr = per task in a saturating "
+                           "batch of independent same-type tasks (bulk decomposition), T_lat = one task alone "
+                           "(critical-path decomposition); reading R9",
         }
 
     if rank == 0 and ws == 1 and not args.no_cpu_baseline:

@@ -179,7 +179,16 @@ int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double
 /* Run `count` independent instances of tile task type `type` concurrently
  * (count GEMMs / SYRKs / TRSMs on distinct output tiles of the store, POTRFs on
  * distinct diagonal tiles) and return the device time per instance in *ms
- * (throughput time T_t^thr, reading R9).  Overwrites the store. */
+ * (throughput time T_t^thr for a saturating count, latency T_t^lat for count = 1;
+ * DESIGN.md reading R9).  Executor CHOL_EXEC_SCHEDULER: the batch runs through the
+ * persistent scheduler kernel in the factorization's own job decompositions (count > 1:
+ * the bulk forms, row-slab TRSMs; count = 1: the critical-path forms, TRSM column steps
+ * and the POTRF block DAG), one untimed warm-up run first; CHOL_EXEC_HOST: one batch
+ * launch of the host-executor tile kernels per rep.  Overwrites the store (a factor in
+ * it is invalidated).  Errors: -6 bad type, count < 1, reps < 1 or count above the
+ * instances available (POTRF N, SYRK N-1, GEMM (N-1)(N-2)/2 at step 0; TRSM N-1 at step 0 on
+ * the host executor, N(N-1)/2 panel tiles TRSM_i_k in Algorithm 1 order on the scheduler);
+ * -8 on multi-GPU plans. */
 int chol_run_batch(chol_plan_t p, int type, int count, int reps, double* ms);
 
 /* ---- multi-GPU: one process (or logical rank) per GPU, 2D block-cyclic owner-computes ----

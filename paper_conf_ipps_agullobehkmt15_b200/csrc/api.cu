@@ -1311,7 +1311,7 @@ extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, doub
   // instances at step k = 0: POTRF on diagonal tiles 0..count-1, TRSM (i, 0),
   // SYRK (j, 0), GEMM (i, j, 0) -- all with distinct output tiles.
   const int maxc = type == T_POTRF ? N : type == T_GEMM ? (N - 1) * (N - 2) / 2 : N - 1;
-  if (count > maxc) return -6;
+  if (count > maxc && !(p->sched && type == T_TRSM)) return -6;  // scheduler: TRSM_i_k over all k
   cudaSetDevice(p->device);
   invalidate_factor(p);
   StepParams sp = base_params(p);
@@ -1319,8 +1319,26 @@ extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, doub
   sp.tr_base = nullptr;
   sp.k = 0;
   CUDA_TRY(launch_init_info(p->d_info, p->stream));
-  CUDA_TRY(cudaEventRecord(p->ev0, p->stream));
   int nl = 0;
+  if (p->sched) {  // the persistent scheduler, the factorization's own executor (reading R9)
+    SchedState* bst = nullptr;
+    if (const int st = sched_create_batch(&bst, p->N, p->nb, p->bs, p->sms, &p->opts, type, count)) return st;
+    int st = 0;
+    for (int r = 0; r <= reps && !st; ++r) {  // r = 0: untimed warm-up
+      if (r == 1) CUDA_TRY(cudaEventRecord(p->ev0, p->stream));
+      st = sched_run(bst, p->map, sp, p->stream, &nl, ++p->epoch);
+    }
+    cudaError_t e = cudaEventRecord(p->ev1, p->stream);
+    if (!e) e = cudaStreamSynchronize(p->stream);
+    sched_destroy(bst);
+    if (st) return st;
+    if (e) return -100 - (int)e;
+    float t = 0.f;
+    CUDA_TRY(cudaEventElapsedTime(&t, p->ev0, p->ev1));
+    if (ms) *ms = t / reps / count;
+    return 0;
+  }
+  CUDA_TRY(cudaEventRecord(p->ev0, p->stream));
   for (int r = 0; r < reps; ++r) {
     if (type == T_POTRF) {
       CUDA_TRY(launch_potrf(p->bs, p->map, sp, count, p->stream, &nl));

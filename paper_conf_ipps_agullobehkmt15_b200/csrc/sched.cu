@@ -637,6 +637,111 @@ struct Builder {
 
 }  // namespace
 
+// POTRF_k as per-step nodes: DIAG b -> PANEL b (nbb-1-b jobs) -> UPDATE b (K = BS) -> DIAG b+1
+static void build_potrf_steps(Builder& B, int k, int pid, int* first, int* last) {
+  const int nbb = B.nbb;
+  int prev = -1;
+  for (int b = 0; b < nbb; ++b) {
+    const int dn = B.add_node(pid, T_POTRF, k, k);
+    B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+    if (prev >= 0) B.edge(prev, dn);
+    if (b == 0) *first = dn;
+    prev = dn;
+    if (b + 1 < nbb) {
+      const int pn = B.add_node(pid, T_POTRF, k, k);
+      for (int r = b + 1; r < nbb; ++r)
+        B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
+      B.edge(prev, pn);
+      const int un = B.add_node(pid, T_POTRF, k, k);
+      for (int r = b + 1; r < nbb; ++r)
+        for (int q = b + 1; q <= r; ++q)
+          B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
+      B.edge(pn, un);
+      prev = un;
+    }
+  }
+  *last = prev;
+}
+
+// POTRF_k as a block-level DAG over the BS x BS blocks of the diagonal tile (right-looking
+// nested Cholesky): D(b) = potf2 of block (b,b); P(r,b) = solve of block (r,b) against
+// L_bb; U(r,q,b) = K=BS update of block (r,q) by blocks (r,b), (q,b).  One job per node, so
+// the chain D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1) never waits for a whole column or
+// trailing update of the step.  D(nbb-1) is the sink (every inner node is its ancestor).
+// With fuse the chain's last update U(b,b,b-1) is done by D(b) itself: the job runs the
+// J_PUPD code (producer stages, DMMA, epilogue) and then potf2 -- one node and one hop less
+// per inner step, the same bits.  blk (hybrid tail): record per block the entry node and
+// the node that leaves it final (tentry / tfin, nbb x nbb).
+static void build_potrf_blockdag(Builder& B, int k, int pid, bool fuse, bool blk, std::vector<int>* tentry,
+                                 std::vector<int>* tfin, int* first, int* last) {
+  const int nbb = B.nbb;
+  std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1), fusedP(nbb, -1);
+  if (blk) tentry->assign((size_t)nbb * nbb, -1), tfin->assign((size_t)nbb * nbb, -1);
+  for (int b = 0; b < nbb; ++b) {
+    const int dn = B.add_node(pid, T_POTRF, k, k);
+    B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)(fusedP[b] >= 0), 0, 0});
+    if (lastU[b * nbb + b] >= 0) B.edge(lastU[b * nbb + b], dn);
+    if (fusedP[b] >= 0) B.edge(fusedP[b], dn);
+    if (blk && b == 1 && fusedP[b] >= 0) (*tentry)[b * nbb + b] = dn;  // first touch of block (1,1)
+    if (b == 0) *first = dn;
+    *last = dn;
+    for (int r = b + 1; r < nbb; ++r) {
+      const int pn = B.add_node(pid, T_POTRF, k, k);
+      B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
+      B.edge(dn, pn);
+      if (lastU[r * nbb + b] >= 0) B.edge(lastU[r * nbb + b], pn);
+      pan[r] = pn;
+    }
+    for (int r = b + 1; r < nbb; ++r)
+      for (int q = b + 1; q <= r; ++q) {
+        if (fuse && r == b + 1 && q == r) {  // U(b+1,b+1,b): fused into D(b+1)
+          fusedP[r] = pan[r];
+          continue;
+        }
+        const int un = B.add_node(pid, T_POTRF, k, k);
+        B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
+        B.edge(pan[r], un);
+        if (q != r) B.edge(pan[q], un);
+        if (lastU[r * nbb + q] >= 0) B.edge(lastU[r * nbb + q], un);  // same block, previous step
+        lastU[r * nbb + q] = un;
+        if (blk && b == 0) (*tentry)[r * nbb + q] = un;
+      }
+    if (blk) {
+      (*tfin)[b * nbb + b] = dn;
+      if (b == 0) (*tentry)[0] = dn;
+      for (int r = b + 1; r < nbb; ++r) {
+        (*tfin)[r * nbb + b] = pan[r];
+        if (b == 0) (*tentry)[r * nbb] = pan[r];
+      }
+    }
+  }
+}
+
+// TRSM_i_k right-looking over the BS-column blocks c of A_ik, one node per column step:
+//   TS(c): A_ik[:, c] <- A_ik[:, c] L_kk[c,c]^{-T}  (nbb row-block jobs)
+//   TU(c): A_ik[:, c'] -= A_ik[:, c] L_kk[c',c]^T, c' > c  (K = BS)
+static void build_trsm_steps(Builder& B, int i, int k, int tid, int* first, int* last) {
+  const int nbb = B.nbb;
+  int prev_t = -1;
+  for (int cb = 0; cb < nbb; ++cb) {
+    const int ts = B.add_node(tid, T_TRSM, i, k);
+    for (int sl = 0; sl < nbb; ++sl)
+      B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+    if (prev_t >= 0) B.edge(prev_t, ts);
+    if (cb == 0) *first = ts;
+    prev_t = ts;
+    if (cb + 1 < nbb) {
+      const int tu = B.add_node(tid, T_TRSM, i, k);
+      for (int sl = 0; sl < nbb; ++sl)
+        for (int c2 = cb + 1; c2 < nbb; ++c2)
+          B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
+      B.edge(ts, tu);
+      prev_t = tu;
+    }
+  }
+  *last = prev_t;
+}
+
 // Streamed-input tile order.  0 (default): row-major, row i = tiles (i, 0..i) -- each
 // arriving row feeds the trailing updates of every factored column at once.  1: column 0
 // first (every TRSM_i_0 can start after N tiles), then the other tiles row-major.
@@ -652,8 +757,171 @@ void sched_arrival_order(const SchedState* st, std::vector<std::pair<int, int>>&
   arrival_order(st->N, st->arrival, tiles);
 }
 
+// Device tables of a built node graph (jobs, CSR successors, queues), the persistent grid
+// size, the abort word.  Takes ownership of st (destroyed on failure).
+static int sched_upload(SchedState** out, SchedState* st, Builder& B, const std::vector<int>& node_queue,
+                        const std::vector<int>& publish, const std::vector<int4>& watch, const chol_opts_t* opts,
+                        int64_t nb, int bs, int sms) {
+  const int nnodes = (int)B.deps.size();
+  // ---- queue capacities
+  std::vector<int> qcap(kQueues, 0), qbase(kQueues, 0);
+  for (int v = 0; v < nnodes; ++v) qcap[node_queue[v]] += 1;
+  for (int q = 1; q < kQueues; ++q) qbase[q] = qbase[q - 1] + qcap[q - 1];
+
+  std::vector<int> succ_off(nnodes + 1, 0), succ;
+  for (int v = 0; v < nnodes; ++v) {
+    succ_off[v + 1] = succ_off[v] + (int)B.succ[v].size();
+    succ.insert(succ.end(), B.succ[v].begin(), B.succ[v].end());
+  }
+  std::vector<int> roots;
+  for (int v = 0; v < nnodes; ++v)
+    if (B.deps[v] == 0) roots.push_back(v);
+
+  st->nnodes = nnodes;
+  st->njobs = (int)B.jobs.size();
+  st->h_job_type.resize(st->njobs);
+  st->h_job_paper.resize(st->njobs);
+  for (int j = 0; j < st->njobs; ++j) {
+    st->h_job_type[j] = B.jobs[j].type;
+    st->h_job_paper[j] = B.paper[B.job_node[j]];
+  }
+  st->nroots = (int)roots.size();
+
+  // ---- device layout: static (read-only) part
+  auto align = [](size_t x) { return (x + 255) & ~size_t(255); };
+  size_t off = 0;
+  const size_t o_jobs = off; off = align(off + B.jobs.size() * sizeof(Job));
+  const size_t o_jnode = off; off = align(off + B.job_node.size() * 4);
+  const size_t o_jbeg = off; off = align(off + nnodes * 4);
+  const size_t o_jcnt = off; off = align(off + nnodes * 4);
+  const size_t o_soff = off; off = align(off + (nnodes + 1) * 4);
+  const size_t o_succ = off; off = align(off + std::max<size_t>(succ.size(), 1) * 4);
+  const size_t o_paper = off; off = align(off + nnodes * 4);
+  const size_t o_nq = off; off = align(off + nnodes * 4);
+  const size_t o_qbase = off; off = align(off + kQueues * 4);
+  const size_t o_roots = off; off = align(off + std::max<size_t>(roots.size(), 1) * 4);
+  const size_t o_pub = off; off = align(off + (publish.empty() ? 4 : publish.size() * 4));
+  const size_t o_watch = off; off = align(off + std::max<size_t>(watch.size(), 1) * 16);
+  const size_t static_bytes = off;
+  std::vector<char> h(static_bytes, 0);
+  memcpy(h.data() + o_jobs, B.jobs.data(), B.jobs.size() * sizeof(Job));
+  memcpy(h.data() + o_jnode, B.job_node.data(), B.job_node.size() * 4);
+  memcpy(h.data() + o_jbeg, B.jbeg.data(), nnodes * 4);
+  memcpy(h.data() + o_jcnt, B.jcnt.data(), nnodes * 4);
+  memcpy(h.data() + o_soff, succ_off.data(), (nnodes + 1) * 4);
+  if (!succ.empty()) memcpy(h.data() + o_succ, succ.data(), succ.size() * 4);
+  memcpy(h.data() + o_paper, B.paper.data(), nnodes * 4);
+  memcpy(h.data() + o_nq, node_queue.data(), nnodes * 4);
+  memcpy(h.data() + o_qbase, qbase.data(), kQueues * 4);
+  if (!roots.empty()) memcpy(h.data() + o_roots, roots.data(), roots.size() * 4);
+  if (!publish.empty()) memcpy(h.data() + o_pub, publish.data(), publish.size() * 4);
+  if (!watch.empty()) memcpy(h.data() + o_watch, watch.data(), watch.size() * 16);
+
+  // dynamic part: node_deps, node_left, q_items, q_head, q_tail, done, finished
+  size_t doff = 0;
+  const size_t d_deps = doff; doff = align(doff + nnodes * 4);
+  const size_t d_left = doff; doff = align(doff + nnodes * 4);
+  const size_t pristine = doff;  // [0, pristine) is restored from the pristine copy
+  const size_t d_items = doff; doff = align(doff + (size_t)nnodes * 4);
+  const size_t d_next = doff; doff = align(doff + (size_t)nnodes * 4);
+  const size_t d_head = doff; doff = align(doff + kQueues * kQStride * 4);
+  const size_t d_tail = doff; doff = align(doff + kQueues * kQStride * 4);
+  const size_t d_done = doff; doff = align(doff + 4);
+  const size_t d_fin = doff; doff = align(doff + 4);
+  const size_t d_fired = doff; doff = align(doff + std::max<size_t>(watch.size(), 1) * 4);
+  std::vector<char> hp(pristine, 0);
+  memcpy(hp.data() + d_deps, B.deps.data(), nnodes * 4);
+  memcpy(hp.data() + d_left, B.jcnt.data(), nnodes * 4);
+
+  cudaError_t e;
+  if ((e = cudaMalloc(&st->dev_static, static_bytes)) || (e = cudaMalloc(&st->dev_dynamic, doff)) ||
+      (e = cudaMalloc(&st->dev_pristine, pristine))) {
+    cudaGetLastError();
+    sched_destroy(st);
+    return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
+  }
+  if ((e = cudaMemcpy(st->dev_static, h.data(), static_bytes, cudaMemcpyHostToDevice)) ||
+      (e = cudaMemcpy(st->dev_pristine, hp.data(), pristine, cudaMemcpyHostToDevice))) {
+    sched_destroy(st);
+    return -100 - (int)e;
+  }
+  st->dyn_bytes = doff;
+  st->pristine_bytes = pristine;
+  char* S = static_cast<char*>(st->dev_static);
+  char* D = static_cast<char*>(st->dev_dynamic);
+  DevSched& d = st->d;
+  d.jobs = reinterpret_cast<const Job*>(S + o_jobs);
+  d.job_node = reinterpret_cast<const int*>(S + o_jnode);
+  d.node_job_begin = reinterpret_cast<const int*>(S + o_jbeg);
+  d.node_job_count = reinterpret_cast<const int*>(S + o_jcnt);
+  d.succ_off = reinterpret_cast<const int*>(S + o_soff);
+  d.succ = reinterpret_cast<const int*>(S + o_succ);
+  d.node_paper = reinterpret_cast<const int*>(S + o_paper);
+  d.node_queue = reinterpret_cast<const int*>(S + o_nq);
+  d.q_base = reinterpret_cast<const int*>(S + o_qbase);
+  st->roots = reinterpret_cast<int*>(S + o_roots);
+  d.node_deps = reinterpret_cast<int*>(D + d_deps);
+  d.node_left = reinterpret_cast<int*>(D + d_left);
+  d.q_items = reinterpret_cast<int*>(D + d_items);
+  d.node_next = reinterpret_cast<int*>(D + d_next);
+  d.q_head = reinterpret_cast<int*>(D + d_head);
+  d.q_tail = reinterpret_cast<int*>(D + d_tail);
+  d.done_nodes = reinterpret_cast<int*>(D + d_done);
+  d.finished = reinterpret_cast<int*>(D + d_fin);
+  d.total_nodes = nnodes;
+  d.node_publish = publish.empty() ? nullptr : reinterpret_cast<const int*>(S + o_pub);
+  d.watch = reinterpret_cast<const int4*>(S + o_watch);
+  d.nwatch = (int)watch.size();
+  d.watch_fired = reinterpret_cast<int*>(D + d_fired);
+  d.nb = (int)nb;
+  st->nrecv_jobs = 0;
+  for (const Job& jb : B.jobs) st->nrecv_jobs += jb.type == J_RECV;
+  if (opts->trace == 2) {
+    if ((e = cudaMalloc(&st->job_trace, (size_t)st->njobs * 4 * sizeof(uint64_t)))) {
+      cudaGetLastError();
+      sched_destroy(st);
+      return -9;
+    }
+  }
+  d.job_trace = st->job_trace;
+  d.policy = opts->policy;
+  d.latency_workers = opts->policy == CHOL_POLICY_STATIC ? (opts->latency_workers > 0 ? opts->latency_workers : 16) : 0;
+
+  // ---- workers: one CTA per SM (all co-resident)
+  int per_sm = 0;
+  const int smem = smem_bytes(bs);
+  cudaError_t ea = cudaSuccess;
+  switch (bs) {
+    case 96: ea = cudaFuncSetAttribute(k_sched<96>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<96>, kWsThreads, smem); break;
+    case 64: ea = cudaFuncSetAttribute(k_sched<64>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<64>, kWsThreads, smem); break;
+    case 32: ea = cudaFuncSetAttribute(k_sched<32>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
+             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<32>, kWsThreads, smem); break;
+  }
+  if (ea || per_sm < 1) {
+    sched_destroy(st);
+    return ea ? -100 - (int)ea : -8;
+  }
+  st->workers = opts->workers > 0 ? std::min(opts->workers, sms * per_sm) : sms;
+  if (d.latency_workers >= st->workers) d.latency_workers = std::max(1, st->workers / 4);
+
+  {
+    // device memory, not host-mapped: the scheduler warps read it whenever they idle
+    cudaError_t ea = cudaMalloc(&st->d_abort, sizeof(int));
+    if (!ea) ea = cudaMemset(st->d_abort, 0, sizeof(int));
+    if (ea) {
+      sched_destroy(st);
+      return -100 - (int)ea;
+    }
+    st->d.abort_flag = st->d_abort;
+  }
+    *out = st;
+  return 0;
+}
+
 int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts,
-                 cudaStream_t s, const DistInfo* dist) {
+                 cudaStream_t /*s*/, const DistInfo* dist) {
   auto* st = new SchedState();
   const char* ear = getenv("CHOL_ARRIVAL");
   st->arrival = ear ? atoi(ear) : 0;
@@ -749,77 +1017,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     // shorter block DAG (CHOL_POTRF0_BLOCKDAG=0 turns this off; development switch)
     const bool pblock = potrf_blockdag || (k == 0 && potrf0_blockdag);
     if (mine(k, k) && !pblock && !blk) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
-      int prev = -1;
-      for (int b = 0; b < nbb; ++b) {
-        const int dn = B.add_node(pid, T_POTRF, k, k);
-        B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
-        if (prev >= 0) B.edge(prev, dn);
-        if (b == 0) first_node[pid] = dn;
-        prev = dn;
-        if (b + 1 < nbb) {
-          const int pn = B.add_node(pid, T_POTRF, k, k);
-          for (int r = b + 1; r < nbb; ++r)
-            B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
-          B.edge(prev, pn);
-          const int un = B.add_node(pid, T_POTRF, k, k);
-          for (int r = b + 1; r < nbb; ++r)
-            for (int q = b + 1; q <= r; ++q)
-              B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
-          B.edge(pn, un);
-          prev = un;
-        }
-      }
-      last_node[pid] = prev;
+      build_potrf_steps(B, k, pid, &first_node[pid], &last_node[pid]);
     } else if (mine(k, k)) {
-      // POTRF_k as a block-level DAG over the BS x BS blocks of the diagonal tile
-      // (right-looking nested Cholesky): D(b) = potf2 of block (b,b); P(r,b) = solve of
-      // block (r,b) against L_bb; U(r,q,b) = K=BS update of block (r,q) by blocks (r,b),
-      // (q,b).  One job per node, so the chain D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1)
-      // never waits for a whole column or trailing update of the step.  D(nbb-1) is the
-      // sink (every inner node is its ancestor).
-      // With potrf_fuse the chain's last update U(b,b,b-1) is done by D(b) itself: the job
-      // runs the J_PUPD code (producer stages, DMMA, epilogue) and then potf2 -- one node
-      // and one hop less per inner step, the same bits.
-      std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1), fusedP(nbb, -1);
-      if (blk) tentry[pid].assign(nbb2, -1), tfin[pid].assign(nbb2, -1);
-      for (int b = 0; b < nbb; ++b) {
-        const int dn = B.add_node(pid, T_POTRF, k, k);
-        B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)(fusedP[b] >= 0), 0, 0});
-        if (lastU[b * nbb + b] >= 0) B.edge(lastU[b * nbb + b], dn);
-        if (fusedP[b] >= 0) B.edge(fusedP[b], dn);
-        if (blk && b == 1 && fusedP[b] >= 0) tentry[pid][b * nbb + b] = dn;  // first touch of block (1,1)
-        if (b == 0) first_node[pid] = dn;
-        last_node[pid] = dn;
-        for (int r = b + 1; r < nbb; ++r) {
-          const int pn = B.add_node(pid, T_POTRF, k, k);
-          B.add_job(pn, Job{J_PANEL, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, 0, 0});
-          B.edge(dn, pn);
-          if (lastU[r * nbb + b] >= 0) B.edge(lastU[r * nbb + b], pn);
-          pan[r] = pn;
-        }
-        for (int r = b + 1; r < nbb; ++r)
-          for (int q = b + 1; q <= r; ++q) {
-            if (potrf_fuse && r == b + 1 && q == r) {  // U(b+1,b+1,b): fused into D(b+1)
-              fusedP[r] = pan[r];
-              continue;
-            }
-            const int un = B.add_node(pid, T_POTRF, k, k);
-            B.add_job(un, Job{J_PUPD, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)r, (int16_t)q, 0});
-            B.edge(pan[r], un);
-            if (q != r) B.edge(pan[q], un);
-            if (lastU[r * nbb + q] >= 0) B.edge(lastU[r * nbb + q], un);  // same block, previous step
-            lastU[r * nbb + q] = un;
-            if (blk && b == 0) tentry[pid][r * nbb + q] = un;
-          }
-        if (blk) {
-          tfin[pid][b * nbb + b] = dn;
-          if (b == 0) tentry[pid][0] = dn;
-          for (int r = b + 1; r < nbb; ++r) {
-            tfin[pid][r * nbb + b] = pan[r];
-            if (b == 0) tentry[pid][r * nbb] = pan[r];
-          }
-        }
-      }
+      build_potrf_blockdag(B, k, pid, potrf_fuse, blk, &tentry[pid], &tfin[pid], &first_node[pid], &last_node[pid]);
       if (blk && k == 0) gate_of(pid, T_POTRF, k, k);
     }
     for (int i = k + 1; i < N && blk; ++i) {
@@ -876,29 +1076,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         first_node[tid] = last_node[tid] = n;
         continue;
       }
-      if (!trsm_slabchain) {
-        // TRSM_i_k, right-looking over the BS-column blocks c of A_ik, one node per
-        // column step:  TS(c): A_ik[:, c] <- A_ik[:, c] L_kk[c,c]^{-T}  (nbb row-block jobs)
-        //               TU(c): A_ik[:, c'] -= A_ik[:, c] L_kk[c',c]^T, c' > c  (K = BS)
+      if (!trsm_slabchain) {  // right-looking column steps TS(c) / TU(c)
         const int tid = (int)id_trsm(N, i, k);
-        int prev_t = -1;
-        for (int cb = 0; cb < nbb; ++cb) {
-          const int ts = B.add_node(tid, T_TRSM, i, k);
-          for (int sl = 0; sl < nbb; ++sl)
-            B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
-          if (prev_t >= 0) B.edge(prev_t, ts);
-          if (cb == 0) first_node[tid] = ts;
-          prev_t = ts;
-          if (cb + 1 < nbb) {
-            const int tu = B.add_node(tid, T_TRSM, i, k);
-            for (int sl = 0; sl < nbb; ++sl)
-              for (int c2 = cb + 1; c2 < nbb; ++c2)
-                B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
-            B.edge(ts, tu);
-            prev_t = tu;
-          }
-        }
-        last_node[tid] = prev_t;
+        build_trsm_steps(B, i, k, tid, &first_node[tid], &last_node[tid]);
         continue;
       }
       // Alternative (CHOL_TRSM_SLABCHAIN=1): rows are independent (X L^{-T}), so each
@@ -1132,161 +1312,73 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     node_queue[v] = bucket + (pinned ? kBuckets : 0);
   }
 
-  // ---- queue capacities
-  std::vector<int> qcap(kQueues, 0), qbase(kQueues, 0);
-  for (int v = 0; v < nnodes; ++v) qcap[node_queue[v]] += 1;
-  for (int q = 1; q < kQueues; ++q) qbase[q] = qbase[q - 1] + qcap[q - 1];
+  return sched_upload(out, st, B, node_queue, publish, watch, opts, nb, bs, sms);
+}
 
-  std::vector<int> succ_off(nnodes + 1, 0), succ;
-  for (int v = 0; v < nnodes; ++v) {
-    succ_off[v + 1] = succ_off[v] + (int)B.succ[v].size();
-    succ.insert(succ.end(), B.succ[v].begin(), B.succ[v].end());
-  }
-  std::vector<int> roots;
-  for (int v = 0; v < nnodes; ++v)
-    if (B.deps[v] == 0) roots.push_back(v);
-
-  st->nnodes = nnodes;
-  st->njobs = (int)B.jobs.size();
-  st->h_job_type.resize(st->njobs);
-  st->h_job_paper.resize(st->njobs);
-  for (int j = 0; j < st->njobs; ++j) {
-    st->h_job_type[j] = B.jobs[j].type;
-    st->h_job_paper[j] = B.paper[B.job_node[j]];
-  }
-  st->nroots = (int)roots.size();
-
-  // ---- device layout: static (read-only) part
-  auto align = [](size_t x) { return (x + 255) & ~size_t(255); };
-  size_t off = 0;
-  const size_t o_jobs = off; off = align(off + B.jobs.size() * sizeof(Job));
-  const size_t o_jnode = off; off = align(off + B.job_node.size() * 4);
-  const size_t o_jbeg = off; off = align(off + nnodes * 4);
-  const size_t o_jcnt = off; off = align(off + nnodes * 4);
-  const size_t o_soff = off; off = align(off + (nnodes + 1) * 4);
-  const size_t o_succ = off; off = align(off + std::max<size_t>(succ.size(), 1) * 4);
-  const size_t o_paper = off; off = align(off + nnodes * 4);
-  const size_t o_nq = off; off = align(off + nnodes * 4);
-  const size_t o_qbase = off; off = align(off + kQueues * 4);
-  const size_t o_roots = off; off = align(off + std::max<size_t>(roots.size(), 1) * 4);
-  const size_t o_pub = off; off = align(off + (publish.empty() ? 4 : publish.size() * 4));
-  const size_t o_watch = off; off = align(off + std::max<size_t>(watch.size(), 1) * 16);
-  const size_t static_bytes = off;
-  std::vector<char> h(static_bytes, 0);
-  memcpy(h.data() + o_jobs, B.jobs.data(), B.jobs.size() * sizeof(Job));
-  memcpy(h.data() + o_jnode, B.job_node.data(), B.job_node.size() * 4);
-  memcpy(h.data() + o_jbeg, B.jbeg.data(), nnodes * 4);
-  memcpy(h.data() + o_jcnt, B.jcnt.data(), nnodes * 4);
-  memcpy(h.data() + o_soff, succ_off.data(), (nnodes + 1) * 4);
-  if (!succ.empty()) memcpy(h.data() + o_succ, succ.data(), succ.size() * 4);
-  memcpy(h.data() + o_paper, B.paper.data(), nnodes * 4);
-  memcpy(h.data() + o_nq, node_queue.data(), nnodes * 4);
-  memcpy(h.data() + o_qbase, qbase.data(), kQueues * 4);
-  if (!roots.empty()) memcpy(h.data() + o_roots, roots.data(), roots.size() * 4);
-  if (!publish.empty()) memcpy(h.data() + o_pub, publish.data(), publish.size() * 4);
-  if (!watch.empty()) memcpy(h.data() + o_watch, watch.data(), watch.size() * 16);
-
-  // dynamic part: node_deps, node_left, q_items, q_head, q_tail, done, finished
-  size_t doff = 0;
-  const size_t d_deps = doff; doff = align(doff + nnodes * 4);
-  const size_t d_left = doff; doff = align(doff + nnodes * 4);
-  const size_t pristine = doff;  // [0, pristine) is restored from the pristine copy
-  const size_t d_items = doff; doff = align(doff + (size_t)nnodes * 4);
-  const size_t d_next = doff; doff = align(doff + (size_t)nnodes * 4);
-  const size_t d_head = doff; doff = align(doff + kQueues * kQStride * 4);
-  const size_t d_tail = doff; doff = align(doff + kQueues * kQStride * 4);
-  const size_t d_done = doff; doff = align(doff + 4);
-  const size_t d_fin = doff; doff = align(doff + 4);
-  const size_t d_fired = doff; doff = align(doff + std::max<size_t>(watch.size(), 1) * 4);
-  std::vector<char> hp(pristine, 0);
-  memcpy(hp.data() + d_deps, B.deps.data(), nnodes * 4);
-  memcpy(hp.data() + d_left, B.jcnt.data(), nnodes * 4);
-
-  cudaError_t e;
-  if ((e = cudaMalloc(&st->dev_static, static_bytes)) || (e = cudaMalloc(&st->dev_dynamic, doff)) ||
-      (e = cudaMalloc(&st->dev_pristine, pristine))) {
-    cudaGetLastError();
-    sched_destroy(st);
-    return e == cudaErrorMemoryAllocation ? -9 : -100 - (int)e;
-  }
-  if ((e = cudaMemcpy(st->dev_static, h.data(), static_bytes, cudaMemcpyHostToDevice)) ||
-      (e = cudaMemcpy(st->dev_pristine, hp.data(), pristine, cudaMemcpyHostToDevice))) {
-    sched_destroy(st);
-    return -100 - (int)e;
-  }
-  st->dyn_bytes = doff;
-  st->pristine_bytes = pristine;
-  char* S = static_cast<char*>(st->dev_static);
-  char* D = static_cast<char*>(st->dev_dynamic);
-  DevSched& d = st->d;
-  d.jobs = reinterpret_cast<const Job*>(S + o_jobs);
-  d.job_node = reinterpret_cast<const int*>(S + o_jnode);
-  d.node_job_begin = reinterpret_cast<const int*>(S + o_jbeg);
-  d.node_job_count = reinterpret_cast<const int*>(S + o_jcnt);
-  d.succ_off = reinterpret_cast<const int*>(S + o_soff);
-  d.succ = reinterpret_cast<const int*>(S + o_succ);
-  d.node_paper = reinterpret_cast<const int*>(S + o_paper);
-  d.node_queue = reinterpret_cast<const int*>(S + o_nq);
-  d.q_base = reinterpret_cast<const int*>(S + o_qbase);
-  st->roots = reinterpret_cast<int*>(S + o_roots);
-  d.node_deps = reinterpret_cast<int*>(D + d_deps);
-  d.node_left = reinterpret_cast<int*>(D + d_left);
-  d.q_items = reinterpret_cast<int*>(D + d_items);
-  d.node_next = reinterpret_cast<int*>(D + d_next);
-  d.q_head = reinterpret_cast<int*>(D + d_head);
-  d.q_tail = reinterpret_cast<int*>(D + d_tail);
-  d.done_nodes = reinterpret_cast<int*>(D + d_done);
-  d.finished = reinterpret_cast<int*>(D + d_fin);
-  d.total_nodes = nnodes;
-  d.node_publish = publish.empty() ? nullptr : reinterpret_cast<const int*>(S + o_pub);
-  d.watch = reinterpret_cast<const int4*>(S + o_watch);
-  d.nwatch = (int)watch.size();
-  d.watch_fired = reinterpret_cast<int*>(D + d_fired);
-  d.nb = (int)nb;
-  st->nrecv_jobs = 0;
-  for (const Job& jb : B.jobs) st->nrecv_jobs += jb.type == J_RECV;
-  if (opts->trace == 2) {
-    if ((e = cudaMalloc(&st->job_trace, (size_t)st->njobs * 4 * sizeof(uint64_t)))) {
-      cudaGetLastError();
-      sched_destroy(st);
-      return -9;
+// Calibration batches (chol_run_batch; reading R9): `count` independent tasks of
+// one type on distinct output tiles, no edges -- POTRF on diagonal tiles 0..count-1,
+// TRSM_{i,k} over the N(N-1)/2 panel tiles in Algorithm 1 order (k, then i: enough
+// instances to saturate the GPU with row-slab jobs), SYRK_{c+1,0}, GEMM_{i,j,0} over the
+// pairs N > i > j >= 1 (j ascending, then i) -- run by the same persistent kernel as the factorization and in the
+// same job decompositions: the bulk forms when count > 1 (row-slab TRSM jobs; per-step POTRF
+// nodes wherever the factorization uses them), the critical-path forms when count == 1
+// (right-looking TRSM column steps, the POTRF block DAG).
+int sched_create_batch(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts, int type,
+                       int count) {
+  const int maxc = type == T_POTRF   ? (int)N
+                   : type == T_GEMM  ? (int)((N - 1) * (N - 2) / 2)
+                   : type == T_TRSM  ? (int)(N * (N - 1) / 2)
+                                     : (int)N - 1;
+  if (type < 0 || type > 3 || count < 1 || count > maxc) return -6;
+  auto* st = new SchedState();
+  st->N = N;
+  st->nb = nb;
+  st->bs = bs;
+  st->opts = *opts;
+  const int nbb = (int)(nb / bs);
+  Builder B{N, nbb, opts->policy, 1};
+  const char* epb = getenv("CHOL_POTRF_BLOCKDAG");
+  const bool potrf_blockdag = count == 1 || (epb ? atoi(epb) != 0 : N * N <= 256);
+  const char* epf = getenv("CHOL_POTRF_FUSE");
+  const bool potrf_fuse = !(epf && atoi(epf) == 0);
+  int first = -1, last = -1, c = 0;
+  if (type == T_POTRF) {
+    for (int k = 0; k < count; ++k) {
+      if (potrf_blockdag)
+        build_potrf_blockdag(B, k, -1, potrf_fuse, false, nullptr, nullptr, &first, &last);
+      else
+        build_potrf_steps(B, k, -1, &first, &last);
     }
-  }
-  d.job_trace = st->job_trace;
-  d.policy = opts->policy;
-  d.latency_workers = opts->policy == CHOL_POLICY_STATIC ? (opts->latency_workers > 0 ? opts->latency_workers : 16) : 0;
-
-  // ---- workers: one CTA per SM (all co-resident)
-  int per_sm = 0;
-  const int smem = smem_bytes(bs);
-  cudaError_t ea = cudaSuccess;
-  switch (bs) {
-    case 96: ea = cudaFuncSetAttribute(k_sched<96>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<96>, kWsThreads, smem); break;
-    case 64: ea = cudaFuncSetAttribute(k_sched<64>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<64>, kWsThreads, smem); break;
-    case 32: ea = cudaFuncSetAttribute(k_sched<32>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem);
-             if (!ea) ea = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_sched<32>, kWsThreads, smem); break;
-  }
-  if (ea || per_sm < 1) {
-    sched_destroy(st);
-    return ea ? -100 - (int)ea : -8;
-  }
-  st->workers = opts->workers > 0 ? std::min(opts->workers, sms * per_sm) : sms;
-  if (d.latency_workers >= st->workers) d.latency_workers = std::max(1, st->workers / 4);
-  (void)s;
-  {
-    // device memory, not host-mapped: the scheduler warps read it whenever they idle
-    cudaError_t ea = cudaMalloc(&st->d_abort, sizeof(int));
-    if (!ea) ea = cudaMemset(st->d_abort, 0, sizeof(int));
-    if (ea) {
-      sched_destroy(st);
-      return -100 - (int)ea;
+  } else if (type == T_TRSM) {
+    for (int k = 0; k < N && c < count; ++k)
+      for (int i = k + 1; i < N && c < count; ++i, ++c) {
+        if (count == 1) {
+          build_trsm_steps(B, i, k, -1, &first, &last);
+          continue;
+        }
+        const int n = B.add_node(-1, T_TRSM, i, k);
+        for (int sl = 0; sl < nbb; ++sl)
+          B.add_job(n, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
+      }
+  } else if (type == T_SYRK) {
+    for (int j = 1; j <= count; ++j) {
+      const int n = B.add_node(-1, T_SYRK, j, 0);
+      for (int bm = 0; bm < nbb; ++bm)
+        for (int bn = 0; bn <= bm; ++bn)
+          B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, 0, (int16_t)bm, (int16_t)bn, 0, 0});
     }
-    st->d.abort_flag = st->d_abort;
+  } else {
+    for (int j = 1; j < N && c < count; ++j)
+      for (int i = j + 1; i < N && c < count; ++i, ++c) {
+        const int g = B.add_node(-1, T_GEMM, i, 0);
+        for (int bm = 0; bm < nbb; ++bm)
+          for (int bn = 0; bn < nbb; ++bn)
+            B.add_job(g, Job{J_UPD, (int16_t)i, (int16_t)j, 0, (int16_t)bm, (int16_t)bn, 0, 0});
+      }
   }
-  *out = st;
-  return 0;
+  std::vector<int> node_queue(B.deps.size(), 0), publish;
+  std::vector<int4> watch;
+  return sched_upload(out, st, B, node_queue, publish, watch, opts, nb, bs, sms);
 }
 
 int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slot, double* const* d_peer_slots,

@@ -21,6 +21,10 @@ __host__ __device__ inline int tile_owner(int i, int j, int p, int q) { return (
 
 int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts, cudaStream_t s,
                  const DistInfo* dist = nullptr);
+// calibration batch: `count` independent tasks of one type (T_POTRF..T_GEMM) at step 0 on
+// distinct output tiles, run by the persistent kernel (chol_run_batch); -6 bad type / count
+int sched_create_batch(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const chol_opts_t* opts, int type,
+                       int count);
 // device pointers of the distributed plan, known after the IPC handle exchange
 int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slot, double* const* d_peer_slots,
                    int* const* d_peer_flags, int* d_my_flags);
