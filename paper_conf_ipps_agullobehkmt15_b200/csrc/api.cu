@@ -143,6 +143,7 @@ extern "C" int chol_destroy(chol_plan_t p) {
   }
   if (p->sched) sched_destroy(p->sched);
   cudaSetDevice(p->device);
+  sched_phase_dump();
   if (p->stream) cudaStreamSynchronize(p->stream);
   for (void* ptr : p->ipc_opened) cudaIpcCloseMemHandle(ptr);
   cudaFree(p->d_inv);

@@ -221,13 +221,14 @@ __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, i
 
 // ------------------------------------------------------------------ warp-specialised worker
 // CTA = 12 warps: warps 0-7 compute (setmaxnreg 232), warp 8 = TMA producer,
-// warp 9 = scheduler, warps 10-11 idle (control warpgroup, setmaxnreg 40).
+// warp 9 = scheduler, warp 10 = multi-GPU / streamed-input watcher (CTA 0), warp 11 = TMA-store
+// epilogue (storer); control warpgroup at setmaxnreg 40.
 // The scheduler pops the next job while the current one computes and does the
 // completion bookkeeping off the compute warps; the producer walks the same job
 // sequence through a 2-deep shared-memory job ring and issues every TMA load,
 // running ahead into the next job as soon as ring stages free up.
 constexpr int kWsThreads = 384;
-constexpr int kProdWarp = 8, kSchedWarp = 9;
+constexpr int kProdWarp = 8, kSchedWarp = 9, kStoreWarp = 11;
 constexpr int kRegsCompute = 232, kRegsControl = 40;
 
 __device__ __forceinline__ void write_desc(int4* slot, int job, const Job& jb, int skip) {
@@ -246,6 +247,21 @@ __device__ __forceinline__ void produce_range(Ctx<BS>& c, uint32_t& pit, int nst
 // scheduler warp): the scheduler claims job q+1 only once job q is fully issued, so a
 // freshly enqueued critical job waits behind at most the tail of a running job.
 __device__ __forceinline__ int* prod_issued_ptr(int4* jdesc) { return reinterpret_cast<int*>(jdesc + 6); }
+
+// The BS x BS output block (store tile, row, column) a K-loop job updates: the C block the
+// producer prefetches into lbuf and the storer writes back.  J_UPD / J_PUPD / J_TU.
+template <int BS>
+__device__ __forceinline__ void job_cblock(const Ctx<BS>& c, int type, const int4& d0, const int4& d1, int64_t* t,
+                                           int* r0, int* c0) {
+  if (type == J_UPD) {
+    *t = c.slot(d0.z, d0.w), *r0 = d1.y * BS, *c0 = d1.z * BS;
+  } else if (type == J_PUPD) {
+    *t = c.slot(d1.x, d1.x), *r0 = d1.z * BS, *c0 = d1.w * BS;
+  } else {  // J_TU
+    *t = c.slot(d0.z, d1.x), *r0 = d1.z * BS, *c0 = d1.w * BS;
+  }
+}
+__device__ __forceinline__ bool tma_store_job(int type) { return type == J_UPD || type == J_PUPD || type == J_TU; }
 
 template <int BS>
 __device__ void producer_loop(Ctx<BS>& c) {
@@ -272,16 +288,16 @@ __device__ void producer_loop(Ctx<BS>& c) {
           ta = c.slot(d0.z, d1.x); ra = d1.y * BS;
           tb = c.slot(d0.w, d1.x); rb = d1.z * BS;
           kb = 0; nst = c.nb / BK;
-          tcb = c.slot(d0.z, d0.w); cr = d1.y * BS; cc = d1.z * BS;
+          job_cblock(c, type, d0, d1, &tcb, &cr, &cc);
         } else if (type == J_PUPD) {  // POTRF update block (k, b, r, q)
-          ta = tb = tcb = c.slot(d1.x, d1.x);
+          ta = tb = c.slot(d1.x, d1.x);
           ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
-          cr = ra; cc = rb;
+          job_cblock(c, type, d0, d1, &tcb, &cr, &cc);
         } else {  // TRSM update (i, k, c, s, c'): A_ik[s, c'] -= A_ik[s, c] L_kk[c', c]^T
-          ta = tcb = c.slot(d0.z, d1.x);
+          ta = c.slot(d0.z, d1.x);
           tb = c.slot(d1.x, d1.x);
           ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
-          cr = ra; cc = rb;
+          job_cblock(c, type, d0, d1, &tcb, &cr, &cc);
         }
         // stages first (they only need ring space), then the C prefetch into lbuf once
         // the previous job has released lbuf, then the rest
@@ -312,6 +328,46 @@ __device__ void producer_loop(Ctx<BS>& c) {
     // never mark themselves issued: their worker claims its next job only when they end,
     // so a critical job is not captured by a worker busy for another 10-20 us
     if (!skip && (type == J_UPD || type == J_PUPD || type == J_TU || type == J_TRSM)) *issued = (int)q;
+  }
+}
+
+// ---- storer (warp 11, one lane): the TMA-store epilogue of the K-loop jobs.  The compute
+// warps stage C - acc in lbuf (epi_sub_stage), arrive on cready and go on with their next
+// job; the storer writes the block back with TMA (the same boxes the producer prefetched),
+// releases lbuf once the store has read it (lfree) and completes the job (jdone) once the
+// store has been performed -- only then does the scheduler warp release the successors.
+// For every other job it just adds its arrival to lfree and jdone (both count compute
+// warps + 1), after the previous job's lfree phase so its arrivals never run ahead.
+template <int BS>
+__device__ void storer_loop(Ctx<BS>& c) {
+  uint32_t q = 0, ns = 0;
+  while (true) {
+    const int e = q & 1;
+    mbar_wait(&c.jfull()[e], (q >> 1) & 1);
+    const int4 d0 = c.jdesc()[e * 3], d1 = c.jdesc()[e * 3 + 1];
+    const int job = d0.x, type = d0.y & 0xff, skip = d0.y >> 8;
+    if (job < 0) break;
+    if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
+    if (!skip && tma_store_job(type)) {
+      int64_t t;
+      int r0, c0;
+      job_cblock(c, type, d0, d1, &t, &r0, &c0);
+      mbar_wait(c.cready(), ns & 1);
+      ++ns;
+      const char* src = reinterpret_cast<const char*>(c.lbuf());
+#pragma unroll 1
+      for (int b = 0; b < BS / 16; ++b) tma_store_3d(c.map, src + b * BS * 128, c0 + 16 * b, r0, (int)t);
+      bulk_commit();
+      bulk_wait_read_all();
+      mbar_arrive(c.lfree());
+      bulk_wait_all();
+      fence_proxy_async();  // the async-proxy global writes before the generic release below
+      __threadfence();
+    } else {
+      mbar_arrive(c.lfree());
+    }
+    mbar_arrive(&c.jdone()[e]);
+    ++q;
   }
 }
 
@@ -383,6 +439,31 @@ __device__ void watcher_loop(const DevSched& d) {
   }
 }
 
+// ---- development instrumentation (build with -DCHOL_PHASES, tools/job_phases.sh): warp 0
+// of every CTA accumulates clock64 phases of the K = nb GEMM/SYRK block jobs -- [0] wait for
+// the job descriptor, [1] job start -> first stage full, [2] mainloop, [3] epilogue,
+// [4] epilogue end -> next descriptor wait, [5] job count; printed by chol_destroy.
+#ifdef CHOL_PHASES
+__device__ unsigned long long g_phase[8];
+__device__ __forceinline__ long long phase_clock() { return clock64(); }
+#define PHASE_ADD(i, v) \
+  if (threadIdx.x == 0) atomicAdd(&g_phase[i], (unsigned long long)(v))
+#else
+#define PHASE_ADD(i, v)
+#endif
+void sched_phase_dump() {
+#ifdef CHOL_PHASES
+  unsigned long long h[8];
+  cudaMemcpyFromSymbol(h, g_phase, sizeof(h));
+  const double nj = h[5] ? (double)h[5] : 1.0;
+  fprintf(stderr, "CHOL_PHASES jobs %llu  cycles/job: wait_desc %.0f  first_stage %.0f  mainloop %.0f  epilogue %.0f  "
+          "to_next %.0f  (drain of the DMMA queue, inside epilogue: %.0f)\n", h[5], h[0] / nj, h[1] / nj, h[2] / nj,
+          h[3] / nj, h[4] / nj, h[6] / nj);
+  const unsigned long long z[8] = {};
+  cudaMemcpyToSymbol(g_phase, z, sizeof(z));
+#endif
+}
+
 // ---- compute warps: run the job's consumer side
 template <int BS>
 __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int type, const int4& d0, const int4& d1,
@@ -392,14 +473,34 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
   if (type == J_UPD) {
     Acc<BS> acc;
     const int i = d0.z, j = d0.w, k = d1.x, bm = d1.y, bn = d1.z;
+#ifdef CHOL_PHASES
+    const long long p0 = phase_clock();
+    mbar_wait(&c.full()[c.it % kStages], (c.it / kStages) & 1);
+    const long long p1 = phase_clock();
+#endif
     gemm_consume(c, c.nb / BK, acc);
-    epi_sub_global(c, acc, c.tile(i, j) + (int64_t)bm * BS * c.nb + bn * BS, c.nb, i == j && bm == bn);
+#ifdef CHOL_PHASES
+    const long long p2 = phase_clock();
+    {  // wait for the last-issued DMMA (its accumulator) -> drain of the DMMA queue
+      volatile double sink = acc[Cfg<BS>::MI - 1][Cfg<BS>::NI - 1][1] + acc[0][0][0];
+      (void)sink;
+      PHASE_ADD(6, phase_clock() - p2);
+    }
+#endif
+    epi_sub_stage(c, acc, i == j && bm == bn);
+#ifdef CHOL_PHASES
+    const long long p3 = phase_clock();
+    PHASE_ADD(1, p1 - p0);
+    PHASE_ADD(2, p2 - p1);
+    PHASE_ADD(3, p3 - p2);
+    PHASE_ADD(5, 1);
+#endif
     (void)k;
   } else if (type == J_PUPD) {
     Acc<BS> acc;
-    const int k = d1.x, r = d1.z, q = d1.w;
+    const int r = d1.z, q = d1.w;
     gemm_consume(c, BS / BK, acc);
-    epi_sub_global(c, acc, c.tile(k, k) + (int64_t)r * BS * c.nb + q * BS, c.nb, r == q);
+    epi_sub_stage(c, acc, r == q);
   } else if (type == J_TRSM) {
     Acc<BS> acc;
     const int i = d0.z, k = d1.x, slab = d1.y, nbb = c.nb / BS;
@@ -420,9 +521,8 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     }
   } else if (type == J_TU) {
     Acc<BS> acc;
-    const int i = d0.z, k = d1.x, sl = d1.z, c2 = d1.w;
     gemm_consume(c, BS / BK, acc);
-    epi_sub_global(c, acc, c.tile(i, k) + (int64_t)sl * BS * c.nb + c2 * BS, c.nb, false);
+    epi_sub_stage(c, acc, false);
   } else if (type == J_TS) {
     const int i = d0.z, k = d1.x, cb = d1.y, sl = d1.z;
     solve_block_job<BS>(c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
@@ -447,9 +547,22 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
 template <int BS>
 __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
   uint32_t q = 0;
+#ifdef CHOL_PHASES
+  long long t_end = 0;
+  bool last_upd = false;
+#endif
   while (true) {
     const int e = q & 1;
+#ifdef CHOL_PHASES
+    const long long w0 = phase_clock();
+#endif
     mbar_wait(&c.jfull()[e], (q >> 1) & 1);
+#ifdef CHOL_PHASES
+    if (last_upd) {
+      PHASE_ADD(0, phase_clock() - w0);
+      PHASE_ADD(4, w0 - t_end);
+    }
+#endif
     const int4 d0 = c.jdesc()[e * 3], d1 = c.jdesc()[e * 3 + 1];
     if (d0.x < 0) break;
     if (c.warp == 0 && c.lane == 0) {
@@ -457,7 +570,18 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
       c.jdesc()[e * 3 + 2] = make_int4((int)(t0 & 0xffffffffull), (int)(t0 >> 32), 0, 0);
     }
     const int type = d0.y & 0xff, skip = d0.y >> 8;
+    // jobs that use lbuf directly (in-block solves, potf2, the fused update's C block is
+    // prefetched behind lfree anyway) wait until the previous job's TMA store has read it
+    if (!skip && q > 0 && (type == J_TRSM || type == J_TS || type == J_PANEL || type == J_DIAG))
+      mbar_wait(c.lfree(), (q - 1) & 1);
     if (!skip) compute_job(c, d, type, d0, d1, info);
+    if (!skip && tma_store_job(type)) {
+      __syncwarp();
+      if (c.lane == 0) mbar_arrive(c.cready());  // C - acc staged: the storer takes over
+    }
+#ifdef CHOL_PHASES
+    last_upd = !skip && type == J_UPD;
+#endif
     __syncwarp();
     if (c.lane == 0) {
       mbar_arrive(c.lfree());  // lbuf (C block / L block / rdiag) no longer needed
@@ -469,6 +593,9 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
       mbar_arrive(&c.jdone()[e]);  // the job's global stores precede this release
     }
     ++q;
+#ifdef CHOL_PHASES
+    t_end = phase_clock();
+#endif
   }
 }
 
@@ -571,6 +698,8 @@ __global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__
       scheduler_loop(c, d, sp, latency_worker);
     } else if (c.warp == kSchedWarp + 1 && blockIdx.x == 0 && d.nwatch > 0) {
       watcher_loop(d);
+    } else if (c.warp == kStoreWarp) {
+      if (c.lane == 0) storer_loop(c);
     }
     return;
   }
@@ -578,8 +707,11 @@ __global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__
   compute_loop(c, d, sp.info);
 }
 
+// Roots pushed in parallel (a calibration batch has up to ~1100 roots: one thread took
+// 70 us); their order within a queue is a scheduling choice, never a numerical one (R15).
 __global__ void k_sched_init(DevSched d, const int* roots, int nroots) {
-  for (int r = 0; r < nroots; ++r) ready_node(d, roots[r]);
+  for (int r = blockIdx.x * blockDim.x + threadIdx.x; r < nroots; r += gridDim.x * blockDim.x)
+    ready_node(d, roots[r]);
 }
 
 // ------------------------------------------------------------------ host planner
@@ -1404,7 +1536,7 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
   st->d.tr_base = base.tr_base;
   if (!base.tr_base) st->d.job_trace = nullptr;  // job trace needs the time base
   else st->d.job_trace = st->job_trace;
-  k_sched_init<<<1, 1, 0, s>>>(st->d, st->roots, st->nroots);
+  k_sched_init<<<std::max(1, std::min(64, (st->nroots + 127) / 128)), 128, 0, s>>>(st->d, st->roots, st->nroots);
   const int smem = smem_bytes(st->bs);
   switch (st->bs) {
     case 96: k_sched<96><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;

@@ -80,7 +80,8 @@ struct Ctx {
   __device__ uint64_t* jdone() const { return jfull() + 2; } // [2] job finished (compute -> scheduler)
   __device__ uint64_t* lfree() const { return jdone() + 2; } // lbuf released (compute -> producer)
   __device__ uint64_t* tstep() const { return lfree() + 1; } // TRSM column block stored (compute -> producer)
-  // 2*kStages + 7 = 17 barriers = 136 bytes; then 2 x 3 int4 job descriptors + producer progress word
+  __device__ uint64_t* cready() const { return tstep() + 1; } // C - acc staged in lbuf (compute -> storer)
+  // 2*kStages + 8 = 18 barriers = 144 bytes; then 2 x 3 int4 job descriptors + producer progress word
   __device__ int4* jdesc() const { return reinterpret_cast<int4*>(bars() + 160); }
   uint32_t it;     // stages consumed so far
   uint32_t cphase; // parity of the next cbar completion
@@ -115,12 +116,15 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
       mbar_init(&c.empty()[s], kComputeWarps);
     }
     mbar_init(c.cbar(), 1);
+    // persistent kernel: jdone / lfree complete when the compute warps AND the storer warp
+    // (TMA-store epilogue, sched.cu) have arrived
     for (int e = 0; e < 2; ++e) {
       mbar_init(&c.jfull()[e], 1);
-      mbar_init(&c.jdone()[e], kComputeWarps);
+      mbar_init(&c.jdone()[e], kComputeWarps + 1);
     }
-    mbar_init(c.lfree(), kComputeWarps);
+    mbar_init(c.lfree(), kComputeWarps + 1);
     mbar_init(c.tstep(), kComputeWarps);
+    mbar_init(c.cready(), kComputeWarps);
     fence_mbar_init();
   }
   if (c.issuer() && map) tma_prefetch_desc(map);
@@ -350,6 +354,40 @@ __device__ __forceinline__ void epi_sub_global(Ctx<BS>& c, const Acc<BS>& acc, d
         if (cc + 1 <= r) __stcg(&p->y, v.y);
       }
     }
+}
+
+// Persistent kernel (sched.cu): C - acc staged IN PLACE in lbuf, the TMA-prefetched C block
+// (BS/16 boxes of BS rows x 128 B, 128B-swizzled -- the layout a TMA store of the same boxes
+// reads back), for the storer warp's TMA store; the compute warps do not wait for it.
+// lower_only: the strictly upper part of the block keeps C, so the stored block leaves
+// memory exactly as epi_sub_global's lower-only stores do.  Ends with the cross-proxy
+// fence; the caller arrives on cready.
+template <int BS>
+__device__ __forceinline__ void epi_sub_stage(Ctx<BS>& c, const Acc<BS>& acc, bool lower_only) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  mbar_wait(c.cbar(), c.cphase);
+  c.cphase ^= 1;
+  const uint32_t cs = smem_u32(c.lbuf());
+  double2 cv[C::MI][C::NI];
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
+      cv[mi][ni] = lds128(cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4));
+    }
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
+      double2 v = cv[mi][ni];
+      if (!lower_only || cc <= r) v.x -= acc[mi][ni][0];
+      if (!lower_only || cc + 1 <= r) v.y -= acc[mi][ni][1];
+      sts128(cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4), v);
+    }
+  fence_proxy_async_shared();  // generic smem writes -> the TMA store (async proxy)
 }
 
 // dst[r*P + c] = src[r*ld + c] for a BS x BS block: 16-byte chunks, every load of
