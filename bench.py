@@ -238,8 +238,10 @@ def calibrate(c, args):
     persistent scheduler kernel (chol_run_batch on a scheduler plan of the same n, nb):
 
     T_thr (area term): device time per task in a saturating batch of independent tasks of
-    the type, in the factorization's bulk decomposition -- all (N-1)(N-2)/2 GEMM_i_j_0, the
-    N(N-1)/2 TRSM_i_k row-slab tasks, the N-1 SYRK_j_0, the N POTRFs.
+    the type, in the factorization's bulk decomposition -- up to (N-1)(N-2)/2 GEMM_i_j_0,
+    N(N-1)/2 TRSM_i_k row-slab tasks, N-1 SYRK_j_0, N POTRFs -- taken as the marginal cost
+    of a task (batch of c tasks minus batch of c/2, divided by c/2), so the launch, the
+    ramp-up and the last partial wave of the batch are not charged to the tasks.
     T_lat (path terms): one task alone on the idle GPU, in the critical-path decomposition
     (TRSM column steps, the POTRF block DAG).  Neither is taken from the factorization
     being bounded."""
@@ -250,7 +252,14 @@ def calibrate(c, args):
     with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=POLICIES[args.policy]) as p:
         c.chol_generate(p.h, args.seed, 0)
         for t in range(4):
-            T_thr.append(c.chol_run_batch(p.h, t, max(counts[t], 1), 2) * 1e-3)
+            full = max(counts[t], 1)
+            half = full // 2
+            t_full = c.chol_run_batch(p.h, t, full, 3) * 1e-3 * full
+            if half >= 1:
+                t_half = c.chol_run_batch(p.h, t, half, 3) * 1e-3 * half
+                T_thr.append((t_full - t_half) / (full - half))
+            else:
+                T_thr.append(t_full / full)
             T_lat.append(c.chol_run_batch(p.h, t, 1, 5) * 1e-3)
     return T_lat, T_thr
 

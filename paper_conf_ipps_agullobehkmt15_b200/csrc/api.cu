@@ -29,6 +29,8 @@ struct chol_plan_s {
   cudaStream_t stream = nullptr;
   double* tiles = nullptr;
   CUtensorMap map{};
+  double* d_dinv = nullptr;  // inverse-form TRSM: inverses of the diagonal blocks of every L_kk
+  CUtensorMap dmap{};
   int* d_info = nullptr;
   uint64_t* d_base = nullptr;
   uint64_t* d_t0 = nullptr;
@@ -88,21 +90,36 @@ typedef CUresult (*PFN_encodeTiled_t)(CUtensorMap*, CUtensorMapDataType, cuuint3
                                       const cuuint64_t*, const cuuint32_t*, const cuuint32_t*, CUtensorMapInterleave,
                                       CUtensorMapSwizzle, CUtensorMapL2promotion, CUtensorMapFloatOOBfill);
 
-static int encode_tile_map(chol_plan_s* p) {
+// 3-D map over `count` row-major d x d FP64 blocks, box {16, bs, 1}, 128-byte swizzle
+static int encode_blocks_map(CUtensorMap* map, double* base, int64_t d, int64_t count, int bs) {
   void* fn = nullptr;
   cudaDriverEntryPointQueryResult q;
   CUDA_TRY(cudaGetDriverEntryPoint("cuTensorMapEncodeTiled", &fn, cudaEnableDefault, &q));
   if (!fn || q != cudaDriverEntryPointSuccess) return -100 - (int)cudaErrorNotSupported;
   auto encode = reinterpret_cast<PFN_encodeTiled_t>(fn);
-  const cuuint64_t dims[3] = {(cuuint64_t)p->nb, (cuuint64_t)p->nb, (cuuint64_t)p->ntiles};
-  const cuuint64_t strides[2] = {(cuuint64_t)p->nb * 8, (cuuint64_t)p->nb * p->nb * 8};
-  const cuuint32_t box[3] = {16, (cuuint32_t)p->bs, 1};
+  const cuuint64_t dims[3] = {(cuuint64_t)d, (cuuint64_t)d, (cuuint64_t)count};
+  const cuuint64_t strides[2] = {(cuuint64_t)d * 8, (cuuint64_t)d * d * 8};
+  const cuuint32_t box[3] = {16, (cuuint32_t)bs, 1};
   const cuuint32_t estr[3] = {1, 1, 1};
-  CUresult r = encode(&p->map, CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 3, p->tiles, dims, strides, box, estr,
+  CUresult r = encode(map, CU_TENSOR_MAP_DATA_TYPE_FLOAT64, 3, base, dims, strides, box, estr,
                       CU_TENSOR_MAP_INTERLEAVE_NONE, CU_TENSOR_MAP_SWIZZLE_128B, CU_TENSOR_MAP_L2_PROMOTION_L2_256B,
                       CU_TENSOR_MAP_FLOAT_OOB_FILL_NONE);
   if (r != CUDA_SUCCESS) return -100 - (int)cudaErrorInvalidValue;
   return 0;
+}
+static int encode_tile_map(chol_plan_s* p) { return encode_blocks_map(&p->map, p->tiles, p->nb, p->ntiles, p->bs); }
+
+// Dinv workspace of the inverse-form TRSM row slabs (sched.cu J_INV / J_TRSM): N * nb/bs
+// blocks of bs x bs (35 MB at n = 46080), and its map
+static int make_dinv(chol_plan_s* p) {
+  const int64_t nblk = p->N * (p->nb / p->bs);
+  cudaError_t e = cudaMalloc(&p->d_dinv, (size_t)nblk * p->bs * p->bs * sizeof(double));
+  if (e == cudaErrorMemoryAllocation) {
+    cudaGetLastError();
+    return -9;
+  }
+  if (e) return -100 - (int)e;
+  return encode_blocks_map(&p->dmap, p->d_dinv, p->bs, nblk, p->bs);
 }
 
 // ------------------------------------------------------------------ errors
@@ -164,6 +181,7 @@ extern "C" int chol_destroy(chol_plan_t p) {
   if (p->s_in) cudaStreamDestroy(p->s_in);
   if (p->s_out) cudaStreamDestroy(p->s_out);
   cudaFree(p->tiles);
+  cudaFree(p->d_dinv);
   cudaFree(p->d_info);
   cudaFree(p->d_base);
   cudaFree(p->d_t0);
@@ -245,9 +263,11 @@ extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t*
   for (cudaEvent_t* ev : {&p->ev0, &p->ev1, &p->ev2, &p->ev3})
     if ((e = cudaEventCreate(ev))) return fail(-100 - (int)e);
   if ((st = encode_tile_map(p))) return fail(st);
+  if ((st = make_dinv(p))) return fail(st);
   if ((e = prepare_kernels(p->bs))) return fail(-100 - (int)e);
   if (opts.executor == CHOL_EXEC_SCHEDULER) {
     if ((st = sched_create(&p->sched, p->N, p->nb, p->bs, p->sms, &p->opts, p->stream))) return fail(st);
+    sched_set_dinv(p->sched, p->d_dinv, p->dmap);
     // arrival flags (device), publish flags (host-mapped, polled by chol_factor), copy streams
     if ((e = cudaMalloc(&p->d_in_flags, p->ntiles * sizeof(int))) ||
         (e = cudaHostAlloc(&p->h_out_flags, p->ntiles * sizeof(int), cudaHostAllocMapped)) ||
@@ -360,6 +380,8 @@ extern "C" int chol_plan_dist(int64_t n, int64_t nb, int nranks, int rank, const
   if ((e = prepare_kernels(p->bs))) return fail(-100 - (int)e);
   DistInfo di{p->p, p->q, rank, nranks, p->h_slot_map.data()};
   if ((st = sched_create(&p->sched, p->N, p->nb, p->bs, p->sms, &p->opts, p->stream, &di))) return fail(st);
+  if ((st = make_dinv(p))) return fail(st);
+  sched_set_dinv(p->sched, p->d_dinv, p->dmap);
   *out = p;
   return 0;
 }
@@ -724,6 +746,7 @@ static StepParams base_params(chol_plan_s* p) {
   sp.nb = (int)p->nb;
   sp.N = (int)p->N;
   sp.info = p->d_info;
+  sp.dinv = p->d_dinv;
   if (p->opts.trace) {
     sp.tr_t0 = p->d_t0;
     sp.tr_t1 = p->d_t1;
@@ -741,7 +764,7 @@ static int run_host_sequenced(chol_plan_s* p, int* nlaunch) {
     CUDA_TRY(launch_potrf(p->bs, p->map, sp, 1, p->stream, nlaunch));
     if (k == N - 1) break;
     sp.i0 = k + 1;
-    CUDA_TRY(launch_trsm(p->bs, p->map, sp, N - 1 - k, p->stream, nlaunch));
+    CUDA_TRY(launch_trsm(p->bs, p->map, p->dmap, sp, N - 1 - k, p->stream, nlaunch));
     const int m = N - 1 - k;
     sp.mode = 0;
     CUDA_TRY(launch_update(p->bs, p->map, sp, m * (m + 1) / 2, p->stream, nlaunch));
@@ -1287,7 +1310,7 @@ extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int r
       CUDA_TRY(launch_potrf(p->bs, p->map, sp, 1, p->stream, &nl));
     } else if (type == T_TRSM) {
       sp.i0 = i;
-      CUDA_TRY(launch_trsm(p->bs, p->map, sp, 1, p->stream, &nl));
+      CUDA_TRY(launch_trsm(p->bs, p->map, p->dmap, sp, 1, p->stream, &nl));
     } else {
       sp.mode = 1;
       sp.i0 = (type == T_SYRK) ? j : i;
@@ -1324,6 +1347,7 @@ extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, doub
   if (p->sched) {  // the persistent scheduler, the factorization's own executor (reading R9)
     SchedState* bst = nullptr;
     if (const int st = sched_create_batch(&bst, p->N, p->nb, p->bs, p->sms, &p->opts, type, count)) return st;
+    sched_set_dinv(bst, p->d_dinv, p->dmap);
     int st = 0;
     for (int r = 0; r <= reps && !st; ++r) {  // r = 0: untimed warm-up
       if (r == 1) CUDA_TRY(cudaEventRecord(p->ev0, p->stream));
@@ -1345,7 +1369,7 @@ extern "C" int chol_run_batch(chol_plan_t p, int type, int count, int reps, doub
       CUDA_TRY(launch_potrf(p->bs, p->map, sp, count, p->stream, &nl));
     } else if (type == T_TRSM) {
       sp.i0 = 1;
-      CUDA_TRY(launch_trsm(p->bs, p->map, sp, count, p->stream, &nl));
+      CUDA_TRY(launch_trsm(p->bs, p->map, p->dmap, sp, count, p->stream, &nl));
     } else {
       sp.mode = type == T_GEMM ? 2 : 3;
       CUDA_TRY(launch_update(p->bs, p->map, sp, count, p->stream, &nl));

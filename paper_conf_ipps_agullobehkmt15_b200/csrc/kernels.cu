@@ -61,14 +61,23 @@ __global__ void __launch_bounds__(kThreads, 1) k_potrf_update(const __grid_const
 }
 
 // ------------------------------------------------------------------ TRSM batch
+// inverses of the diagonal blocks of L_kk (blockIdx.x = b), for the inverse-form slabs
+template <int BS>
+__global__ void __launch_bounds__(kThreads, 1) k_inv(const __grid_constant__ CUtensorMap map, StepParams p) {
+  auto c = make_ctx<BS>(&map, p.tiles, p.nb, p.N);
+  const int nbb = p.nb / BS, b = blockIdx.x;
+  inv_block(c, c.tile(p.k, p.k) + (int64_t)b * BS * p.nb + b * BS, p.nb, p.dinv + ((int64_t)p.k * nbb + b) * BS * BS);
+}
+
 // blockIdx.x = task * nbb + slab, task -> i = i0 + task (all with the same k)
 template <int BS>
-__global__ void __launch_bounds__(kThreads, 1) k_trsm(const __grid_constant__ CUtensorMap map, StepParams p) {
+__global__ void __launch_bounds__(kThreads, 1) k_trsm(const __grid_constant__ CUtensorMap map,
+                                                      const __grid_constant__ CUtensorMap dmap, StepParams p) {
   const uint64_t t0 = trace_now(p);
   auto c = make_ctx<BS>(&map, p.tiles, p.nb, p.N);
   const int nbb = p.nb / BS;
   const int i = p.i0 + blockIdx.x / nbb, slab = blockIdx.x % nbb;
-  sub_trsm(c, i, p.k, slab);
+  sub_trsm_inv(c, &dmap, i, p.k, slab);
   trace_record(p, id_trsm(p.N, i, p.k), t0);
 }
 
@@ -204,6 +213,7 @@ static cudaError_t set_attrs() {
   if ((e = cudaFuncSetAttribute(k_potrf_panel<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
   if ((e = cudaFuncSetAttribute(k_potrf_update<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
   if ((e = cudaFuncSetAttribute(k_trsm<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
+  if ((e = cudaFuncSetAttribute(k_inv<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
   if ((e = cudaFuncSetAttribute(k_update<BS>, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes))) return e;
   return cudaSuccess;
 }
@@ -226,10 +236,12 @@ static int launch_potrf_t(const CUtensorMap& map, StepParams p, int count, cudaS
 }
 
 template <int BS>
-static int launch_trsm_t(const CUtensorMap& map, StepParams p, int count, cudaStream_t s, int* nlaunch) {
+static int launch_trsm_t(const CUtensorMap& map, const CUtensorMap& dmap, StepParams p, int count, cudaStream_t s,
+                         int* nlaunch) {
   const int nbb = p.nb / BS;
-  k_trsm<BS><<<count * nbb, kThreads, Cfg<BS>::kSmemBytes, s>>>(map, p);
-  ++*nlaunch;
+  k_inv<BS><<<nbb, kThreads, Cfg<BS>::kSmemBytes, s>>>(map, p);
+  k_trsm<BS><<<count * nbb, kThreads, Cfg<BS>::kSmemBytes, s>>>(map, dmap, p);
+  *nlaunch += 2;
   return 0;
 }
 
@@ -271,8 +283,9 @@ cudaError_t launch_potrf(int bs, const CUtensorMap& map, const StepParams& p, in
 #undef L
   return cudaGetLastError();
 }
-cudaError_t launch_trsm(int bs, const CUtensorMap& map, const StepParams& p, int count, cudaStream_t s, int* nl) {
-#define L(B) launch_trsm_t<B>(map, p, count, s, nl)
+cudaError_t launch_trsm(int bs, const CUtensorMap& map, const CUtensorMap& dmap, const StepParams& p, int count,
+                        cudaStream_t s, int* nl) {
+#define L(B) launch_trsm_t<B>(map, dmap, p, count, s, nl)
   CHOL_DISPATCH(bs, L)
 #undef L
   return cudaGetLastError();

@@ -33,13 +33,17 @@ constexpr int kBuckets = 64;           // priority buckets per queue class
 constexpr int kQueues = 2 * kBuckets;  // [0, 64) normal, [64, 128) pinned
 constexpr int kQStride = 32;           // ints between queue heads (separate 128B lines)
 
-// Job types: J_UPD GEMM/SYRK block (K = nb); J_TRSM row slab (left-looking, unused by the
+// Job types: J_UPD GEMM/SYRK block (K = nb); J_TRSM row slab (left-looking, inverse form:
+// per column block one GEMM over the solved blocks and one product with Dinv); J_INV
+// Dinv_b = inv(L_kk[b, b]) for the slabs (one per diagonal block of L_kk); (older text:
 // default plan); POTRF inner: J_DIAG potf2 of block (b,b), J_PANEL solve of block (r,b),
 // J_PUPD K=BS update of block (r,q); TRSM right-looking: J_TS solve of block (s,c) of
 // A_ik against L_kk[c,c], J_TU K=BS update A_ik[s,c'] -= A_ik[s,c] L_kk[c',c]^T.
 // Multi-GPU: J_RECV copies row slab a of remote panel tile (i, j) from its owner b (peer
 // memory over NVLink) into this rank's cache slot.
-enum JobType : int16_t { J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6, J_RECV = 7 };
+enum JobType : int16_t {
+  J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6, J_RECV = 7, J_INV = 8
+};
 struct Job {
   int16_t type, i, j, k, a, b, c, pad;
 };
@@ -80,6 +84,7 @@ struct DevSched {
   int nwatch;
   unsigned epoch;             // factorization number (flags hold the epoch they became final in)
   int nb;
+  double* dinv;               // [N][nb/BS] BS x BS inverses of the diagonal blocks of each L_kk (J_INV)
 };
 
 // ------------------------------------------------------------------ device queue ops
@@ -257,15 +262,19 @@ __device__ __forceinline__ void job_cblock(const Ctx<BS>& c, int type, const int
     *t = c.slot(d0.z, d0.w), *r0 = d1.y * BS, *c0 = d1.z * BS;
   } else if (type == J_PUPD) {
     *t = c.slot(d1.x, d1.x), *r0 = d1.z * BS, *c0 = d1.w * BS;
-  } else {  // J_TU
+  } else if (type == J_TU) {
     *t = c.slot(d0.z, d1.x), *r0 = d1.z * BS, *c0 = d1.w * BS;
+  } else {  // J_TS: block (sl, cb) of A_ik
+    *t = c.slot(d0.z, d1.x), *r0 = d1.z * BS, *c0 = d1.y * BS;
   }
 }
-__device__ __forceinline__ bool tma_store_job(int type) { return type == J_UPD || type == J_PUPD || type == J_TU; }
+__device__ __forceinline__ bool tma_store_job(int type) {
+  return type == J_UPD || type == J_PUPD || type == J_TU || type == J_TS;
+}
 
 template <int BS>
-__device__ void producer_loop(Ctx<BS>& c) {
-  uint32_t q = 0, pit = 0, tcount = 0;
+__device__ void producer_loop(Ctx<BS>& c, const CUtensorMap* dmap) {
+  uint32_t q = 0, pit = 0, tcount = 0, scount = 0;
   volatile int* issued = prod_issued_ptr(c.jdesc());
   while (true) {
     const int e = q & 1;
@@ -306,20 +315,50 @@ __device__ void producer_loop(Ctx<BS>& c) {
         prefetch_c_issue(c, tcb, cr, cc);
         produce_range(c, pit, nst, ta, ra, tb, rb, kb, kStages, nst);
         pit += nst;
-      } else if (type == J_TRSM) {  // row slab (i, k, slab): mainloop cb reads X[:, :cb] (solved)
-        const int nbb = c.nb / BS;
-        for (int cb = 1; cb < nbb; ++cb) {
-          // K chunks of the column blocks solved before cb-1 are final already: stream
-          // them into the ring while the compute warps still solve block cb-1; only the
-          // last BS/BK stages (column block cb-1) wait for its tstep.  Same K order.
-          const int nst = cb * BS / BK, nold = (cb - 1) * BS / BK;
-          const int64_t ta = c.slot(d0.z, d1.x), tb = c.slot(d1.x, d1.x);
-          produce_range(c, pit, nst, ta, d1.y * BS, tb, cb * BS, 0, 0, nold);
-          mbar_wait(c.tstep(), tcount & 1);
-          ++tcount;
-          fence_proxy_async();
-          produce_range(c, pit, nst, ta, d1.y * BS, tb, cb * BS, 0, nold, nst);
-          pit += nst;
+      } else if (type == J_TS) {
+        // TS(cb, sl), inverse form: A_ik[sl, cb] Dinv_{k,cb}^T, K = BS -- A stages from the
+        // tile store, B stages from the Dinv workspace; no C block (the result overwrites)
+        using Cf = Cfg<BS>;
+        const int64_t ta = c.slot(d0.z, d1.x);
+        const int nbb = c.nb / BS, k = d1.x, cb = d1.y, ra = d1.z * BS;
+        for (int s2 = 0; s2 < BS / BK; ++s2) {
+          const uint32_t qq = pit + s2, st = qq % kStages, ph = (qq / kStages) & 1;
+          mbar_wait(&c.empty()[st], ph ^ 1);
+          mbar_arrive_expect_tx(&c.full()[st], 2 * Cf::kOpBytes);
+          char* sa = c.pipe() + st * 2 * Cf::kOpBytes;
+          tma_load_3d(sa, c.map, &c.full()[st], cb * BS + s2 * BK, ra, (int)ta);
+          tma_load_3d(sa + Cf::kOpBytes, dmap, &c.full()[st], s2 * BK, 0, k * nbb + cb);
+        }
+        pit += BS / BK;
+      } else if (type == J_TRSM) {
+        // row slab (i, k, sl), inverse form; per column block cb: (1) cb*BS/BK stages of
+        // X[sl, :cb] (solved) x L_kk[cb, :cb] -- the chunks of blocks solved before cb-1 are
+        // final already and stream while the compute warps still work on block cb-1, the
+        // last BS/BK wait for its write-back (tstep, from the storer); (2) X[sl, cb] into
+        // lbuf once the previous staged block has been read (sfree; lfree of the previous
+        // job for cb = 0); (3) BS/BK B-only stages of Dinv_{k,cb} (the A operand, Y, is
+        // staged in lbuf).  The C prefetch precedes (3): the compute warps need it to form Y
+        // before they can free the ring slots (3) waits for.
+        const int nbb = c.nb / BS, k = d1.x;
+        const int64_t ta = c.slot(d0.z, k), tb = c.slot(k, k);
+        const int ra = d1.y * BS;
+        for (int cb = 0; cb < nbb; ++cb) {
+          if (cb > 0) {
+            const int nst = cb * BS / BK, nold = (cb - 1) * BS / BK;
+            produce_range(c, pit, nst, ta, ra, tb, cb * BS, 0, 0, nold);
+            mbar_wait(c.tstep(), tcount & 1);
+            ++tcount;
+            fence_proxy_async();
+            produce_range(c, pit, nst, ta, ra, tb, cb * BS, 0, nold, nst);
+            pit += nst;
+            mbar_wait(c.sfree(), scount & 1);
+            ++scount;
+          } else if (q > 0) {
+            mbar_wait(c.lfree(), (q - 1) & 1);
+          }
+          prefetch_c_issue(c, ta, ra, cb * BS);
+          for (int s2 = 0; s2 < BS / BK; ++s2) issue_stage_b(c, pit + s2, dmap, k * nbb + cb, s2 * BK);
+          pit += BS / BK;
         }
       }
     }
@@ -327,7 +366,7 @@ __device__ void producer_loop(Ctx<BS>& c) {
     // jobs without TMA stages (in-register solves, POTRF diagonal blocks, RECV copies)
     // never mark themselves issued: their worker claims its next job only when they end,
     // so a critical job is not captured by a worker busy for another 10-20 us
-    if (!skip && (type == J_UPD || type == J_PUPD || type == J_TU || type == J_TRSM)) *issued = (int)q;
+    if (!skip && (type == J_UPD || type == J_PUPD || type == J_TU || type == J_TRSM || type == J_TS)) *issued = (int)q;
   }
 }
 
@@ -363,6 +402,26 @@ __device__ void storer_loop(Ctx<BS>& c) {
       bulk_wait_all();
       fence_proxy_async();  // the async-proxy global writes before the generic release below
       __threadfence();
+    } else if (!skip && type == J_TRSM) {
+      // every solved column block Z_cb of the row slab: written back in place, then the
+      // producer may stream it (tstep) as the last K chunk of block cb+1
+      const int nbb = c.nb / BS;
+      const int64_t t = c.slot(d0.z, d1.x);
+      const int r0 = d1.y * BS;
+      const char* src = reinterpret_cast<const char*>(c.lbuf());
+      for (int cb = 0; cb < nbb; ++cb) {
+        mbar_wait(c.cready(), ns & 1);
+        ++ns;
+#pragma unroll 1
+        for (int b = 0; b < BS / 16; ++b) tma_store_3d(c.map, src + b * BS * 128, cb * BS + 16 * b, r0, (int)t);
+        bulk_commit();
+        bulk_wait_read_all();
+        mbar_arrive(cb + 1 < nbb ? c.sfree() : c.lfree());
+        bulk_wait_all();
+        fence_proxy_async();
+        __threadfence();
+        if (cb + 1 < nbb) mbar_arrive(c.tstep());
+      }
     } else {
       mbar_arrive(c.lfree());
     }
@@ -502,31 +561,35 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     gemm_consume(c, BS / BK, acc);
     epi_sub_stage(c, acc, r == q);
   } else if (type == J_TRSM) {
-    Acc<BS> acc;
+    // row slab X = A_ik[sl, :] <- X L_kk^{-T} (L200-202), left-looking over the BS-column
+    // blocks, inverse form (reading R19): Y = X[:, cb] - X[:, :cb] L_kk[cb, :cb]^T, then
+    // X[:, cb] = Y Dinv_cb^T -- two DMMA products per block, no in-block substitution
     const int i = d0.z, k = d1.x, slab = d1.y, nbb = c.nb / BS;
-    double* X = c.tile(i, k) + (int64_t)slab * BS * c.nb;
-    const double* L = c.tile(k, k);
-    prefetch_l2_rows<BS>(X, c.nb, BS, c.nb);
+    prefetch_l2_rows<BS>(c.tile(i, k) + (int64_t)slab * BS * c.nb, c.nb, BS, c.nb);
     for (int cb = 0; cb < nbb; ++cb) {
-      if (cb > 0) gemm_consume(c, cb * BS / BK, acc);
-      if (cb > 0) acc_sub_global(c, acc, X + cb * BS, c.nb);
-      solve_block_job<BS>(X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
-      if (cb + 1 < nbb) {
-        // X[:, cb] is read by the producer's TMA for the next column block
-        __threadfence();
-        fence_proxy_async();
-        __syncwarp();
-        if (c.lane == 0) mbar_arrive(c.tstep());
+      {
+        Acc<BS> acc;
+        gemm_consume(c, cb * BS / BK, acc);  // zero for cb = 0
+        trsm_stage_y(c, acc);
       }
+      Acc<BS> z;
+      gemm_consume<BS, true>(c, BS / BK, z);
+      trsm_stage_z(c, z);
+      __syncwarp();
+      if (c.lane == 0) mbar_arrive(c.cready());  // the storer writes Z_cb back
     }
+  } else if (type == J_INV) {
+    const int k = d1.x, b = d1.y, nbb = c.nb / BS;
+    inv_block_job<BS>(c.tile(k, k) + (int64_t)b * BS * c.nb + b * BS, c.nb,
+                      d.dinv + ((int64_t)k * nbb + b) * BS * BS);
   } else if (type == J_TU) {
     Acc<BS> acc;
     gemm_consume(c, BS / BK, acc);
     epi_sub_stage(c, acc, false);
-  } else if (type == J_TS) {
-    const int i = d0.z, k = d1.x, cb = d1.y, sl = d1.z;
-    solve_block_job<BS>(c.tile(i, k) + (int64_t)sl * BS * c.nb + cb * BS, c.nb,
-                        c.tile(k, k) + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
+  } else if (type == J_TS) {  // X[sl, cb] <- X[sl, cb] Dinv_{k,cb}^T (inverse form, reading R19)
+    Acc<BS> z;
+    gemm_consume(c, BS / BK, z);
+    trsm_stage_z(c, z);  // the storer writes it back
   } else if (type == J_RECV) {  // copy BS rows of a remote panel tile into the local cache
     const int i = d0.z, j = d0.w, sl = d1.y, owner = d1.z;
     (void)owner;
@@ -572,7 +635,7 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
     const int type = d0.y & 0xff, skip = d0.y >> 8;
     // jobs that use lbuf directly (in-block solves, potf2, the fused update's C block is
     // prefetched behind lfree anyway) wait until the previous job's TMA store has read it
-    if (!skip && q > 0 && (type == J_TRSM || type == J_TS || type == J_PANEL || type == J_DIAG))
+    if (!skip && q > 0 && (type == J_INV || type == J_TS || type == J_PANEL || type == J_DIAG))
       mbar_wait(c.lfree(), (q - 1) & 1);
     if (!skip) compute_job(c, d, type, d0, d1, info);
     if (!skip && tma_store_job(type)) {
@@ -686,14 +749,15 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
 }
 
 template <int BS>
-__global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__ CUtensorMap map, StepParams sp,
+__global__ void __launch_bounds__(kWsThreads, 1) k_sched(const __grid_constant__ CUtensorMap map,
+                                                         const __grid_constant__ CUtensorMap dmap, StepParams sp,
                                                          DevSched d) {
   auto c = make_ctx<BS>(&map, sp.tiles, sp.nb, sp.N, d.slot_map);
   const bool latency_worker = d.policy == 2 && (int)blockIdx.x < d.latency_workers;
   if (c.warp >= kComputeWarps) {
     asm volatile("setmaxnreg.dec.sync.aligned.u32 %0;\n" ::"n"(kRegsControl));
     if (c.warp == kProdWarp) {
-      if (c.lane == 0) producer_loop(c);
+      if (c.lane == 0) producer_loop(c, &dmap);
     } else if (c.warp == kSchedWarp) {
       scheduler_loop(c, d, sp, latency_worker);
     } else if (c.warp == kSchedWarp + 1 && blockIdx.x == 0 && d.nwatch > 0) {
@@ -731,6 +795,7 @@ struct SchedState {
   int nrecv_jobs = 0;
   uint64_t* job_trace = nullptr;           // device, 4 per job (trace == 2)
   int* d_abort = nullptr;                  // device abort flag (d.abort_flag), written by sched_abort
+  CUtensorMap dmap{};                      // Dinv workspace map (sched_set_dinv)
   std::vector<int16_t> h_job_type;         // host copies for chol_job_trace
   std::vector<int> h_job_paper;
 };
@@ -770,12 +835,14 @@ struct Builder {
 }  // namespace
 
 // POTRF_k as per-step nodes: DIAG b -> PANEL b (nbb-1-b jobs) -> UPDATE b (K = BS) -> DIAG b+1
-static void build_potrf_steps(Builder& B, int k, int pid, int* first, int* last) {
+static void build_potrf_steps(Builder& B, int k, int pid, int* first, int* last, std::vector<int>* dnodes = nullptr) {
   const int nbb = B.nbb;
   int prev = -1;
+  if (dnodes) dnodes->assign(nbb, -1);
   for (int b = 0; b < nbb; ++b) {
     const int dn = B.add_node(pid, T_POTRF, k, k);
     B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+    if (dnodes) (*dnodes)[b] = dn;
     if (prev >= 0) B.edge(prev, dn);
     if (b == 0) *first = dn;
     prev = dn;
@@ -805,13 +872,15 @@ static void build_potrf_steps(Builder& B, int k, int pid, int* first, int* last)
 // per inner step, the same bits.  blk (hybrid tail): record per block the entry node and
 // the node that leaves it final (tentry / tfin, nbb x nbb).
 static void build_potrf_blockdag(Builder& B, int k, int pid, bool fuse, bool blk, std::vector<int>* tentry,
-                                 std::vector<int>* tfin, int* first, int* last) {
+                                 std::vector<int>* tfin, int* first, int* last, std::vector<int>* dnodes = nullptr) {
   const int nbb = B.nbb;
   std::vector<int> lastU((size_t)nbb * nbb, -1), pan(nbb, -1), fusedP(nbb, -1);
   if (blk) tentry->assign((size_t)nbb * nbb, -1), tfin->assign((size_t)nbb * nbb, -1);
+  if (dnodes) dnodes->assign(nbb, -1);
   for (int b = 0; b < nbb; ++b) {
     const int dn = B.add_node(pid, T_POTRF, k, k);
     B.add_job(dn, Job{J_DIAG, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, (int16_t)(fusedP[b] >= 0), 0, 0});
+    if (dnodes) (*dnodes)[b] = dn;
     if (lastU[b * nbb + b] >= 0) B.edge(lastU[b * nbb + b], dn);
     if (fusedP[b] >= 0) B.edge(fusedP[b], dn);
     if (blk && b == 1 && fusedP[b] >= 0) (*tentry)[b * nbb + b] = dn;  // first touch of block (1,1)
@@ -849,14 +918,42 @@ static void build_potrf_blockdag(Builder& B, int k, int pid, bool fuse, bool blk
   }
 }
 
+// The inverses of the diagonal blocks of L_kk that the inverse-form TRSM row slabs of step k
+// apply (J_TRSM): INV(k, b) after the node that makes block (b, b) of L_kk final (pred[b],
+// or pred[0] alone for a received tile), a job-less join INVJ(k), and INVJ(k) -> every row
+// slab node of step k.  Untraced (paper id -1, highest priority bucket: it gates TRSM work).
+// The right-looking TS(cb, .) nodes (TRSM column-step solves, also inverse form) wait for
+// INV(k, cb) alone: ts[cb] lists them.
+static void build_inverses(Builder& B, int k, const std::vector<int>& pred, const std::vector<int>& slabs,
+                           const std::vector<std::vector<int>>& ts = {}) {
+  bool any_ts = false;
+  for (const auto& v : ts) any_ts |= !v.empty();
+  if (slabs.empty() && !any_ts) return;
+  const int nbb = B.nbb;
+  const int join = slabs.empty() ? -1 : B.add_node(-1, T_POTRF, k, k);
+  for (int b = 0; b < nbb; ++b) {
+    const int v = B.add_node(-1, T_POTRF, k, k);
+    B.add_job(v, Job{J_INV, (int16_t)k, (int16_t)k, (int16_t)k, (int16_t)b, 0, 0, 0});
+    const int p = pred.size() == (size_t)nbb ? pred[b] : (pred.empty() ? -1 : pred[0]);
+    if (p >= 0) B.edge(p, v);
+    if (join >= 0) B.edge(v, join);
+    if (b < (int)ts.size())
+      for (int t : ts[b]) B.edge(v, t);
+  }
+  for (int sn : slabs) B.edge(join, sn);
+}
+
 // TRSM_i_k right-looking over the BS-column blocks c of A_ik, one node per column step:
 //   TS(c): A_ik[:, c] <- A_ik[:, c] L_kk[c,c]^{-T}  (nbb row-block jobs)
 //   TU(c): A_ik[:, c'] -= A_ik[:, c] L_kk[c',c]^T, c' > c  (K = BS)
-static void build_trsm_steps(Builder& B, int i, int k, int tid, int* first, int* last) {
+static void build_trsm_steps(Builder& B, int i, int k, int tid, int* first, int* last,
+                             std::vector<std::vector<int>>* ts_nodes = nullptr) {
   const int nbb = B.nbb;
   int prev_t = -1;
+  if (ts_nodes && ts_nodes->empty()) ts_nodes->resize(nbb);
   for (int cb = 0; cb < nbb; ++cb) {
     const int ts = B.add_node(tid, T_TRSM, i, k);
+    if (ts_nodes) (*ts_nodes)[cb].push_back(ts);
     for (int sl = 0; sl < nbb; ++sl)
       B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
     if (prev_t >= 0) B.edge(prev_t, ts);
@@ -895,6 +992,10 @@ static int sched_upload(SchedState** out, SchedState* st, Builder& B, const std:
                         const std::vector<int>& publish, const std::vector<int4>& watch, const chol_opts_t* opts,
                         int64_t nb, int bs, int sms) {
   const int nnodes = (int)B.deps.size();
+  if (!publish.empty() && publish.size() != (size_t)nnodes) {  // one entry per node (or none)
+    sched_destroy(st);
+    return -8;
+  }
   // ---- queue capacities
   std::vector<int> qcap(kQueues, 0), qbase(kQueues, 0);
   for (int v = 0; v < nnodes; ++v) qcap[node_queue[v]] += 1;
@@ -1129,6 +1230,10 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // first touches it (tentry) and the node that leaves it final (tfin); TRSM: the node
   // that finishes each row slab (tslab)
   std::vector<std::vector<int>> tentry(n_tasks(N)), tfin(n_tasks(N)), tslab(n_tasks(N));
+  // inverse-form TRSM row slabs of each step and the D(b) nodes of each local POTRF
+  // (build_inverses, after the task edges)
+  std::vector<std::vector<int>> slab_nodes(N), dnodes(N);
+  std::vector<std::vector<std::vector<int>>> ts_nodes(N, std::vector<std::vector<int>>(nbb));
   const int nbb2 = nbb * nbb;
   auto gate_of = [&](int tid, int type, int i, int k) {
     // job-less node in front of a blocked task's entry nodes: the target of task-level
@@ -1149,9 +1254,10 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     // shorter block DAG (CHOL_POTRF0_BLOCKDAG=0 turns this off; development switch)
     const bool pblock = potrf_blockdag || (k == 0 && potrf0_blockdag);
     if (mine(k, k) && !pblock && !blk) {  // per-step nodes: DIAG b -> PANEL b -> UPDATE b
-      build_potrf_steps(B, k, pid, &first_node[pid], &last_node[pid]);
+      build_potrf_steps(B, k, pid, &first_node[pid], &last_node[pid], &dnodes[k]);
     } else if (mine(k, k)) {
-      build_potrf_blockdag(B, k, pid, potrf_fuse, blk, &tentry[pid], &tfin[pid], &first_node[pid], &last_node[pid]);
+      build_potrf_blockdag(B, k, pid, potrf_fuse, blk, &tentry[pid], &tfin[pid], &first_node[pid], &last_node[pid],
+                           &dnodes[k]);
       if (blk && k == 0) gate_of(pid, T_POTRF, k, k);
     }
     for (int i = k + 1; i < N && blk; ++i) {
@@ -1168,6 +1274,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
           const int sn = B.add_node(tid, T_TRSM, i, k);
           B.add_job(sn, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
           B.edge(tfin[pid][(nbb - 1) * nbb + nbb - 1], sn);  // D(nbb-1): all of L_kk
+          slab_nodes[k].push_back(sn);
           for (int c = 0; c < nbb; ++c) tentry[tid][sl * nbb + c] = tfin[tid][sl * nbb + c] = sn;
           tslab[tid][sl] = sn;
           B.edge(sn, exit_);
@@ -1177,6 +1284,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         for (int cb = 0; cb < nbb; ++cb) {
           const int ts = B.add_node(tid, T_TRSM, i, k);
           B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+          ts_nodes[k][cb].push_back(ts);
           B.edge(tfin[pid][cb * nbb + cb], ts);
           if (cb > 0) B.edge(lastTU[cb], ts);
           else tentry[tid][sl * nbb] = ts;
@@ -1206,11 +1314,12 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         for (int sl = 0; sl < nbb; ++sl)
           B.add_job(n, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
         first_node[tid] = last_node[tid] = n;
+        slab_nodes[k].push_back(n);
         continue;
       }
       if (!trsm_slabchain) {  // right-looking column steps TS(c) / TU(c)
         const int tid = (int)id_trsm(N, i, k);
-        build_trsm_steps(B, i, k, tid, &first_node[tid], &last_node[tid]);
+        build_trsm_steps(B, i, k, tid, &first_node[tid], &last_node[tid], &ts_nodes[k]);
         continue;
       }
       // Alternative (CHOL_TRSM_SLABCHAIN=1): rows are independent (X L^{-T}), so each
@@ -1229,6 +1338,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         for (int cb = 0; cb < nbb; ++cb) {
           const int ts = B.add_node(tid, T_TRSM, i, k);
           B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
+          ts_nodes[k][cb].push_back(ts);
           B.edge(cb == 0 ? entry : lastTU[cb], ts);
           if (cb + 1 == nbb) B.edge(ts, exit_);
           for (int c2 = cb + 1; c2 < nbb; ++c2) {
@@ -1291,6 +1401,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // ---- task edges: direct data dependencies of Algorithm 1 (dag.cpp, L213-220),
   // mapped onto the nodes (POTRF_k enters at its first inner node, leaves at its last).
   std::vector<int4> watch;  // multi-GPU: {RECV node, owner, tile, step}
+  std::vector<int> recv_node((size_t)(N * (N + 1) / 2), -1);  // multi-GPU: RECV node of a remote tile
   if (!dist) {
     std::vector<std::pair<int64_t, int64_t>> E;
     std::vector<int> type_of;
@@ -1373,7 +1484,6 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     // reached through this rank's RECV node for it, fired by the watcher when the owner
     // publishes the tile.
     std::vector<int64_t> last_writer((size_t)(N * (N + 1) / 2), -1);
-    std::vector<int> recv_node((size_t)(N * (N + 1) / 2), -1);
     std::vector<int> preds;
     auto visit = [&](int64_t task, std::initializer_list<std::pair<int64_t, int64_t>> touched, int64_t wi,
                      int64_t wj) {
@@ -1420,6 +1530,15 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         if (mine(i, k)) publish[last_node[id_trsm(N, i, k)]] = (int)tile_index(i, k);
     }
   }
+
+  // ---- inverses of the diagonal blocks of L_kk for the inverse-form TRSM row slabs: after
+  // the local D(b) nodes, or after the RECV of a remote L_kk
+  for (int k = 0; k < N; ++k) {
+    std::vector<int> pred = dnodes[k];
+    if (pred.empty() && recv_node[tile_index(k, k)] >= 0) pred.assign(1, recv_node[tile_index(k, k)]);
+    build_inverses(B, k, pred, slab_nodes[k], ts_nodes[k]);
+  }
+  if (!publish.empty()) publish.resize(B.deps.size(), -1);  // the inverse nodes publish nothing
 
   // ---- priorities: bottom-level of each Algorithm 1 task (HEFT / dmdas, L299-301,
   // L655-660; reading R13) with latency-estimate weights, quantised into kBuckets;
@@ -1482,16 +1601,21 @@ int sched_create_batch(SchedState** out, int64_t N, int64_t nb, int bs, int sms,
         build_potrf_steps(B, k, -1, &first, &last);
     }
   } else if (type == T_TRSM) {
+    std::vector<std::vector<int>> slabs(N);
     for (int k = 0; k < N && c < count; ++k)
       for (int i = k + 1; i < N && c < count; ++i, ++c) {
         if (count == 1) {
-          build_trsm_steps(B, i, k, -1, &first, &last);
+          std::vector<std::vector<int>> ts;
+          build_trsm_steps(B, i, k, -1, &first, &last, &ts);
+          build_inverses(B, k, {}, {}, ts);
           continue;
         }
         const int n = B.add_node(-1, T_TRSM, i, k);
         for (int sl = 0; sl < nbb; ++sl)
           B.add_job(n, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
+        slabs[k].push_back(n);
       }
+    for (int k = 0; k < N; ++k) build_inverses(B, k, {}, slabs[k]);  // part of the TRSM cost
   } else if (type == T_SYRK) {
     for (int j = 1; j <= count; ++j) {
       const int n = B.add_node(-1, T_SYRK, j, 0);
@@ -1511,6 +1635,12 @@ int sched_create_batch(SchedState** out, int64_t N, int64_t nb, int bs, int sms,
   std::vector<int> node_queue(B.deps.size(), 0), publish;
   std::vector<int4> watch;
   return sched_upload(out, st, B, node_queue, publish, watch, opts, nb, bs, sms);
+}
+
+int sched_set_dinv(SchedState* st, double* dinv, const CUtensorMap& dmap) {
+  st->d.dinv = dinv;
+  st->dmap = dmap;
+  return 0;
 }
 
 int sched_set_dist(SchedState* st, const int* d_slot_map, const int* d_owner_slot, double* const* d_peer_slots,
@@ -1539,9 +1669,9 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
   k_sched_init<<<std::max(1, std::min(64, (st->nroots + 127) / 128)), 128, 0, s>>>(st->d, st->roots, st->nroots);
   const int smem = smem_bytes(st->bs);
   switch (st->bs) {
-    case 96: k_sched<96><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;
-    case 64: k_sched<64><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;
-    case 32: k_sched<32><<<st->workers, kWsThreads, smem, s>>>(map, base, st->d); break;
+    case 96: k_sched<96><<<st->workers, kWsThreads, smem, s>>>(map, st->dmap, base, st->d); break;
+    case 64: k_sched<64><<<st->workers, kWsThreads, smem, s>>>(map, st->dmap, base, st->d); break;
+    case 32: k_sched<32><<<st->workers, kWsThreads, smem, s>>>(map, st->dmap, base, st->d); break;
   }
   *nlaunch += 2;
   if ((e = cudaGetLastError())) return -100 - (int)e;

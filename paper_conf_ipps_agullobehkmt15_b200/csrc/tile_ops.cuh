@@ -81,7 +81,8 @@ struct Ctx {
   __device__ uint64_t* lfree() const { return jdone() + 2; } // lbuf released (compute -> producer)
   __device__ uint64_t* tstep() const { return lfree() + 1; } // TRSM column block stored (compute -> producer)
   __device__ uint64_t* cready() const { return tstep() + 1; } // C - acc staged in lbuf (compute -> storer)
-  // 2*kStages + 8 = 18 barriers = 144 bytes; then 2 x 3 int4 job descriptors + producer progress word
+  __device__ uint64_t* sfree() const { return cready() + 1; } // staged TRSM block read by the store (storer -> producer)
+  // 2*kStages + 9 = 19 barriers = 152 bytes; then 2 x 3 int4 job descriptors + producer progress word
   __device__ int4* jdesc() const { return reinterpret_cast<int4*>(bars() + 160); }
   uint32_t it;     // stages consumed so far
   uint32_t cphase; // parity of the next cbar completion
@@ -123,8 +124,9 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
       mbar_init(&c.jdone()[e], kComputeWarps + 1);
     }
     mbar_init(c.lfree(), kComputeWarps + 1);
-    mbar_init(c.tstep(), kComputeWarps);
+    mbar_init(c.tstep(), 1);  // the storer: TRSM column block written back (sched.cu)
     mbar_init(c.cready(), kComputeWarps);
+    mbar_init(c.sfree(), 1);
     fence_mbar_init();
   }
   if (c.issuer() && map) tma_prefetch_desc(map);
@@ -172,14 +174,28 @@ __device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, 
   tma_load_3d(sa + C::kOpBytes, c.map, &c.full()[st], kk, rb, (int)tb);
 }
 
-// Consume one TMA stage: wait for it, DMMA it into acc, release it to the producer.
+// B-only stage (the A operand is staged in lbuf): BS rows x BK of block `blk` of map m
+// (the Dinv workspace of the inverse-form TRSM), into the B half of ring slot q % kStages.
 template <int BS>
-__device__ __forceinline__ void consume_stage(Ctx<BS>& c, uint32_t q, Acc<BS>& acc, uint32_t rt_zero) {
+__device__ __forceinline__ void issue_stage_b(Ctx<BS>& c, uint32_t q, const CUtensorMap* m, int blk, int kk) {
+  using C = Cfg<BS>;
+  const uint32_t st = q % kStages, ph = (q / kStages) & 1;
+  mbar_wait(&c.empty()[st], ph ^ 1);
+  mbar_arrive_expect_tx(&c.full()[st], C::kOpBytes);
+  tma_load_3d(c.pipe() + st * 2 * C::kOpBytes + C::kOpBytes, m, &c.full()[st], kk, 0, blk);
+}
+
+// Consume one TMA stage: wait for it, DMMA it into acc, release it to the producer.
+// a_box >= 0: the A operand is box a_box of lbuf instead of the ring stage's A half.
+template <int BS>
+__device__ __forceinline__ void consume_stage(Ctx<BS>& c, uint32_t q, Acc<BS>& acc, uint32_t rt_zero,
+                                              int a_box = -1) {
   using C = Cfg<BS>;
   const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
   const uint32_t st = q % kStages, ph = (q / kStages) & 1;
   mbar_wait(&c.full()[st], ph);
-  const uint32_t As = smem_u32(c.pipe()) + st * 2 * C::kOpBytes + (wm * C::WM + g) * 128;
+  const uint32_t As = (a_box >= 0 ? smem_u32(c.lbuf()) + (uint32_t)a_box * BS * 128
+                                  : smem_u32(c.pipe()) + st * 2 * C::kOpBytes) + (wm * C::WM + g) * 128;
   const uint32_t Bs = smem_u32(c.pipe()) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
   uint32_t dep = 0;
 #pragma unroll
@@ -229,7 +245,10 @@ __device__ __forceinline__ void zero_acc(Acc<BS>& acc) {
 // stage's second half, so the shared-memory latency at a stage boundary hides behind
 // ~36 queued DMMAs per warp instead of stalling the pipe (consume_stage paid it every
 // 16 k).  Same DMMA sequence per accumulator as consume_stage (bitwise-identical).
-template <int BS>
+// A_LBUF: the A operand of stage s is box s of lbuf (a block staged there in the TMA box
+// layout, e.g. the TRSM's Y = X[:, cb] - acc) instead of the ring stage's A half; the ring
+// stages then carry the B operand only.
+template <int BS, bool A_LBUF = false>
 __device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) {
   using C = Cfg<BS>;
   zero_acc<BS>(acc);
@@ -239,23 +258,28 @@ __device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) 
   const uint32_t base = smem_u32(c.pipe());
   const uint32_t aoff = (wm * C::WM + g) * 128, boff = C::kOpBytes + (wn * C::WN + g) * 128;
   const uint32_t ch0 = ((2 * t) ^ g) << 4, ch1 = ((2 * t + 1) ^ g) << 4;  // logical chunks 2t, 2t+1
+  // A operand base of stage s (ring slot st): the ring, or box s of lbuf
+  auto abase = [&](uint32_t st, int s) -> uint32_t {
+    if constexpr (A_LBUF) return smem_u32(c.lbuf()) + (uint32_t)s * BS * 128;
+    else return base + st * 2 * C::kOpBytes;
+  };
   double2 a0[C::MI], b0[C::NI];
   uint32_t q = c.it;
   {
     const uint32_t st = q % kStages;
     mbar_wait(&c.full()[st], (q / kStages) & 1);
-    const uint32_t sa = base + st * 2 * C::kOpBytes;
+    const uint32_t sa = base + st * 2 * C::kOpBytes, sa_a = abase(st, 0);
 #pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(sa + aoff + mi * 8 * 128 + ch0);
+    for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(sa_a + aoff + mi * 8 * 128 + ch0);
 #pragma unroll
     for (int ni = 0; ni < C::NI; ++ni) b0[ni] = lds128(sa + boff + ni * 8 * 128 + ch0);
   }
   for (int s = 0; s < nst; ++s, ++q) {
     const uint32_t st = q % kStages;
-    const uint32_t sa = base + st * 2 * C::kOpBytes;
+    const uint32_t sa = base + st * 2 * C::kOpBytes, sa_a = abase(st, s);
     double2 a1[C::MI], b1[C::NI];
 #pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) a1[mi] = lds128(sa + aoff + mi * 8 * 128 + ch1);
+    for (int mi = 0; mi < C::MI; ++mi) a1[mi] = lds128(sa_a + aoff + mi * 8 * 128 + ch1);
 #pragma unroll
     for (int ni = 0; ni < C::NI; ++ni) b1[ni] = lds128(sa + boff + ni * 8 * 128 + ch1);
     uint32_t dep = 0;
@@ -277,9 +301,9 @@ __device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) 
     if (s + 1 < nst) {  // next stage, first half, while the second half's DMMAs run
       const uint32_t sn = (q + 1) % kStages;
       mbar_wait(&c.full()[sn], ((q + 1) / kStages) & 1);
-      const uint32_t san = base + sn * 2 * C::kOpBytes;
+      const uint32_t san = base + sn * 2 * C::kOpBytes, san_a = abase(sn, s + 1);
 #pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(san + aoff + mi * 8 * 128 + ch0);
+      for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(san_a + aoff + mi * 8 * 128 + ch0);
 #pragma unroll
       for (int ni = 0; ni < C::NI; ++ni) b0[ni] = lds128(san + boff + ni * 8 * 128 + ch0);
     }
@@ -388,6 +412,58 @@ __device__ __forceinline__ void epi_sub_stage(Ctx<BS>& c, const Acc<BS>& acc, bo
       sts128(cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4), v);
     }
   fence_proxy_async_shared();  // generic smem writes -> the TMA store (async proxy)
+}
+
+// lbuf offset (bytes) of element (r, cc), cc even, of a BS x BS block in the TMA box layout
+// (box cc/16, row r, logical 16-byte chunk (cc%16)/2, 128B swizzle)
+template <int BS>
+__device__ __forceinline__ uint32_t lbuf_off(int r, int cc) {
+  return (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4);
+}
+
+// TRSM row slab, inverse form (sched.cu J_TRSM): Y = C - acc with C = X[:, cb] prefetched
+// into lbuf, written back in place -- the A operand of the Dinv product that follows
+// (gemm_consume<BS, true>); a compute barrier makes every warp's part visible first.
+template <int BS>
+__device__ __forceinline__ void trsm_stage_y(Ctx<BS>& c, const Acc<BS>& acc) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  mbar_wait(c.cbar(), c.cphase);
+  c.cphase ^= 1;
+  const uint32_t cs = smem_u32(c.lbuf());
+  double2 cv[C::MI][C::NI];
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni)
+      cv[mi][ni] = lds128(cs + lbuf_off<BS>(wm * C::WM + mi * 8 + g, wn * C::WN + ni * 8 + 2 * t));
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      double2 v = cv[mi][ni];
+      v.x -= acc[mi][ni][0];
+      v.y -= acc[mi][ni][1];
+      sts128(cs + lbuf_off<BS>(wm * C::WM + mi * 8 + g, wn * C::WN + ni * 8 + 2 * t), v);
+    }
+  bar_sync(kBarCompute, kComputeThreads);
+}
+
+// ... and Z = acc (the solved column block) staged over Y once every warp has read Y,
+// for the storer's TMA store (the caller arrives on cready).
+template <int BS>
+__device__ __forceinline__ void trsm_stage_z(Ctx<BS>& c, const Acc<BS>& acc) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  bar_sync(kBarCompute, kComputeThreads);
+  const uint32_t cs = smem_u32(c.lbuf());
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni)
+      sts128(cs + lbuf_off<BS>(wm * C::WM + mi * 8 + g, wn * C::WN + ni * 8 + 2 * t),
+             make_double2(acc[mi][ni][0], acc[mi][ni][1]));
+  fence_proxy_async_shared();
 }
 
 // dst[r*P + c] = src[r*ld + c] for a BS x BS block: 16-byte chunks, every load of
@@ -602,6 +678,79 @@ __device__ __forceinline__ void solve_block(const Ctx<BS>& c, double* X, int ldx
                make_double2(x.v[mi][cb][0], x.v[mi][cb][1]));
   }
   bar_sync(kBarCompute, kComputeThreads);  // lbuf free for the next user; X stores issued
+}
+
+// Dinv = L^{-1} for the lower triangular BS x BS block Ld (ld ldl), row-major into Dinv
+// (ld BS): the substitution of solve_block applied to the identity, Z L^T = I, so Z =
+// L^{-T} and Dinv = Z^T (stored transposed; zeros above the diagonal).  One job per
+// diagonal block of L_kk (sched.cu J_INV), off the POTRF chain; the TRSM row slabs then
+// apply each diagonal block as a DMMA product with Dinv (reading R19).
+template <int BS>
+__device__ __forceinline__ void inv_block(const Ctx<BS>& c, const double* Ld, int ldl, double* Dinv) {
+  using C = Cfg<BS>;
+  constexpr int P = C::kPitch, NB = BS / 8;
+  const int tid = threadIdx.x, g = c.lane >> 2, t = c.lane & 3;
+  double* lb = c.lbuf();
+  bar_sync(kBarCompute, kComputeThreads);
+  load_block<BS>(lb, Ld, ldl);
+  if (tid < BS) lb[tid * P + BS] = 1.0 / __ldcg(Ld + (int64_t)tid * ldl + tid);
+  bar_sync(kBarCompute, kComputeThreads);
+  if (c.warp < BS / 16) {
+    RowX<BS> x;
+    const int r0 = 16 * c.warp;
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb) {
+        const int r = r0 + 8 * mi + g, cc = 8 * cb + 2 * t;
+        x.v[mi][cb][0] = r == cc ? 1.0 : 0.0;
+        x.v[mi][cb][1] = r == cc + 1 ? 1.0 : 0.0;
+      }
+    const int qbase = c.lane & ~3;
+#pragma unroll
+    for (int p = 0; p < NB; ++p) {
+      const int c0 = 8 * p;
+#pragma unroll
+      for (int j = 0; j < 8; ++j) {
+        const double rd = lb[(c0 + j) * P + BS];
+        const double l0 = lb[(c0 + 2 * t) * P + c0 + j], l1 = lb[(c0 + 2 * t + 1) * P + c0 + j];
+#pragma unroll
+        for (int mi = 0; mi < 2; ++mi) {
+          const double xj = __shfl_sync(0xffffffffu, x.v[mi][p][j & 1], qbase | (j >> 1)) * rd;
+          if (t == (j >> 1)) x.v[mi][p][j & 1] = xj;
+          if (2 * t > j) x.v[mi][p][0] = fma(-xj, l0, x.v[mi][p][0]);
+          if (2 * t + 1 > j) x.v[mi][p][1] = fma(-xj, l1, x.v[mi][p][1]);
+        }
+      }
+#pragma unroll
+      for (int cb = 1; cb < NB; ++cb) {
+        if (cb <= p) continue;
+        const double2 bv = *reinterpret_cast<const double2*>(lb + (8 * cb + g) * P + c0 + 2 * t);
+#pragma unroll
+        for (int mi = 0; mi < 2; ++mi) {
+          dmma884(x.v[mi][cb][0], x.v[mi][cb][1], -x.v[mi][p][0], bv.x);
+          dmma884(x.v[mi][cb][0], x.v[mi][cb][1], -x.v[mi][p][1], bv.y);
+        }
+      }
+    }
+    // Z[r][c] -> Dinv[c][r]
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi)
+#pragma unroll
+      for (int cb = 0; cb < NB; ++cb) {
+        const int r = r0 + 8 * mi + g, cc = 8 * cb + 2 * t;
+        __stcg(Dinv + (int64_t)cc * BS + r, x.v[mi][cb][0]);
+        __stcg(Dinv + (int64_t)(cc + 1) * BS + r, x.v[mi][cb][1]);
+      }
+  }
+  bar_sync(kBarCompute, kComputeThreads);
+}
+template <int BS>
+__device__ __noinline__ void inv_block_job(const double* Ld, int ldl, double* Dinv) {
+  Ctx<BS> c{};
+  c.warp = threadIdx.x >> 5;
+  c.lane = threadIdx.x & 31;
+  inv_block(c, Ld, ldl, Dinv);
 }
 
 // One thread factors the 8x8 lower block dd (pitch 8) in registers, column by column
@@ -861,6 +1010,54 @@ __device__ __forceinline__ void sub_trsm(Ctx<BS>& c, int i, int k, int slab) {
     solve_block(c, X + cb * BS, c.nb, L + (int64_t)cb * BS * c.nb + cb * BS, c.nb);
     // X[:, cb] (generic stores) is read by TMA in the next block: complete the stores
     // at L2 (gpu-scope fence), then order them before async-proxy accesses.
+    __threadfence();
+    fence_proxy_async();
+    bar_sync(kBarAll, kThreads);
+  }
+}
+
+// The same row slab in the inverse form of the persistent scheduler's J_TRSM (reading R19):
+// per column block cb, Y = X[:, cb] - X[:, :cb] L[cb, :cb]^T staged in lbuf, then
+// X[:, cb] = Y Dinv_cb^T with Dinv_cb = inv(L[cb, cb]) (inv_block, computed by k_inv before
+// the TRSM batch).  Same DMMA order per accumulator as the scheduler's path, so the factor
+// is bitwise identical across executors (R15); here Z is written back with global stores.
+template <int BS>
+__device__ __forceinline__ void sub_trsm_inv(Ctx<BS>& c, const CUtensorMap* dmap, int i, int k, int slab) {
+  using C = Cfg<BS>;
+  const int nbb = c.nb / BS;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  double* X = c.tile(i, k) + (int64_t)slab * BS * c.nb;
+  prefetch_l2_rows<BS>(X, c.nb, BS, c.nb);
+  const uint32_t rt_zero = threadIdx.y;
+  for (int cb = 0; cb < nbb; ++cb) {
+    {
+      Acc<BS> acc;
+      if (cb > 0)
+        gemm_mainloop(c, c.slot(i, k), slab * BS, c.slot(k, k), cb * BS, 0, cb * BS, acc);
+      else
+        zero_acc<BS>(acc);
+      prefetch_c(c, c.slot(i, k), slab * BS, cb * BS);  // lbuf is free: barrier ending block cb-1
+      trsm_stage_y(c, acc);
+    }
+    Acc<BS> z;
+    constexpr int nst = BS / BK;
+    if (c.issuer())
+      for (int s = 0; s < kStages - 1 && s < nst; ++s) issue_stage_b(c, c.it + s, dmap, k * nbb + cb, s * BK);
+    zero_acc<BS>(z);
+    for (int s = 0; s < nst; ++s) {
+      if (c.issuer() && s + kStages - 1 < nst)
+        issue_stage_b(c, c.it + s + kStages - 1, dmap, k * nbb + cb, (s + kStages - 1) * BK);
+      consume_stage(c, c.it + s, z, rt_zero, s);
+    }
+    c.it += nst;
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni)
+        __stcg(reinterpret_cast<double2*>(X + (int64_t)(wm * C::WM + mi * 8 + g) * c.nb + cb * BS + wn * C::WN +
+                                          ni * 8 + 2 * t),
+               make_double2(z[mi][ni][0], z[mi][ni][1]));
+    // X[:, cb] is read by TMA in the next block's GEMM; every warp is done with lbuf
     __threadfence();
     fence_proxy_async();
     bar_sync(kBarAll, kThreads);

@@ -1,0 +1,5 @@
+set -x
+timeout 1500 python -m pytest tests -m gpu -q 2>&1 | tail -25
+python tools/env_time.py 3840,9600,19200,46080 ""
+python tools/job_trace.py 19200 0 2>&1 | tail -2
+python tools/job_trace.py 3840 0 2>&1 | tail -2

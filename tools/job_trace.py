@@ -7,7 +7,7 @@ import paper_conf_ipps_agullobehkmt15_b200 as c
 n = int(sys.argv[1]) if len(sys.argv) > 1 else 19200
 pol = int(sys.argv[2]) if len(sys.argv) > 2 else 0  # 0 = CP_PRIORITY
 nb = 960
-JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU"]
+JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU", "RECV", "INV"]
 with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=pol, trace=2) as p:
     for rep in range(2):
         c.chol_generate(p.h, 0, 0)
@@ -22,7 +22,7 @@ span = t1.max() - t0.min()
 busy = (t1 - t0).sum()
 out = {"n": n, "policy": pol, "factor_ms": t_f * 1e3, "span_ms": span / 1e6, "jobs": len(jt), "workers": int(W),
        "utilisation": busy / (W * span)}
-for k in range(7):
+for k in range(len(JT)):
     m = typ == k
     if m.any():
         d = (t1[m] - t0[m]) / 1e3
@@ -49,7 +49,7 @@ for i in range(20):
 out["util_timeline"] = util
 tq = jt[:, 4].astype(np.int64)
 wait = (t0 - tq) / 1e3
-for k in range(7):
+for k in range(len(JT)):
     m = typ == k
     if m.any():
         out[JT[k]]["wait_p50_us"] = round(float(np.median(wait[m])), 1)
