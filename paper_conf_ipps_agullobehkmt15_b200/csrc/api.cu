@@ -671,11 +671,20 @@ static int gather_impl(chol_plan_s* p, double* L, int64_t ldl) {
 extern "C" int chol_scatter(chol_plan_t p, const double* A, int64_t lda) {
   if (!p || !A || (reinterpret_cast<uintptr_t>(A) & 7)) return -4;
   if (lda < p->n) return -5;
-  if (is_multi(p)) {
-    for (chol_plan_s* sp : p->subs)
-      if (const int st = chol_scatter(sp, A, lda)) return st;
+  if (is_multi(p)) {  // every rank copies its own tiles at once (one stream per device), then wait
+    invalidate_factor(p);
+    int st = 0;
+    for (chol_plan_s* sp : p->subs) {
+      cudaSetDevice(sp->device);
+      if (!st) st = scatter_impl(sp, A, lda);
+    }
+    for (chol_plan_s* sp : p->subs) {
+      cudaSetDevice(sp->device);
+      const cudaError_t e = cudaStreamSynchronize(sp->stream);
+      if (e && !st) st = -100 - (int)e;
+    }
     cudaSetDevice(p->device);
-    return 0;
+    return st;
   }
   cudaSetDevice(p->device);
   invalidate_factor(p);
@@ -688,11 +697,19 @@ extern "C" int chol_scatter(chol_plan_t p, const double* A, int64_t lda) {
 extern "C" int chol_gather(chol_plan_t p, double* L, int64_t ldl) {
   if (!p || !L || (reinterpret_cast<uintptr_t>(L) & 7)) return -4;
   if (ldl < p->n) return -5;
-  if (is_multi(p)) {
-    for (chol_plan_s* sp : p->subs)
-      if (const int st = chol_gather(sp, L, ldl)) return st;
+  if (is_multi(p)) {  // all ranks at once (one stream per device), then wait
+    int st = 0;
+    for (chol_plan_s* sp : p->subs) {
+      cudaSetDevice(sp->device);
+      if (!st) st = gather_impl(sp, L, ldl);
+    }
+    for (chol_plan_s* sp : p->subs) {
+      cudaSetDevice(sp->device);
+      const cudaError_t e = cudaStreamSynchronize(sp->stream);
+      if (e && !st) st = -100 - (int)e;
+    }
     cudaSetDevice(p->device);
-    return 0;
+    return st;
   }
   cudaSetDevice(p->device);
   int st = gather_impl(p, L, ldl);
@@ -726,11 +743,22 @@ extern "C" int chol_generate(chol_plan_t p, uint64_t seed, int family) {
   if (!p) return -4;
   if (family < 0 || family > 1) return -6;
   invalidate_factor(p);
-  if (is_multi(p)) {
-    for (chol_plan_s* sp : p->subs)
-      if (const int st = chol_generate(sp, seed, family)) return st;
+  if (is_multi(p)) {  // every rank generates its owned tiles at once, then wait
+    int st = 0;
+    for (chol_plan_s* sp : p->subs) {
+      cudaSetDevice(sp->device);
+      if (st) break;
+      const cudaError_t e = launch_generate(sp->tiles, sp->n, (int)sp->nb, (int)sp->N, seed, family, sp->stream,
+                                            sp->d_owned_tile, sp->nowned);
+      if (e) st = -100 - (int)e;
+    }
+    for (chol_plan_s* sp : p->subs) {
+      cudaSetDevice(sp->device);
+      const cudaError_t e = cudaStreamSynchronize(sp->stream);
+      if (e && !st) st = -100 - (int)e;
+    }
     cudaSetDevice(p->device);
-    return 0;
+    return st;
   }
   cudaSetDevice(p->device);
   CUDA_TRY(launch_generate(p->tiles, p->n, (int)p->nb, (int)p->N, seed, family, p->stream,

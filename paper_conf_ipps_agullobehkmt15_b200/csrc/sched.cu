@@ -430,28 +430,51 @@ __device__ void storer_loop(Ctx<BS>& c) {
   }
 }
 
-// ---- multi-GPU receive: peer (NVLink) -> local cache, 16-byte loads, 8 in flight per thread
+// ---- multi-GPU receive: row slab sl of remote panel tile (i, j) (BS rows x nb, contiguous:
+// 737 KB at nb = 960), peer memory (NVLink) -> this rank's cache slot, by the TMA engine:
+// thread 0 streams it through the two halves of lbuf with 1-D bulk copies -- peer -> shared
+// (completion on rbar[h]), shared -> local global (bulk group) -- the load of chunk c+1
+// overlapping the store of chunk c; the compute warps wait at the end.  The stores are
+// complete and fenced before the job ends (its successors read the cache slot).
 template <int BS>
 __device__ __forceinline__ void recv_slab(Ctx<BS>& c, const DevSched& d, int i, int j, int sl, int owner) {
-  const int64_t t = tile_index(i, j);
-  const int64_t tile_elems = (int64_t)c.nb * c.nb, off = (int64_t)sl * BS * c.nb;
-  const double2* src = reinterpret_cast<const double2*>(d.peer_slots[owner] + (int64_t)d.owner_slot[t] * tile_elems + off);
-  double2* dst = reinterpret_cast<double2*>(c.tiles + c.slot(i, j) * tile_elems + off);
-  const int n2 = BS * c.nb / 2;
-  constexpr int U = 8;
-  for (int base = threadIdx.x; base < n2; base += U * kComputeThreads) {
-    double2 v[U];
-#pragma unroll
-    for (int u = 0; u < U; ++u) {
-      const int idx = base + u * kComputeThreads;
-      if (idx < n2) v[u] = __ldcg(src + idx);
+  if (threadIdx.x == 0) {
+    const int64_t t = tile_index(i, j);
+    const int64_t tile_elems = (int64_t)c.nb * c.nb, off = (int64_t)sl * BS * c.nb;
+    const char* src = reinterpret_cast<const char*>(d.peer_slots[owner] + (int64_t)d.owner_slot[t] * tile_elems + off);
+    char* dst = reinterpret_cast<char*>(c.tiles + c.slot(i, j) * tile_elems + off);
+    char* buf = reinterpret_cast<char*>(c.lbuf());
+    constexpr uint32_t kHalf = (Cfg<BS>::kBufBytes / 2) & ~1023u;  // bytes per chunk
+    const int64_t total = (int64_t)BS * c.nb * 8;
+    const int nch = (int)((total + kHalf - 1) / kHalf);
+    auto load = [&](int ch) {
+      const int64_t left = total - (int64_t)ch * kHalf;
+      const uint32_t bytes = (uint32_t)(left < kHalf ? left : kHalf);
+      uint64_t* bar = &c.rbar()[ch & 1];
+      mbar_arrive_expect_tx(bar, bytes);
+      bulk_load(buf + (ch & 1) * kHalf, src + (int64_t)ch * kHalf, bytes, bar);
+    };
+    fence_proxy_async();
+    load(0);
+    for (int ch = 0; ch < nch; ++ch) {
+      const int64_t left = total - (int64_t)ch * kHalf;
+      const uint32_t bytes = (uint32_t)(left < kHalf ? left : kHalf);
+      if (ch + 1 < nch) {
+        if (ch >= 1) bulk_wait_read<0>();  // buffer (ch+1)&1 = (ch-1)&1: its store has read it
+        load(ch + 1);
+      }
+      // chunk ch landed (bit h of rcount: parity of the next completion of rbar[h])
+      const int h = ch & 1;
+      mbar_wait(&c.rbar()[h], (c.rcount >> h) & 1u);
+      c.rcount ^= 1u << h;
+      bulk_store(dst + (int64_t)ch * kHalf, buf + (ch & 1) * kHalf, bytes);
+      bulk_commit();
     }
-#pragma unroll
-    for (int u = 0; u < U; ++u) {
-      const int idx = base + u * kComputeThreads;
-      if (idx < n2) __stcg(dst + idx, v[u]);
-    }
+    bulk_wait_all();
+    fence_proxy_async();
+    __threadfence();
   }
+  bar_sync(kBarCompute, kComputeThreads);
 }
 
 // ---- multi-GPU watcher (warp 10 of CTA 0): fires the RECV nodes whose remote tile became
@@ -635,7 +658,7 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
     const int type = d0.y & 0xff, skip = d0.y >> 8;
     // jobs that use lbuf directly (in-block solves, potf2, the fused update's C block is
     // prefetched behind lfree anyway) wait until the previous job's TMA store has read it
-    if (!skip && q > 0 && (type == J_INV || type == J_TS || type == J_PANEL || type == J_DIAG))
+    if (!skip && q > 0 && (type == J_INV || type == J_TS || type == J_PANEL || type == J_DIAG || type == J_RECV))
       mbar_wait(c.lfree(), (q - 1) & 1);
     if (!skip) compute_job(c, d, type, d0, d1, info);
     if (!skip && tma_store_job(type)) {

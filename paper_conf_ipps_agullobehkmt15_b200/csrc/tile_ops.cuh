@@ -39,7 +39,7 @@ struct Cfg {
   static constexpr int kPitch = BS + 2;            // doubles; keeps double2 alignment
   static constexpr int kBufBytes = BS * kPitch * 8;
   static constexpr int kPanBytes = 2 * BS * 10 * 8;  // two BS x 8 panels (pitch 10)
-  static constexpr int kBarBytes = 256;               // mbarriers + job ring descriptors
+  static constexpr int kBarBytes = 320;               // 21 mbarriers (176 B) + job ring descriptors + progress word
   static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kPanBytes + kBarBytes + 1024;
   static_assert(kBufBytes >= BS * BS * 8, "lbuf holds a TMA-prefetched BS x BS C block");
   static constexpr int RW = BS / kComputeWarps;    // rows per warp in the solves
@@ -82,10 +82,12 @@ struct Ctx {
   __device__ uint64_t* tstep() const { return lfree() + 1; } // TRSM column block stored (compute -> producer)
   __device__ uint64_t* cready() const { return tstep() + 1; } // C - acc staged in lbuf (compute -> storer)
   __device__ uint64_t* sfree() const { return cready() + 1; } // staged TRSM block read by the store (storer -> producer)
-  // 2*kStages + 9 = 19 barriers = 152 bytes; then 2 x 3 int4 job descriptors + producer progress word
-  __device__ int4* jdesc() const { return reinterpret_cast<int4*>(bars() + 160); }
+  __device__ uint64_t* rbar() const { return sfree() + 1; }   // [2] RECV bulk-copy buffers (thread 0 only)
+  // 2*kStages + 11 = 21 barriers = 168 bytes; then 2 x 3 int4 job descriptors + producer progress word
+  __device__ int4* jdesc() const { return reinterpret_cast<int4*>(bars() + 176); }
   uint32_t it;     // stages consumed so far
   uint32_t cphase; // parity of the next cbar completion
+  uint32_t rcount; // RECV bulk copies (thread 0): bit h = parity of the next completion of rbar[h]
   int warp, lane;
 
   const int* slot_map;  // multi-GPU: store slot of tile (i,j) (tile_index order); null = identity
@@ -109,6 +111,7 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
   if (threadIdx.x == 0) *reinterpret_cast<int*>(c.jdesc() + 6) = 0;
   c.it = 0;
   c.cphase = 0;
+  c.rcount = 0;
   c.warp = threadIdx.x >> 5;
   c.lane = threadIdx.x & 31;
   if (threadIdx.x == 0) {
@@ -127,6 +130,8 @@ __device__ __forceinline__ Ctx<BS> make_ctx(const CUtensorMap* map, double* tile
     mbar_init(c.tstep(), 1);  // the storer: TRSM column block written back (sched.cu)
     mbar_init(c.cready(), kComputeWarps);
     mbar_init(c.sfree(), 1);
+    mbar_init(&c.rbar()[0], 1);
+    mbar_init(&c.rbar()[1], 1);
     fence_mbar_init();
   }
   if (c.issuer() && map) tma_prefetch_desc(map);
