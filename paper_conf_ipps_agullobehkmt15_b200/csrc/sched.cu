@@ -318,17 +318,10 @@ __device__ void producer_loop(Ctx<BS>& c, const CUtensorMap* dmap) {
       } else if (type == J_TS) {
         // TS(cb, sl), inverse form: A_ik[sl, cb] Dinv_{k,cb}^T, K = BS -- A stages from the
         // tile store, B stages from the Dinv workspace; no C block (the result overwrites)
-        using Cf = Cfg<BS>;
         const int64_t ta = c.slot(d0.z, d1.x);
         const int nbb = c.nb / BS, k = d1.x, cb = d1.y, ra = d1.z * BS;
-        for (int s2 = 0; s2 < BS / BK; ++s2) {
-          const uint32_t qq = pit + s2, st = qq % kStages, ph = (qq / kStages) & 1;
-          mbar_wait(&c.empty()[st], ph ^ 1);
-          mbar_arrive_expect_tx(&c.full()[st], 2 * Cf::kOpBytes);
-          char* sa = c.pipe() + st * 2 * Cf::kOpBytes;
-          tma_load_3d(sa, c.map, &c.full()[st], cb * BS + s2 * BK, ra, (int)ta);
-          tma_load_3d(sa + Cf::kOpBytes, dmap, &c.full()[st], s2 * BK, 0, k * nbb + cb);
-        }
+        for (int s2 = 0; s2 < BS / BK; ++s2)
+          issue_stage_ab(c, pit + s2, c.map, ta, ra, cb * BS + s2 * BK, dmap, k * nbb + cb, 0, s2 * BK);
         pit += BS / BK;
       } else if (type == J_TRSM) {
         // row slab (i, k, sl), inverse form; per column block cb: (1) cb*BS/BK stages of

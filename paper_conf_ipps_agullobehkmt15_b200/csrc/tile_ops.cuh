@@ -23,8 +23,13 @@ namespace chol {
 constexpr int kComputeWarps = 8;
 constexpr int kComputeThreads = kComputeWarps * 32;
 constexpr int kThreads = kComputeThreads;
-constexpr int kStages = 5;
-constexpr int BK = 16;  // doubles per TMA box row (128 bytes)
+// The K loop runs in stages of BK = 32: per operand two TMA boxes of kBox = 16 doubles
+// (128-byte rows, the 128B-swizzle limit) -- half as many stage hand-offs as 16-wide stages
+// (tools/microbench/mainloop_bench: 97.4% -> 98.6% of the DMMA bound per 96x96x960 block),
+// in a 3-deep ring (the same 4.6 us of TMA lead as 5 stages of 16).
+constexpr int kStages = 3;
+constexpr int BK = 32;    // doubles per stage
+constexpr int kBox = 16;  // doubles per TMA box row (128 bytes)
 constexpr int kBarCompute = 1;  // named barrier id: compute warps only
 constexpr int kBarAll = 2;      // named barrier id: all warps
 constexpr int kBarDiag = 3;     // named barrier id: panel owner warp -> diagonal-factor warp (potf2_block)
@@ -34,13 +39,14 @@ template <int BS>
 struct Cfg {
   static constexpr int WM = BS / 2, WN = BS / 4;  // warp tile
   static constexpr int MI = WM / 8, NI = WN / 8;  // m8n8 blocks per warp
-  static constexpr int kOpBytes = BS * BK * 8;    // one operand, one stage
-  static constexpr int kPipeBytes = kStages * 2 * kOpBytes;
+  static constexpr int kOpBytes = BS * kBox * 8;  // one TMA box: BS rows x 128 B
+  static constexpr int kStageBytes = 4 * kOpBytes; // A box 0, A box 1, B box 0, B box 1
+  static constexpr int kPipeBytes = kStages * kStageBytes;
   static constexpr int kPitch = BS + 2;            // doubles; keeps double2 alignment
   static constexpr int kBufBytes = BS * kPitch * 8;
-  static constexpr int kPanBytes = 2 * BS * 10 * 8;  // two BS x 8 panels (pitch 10)
   static constexpr int kBarBytes = 320;               // 21 mbarriers (176 B) + job ring descriptors + progress word
-  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kPanBytes + kBarBytes + 1024;
+  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kBarBytes + 1024;
+  static_assert(2 * BS * 10 + 128 <= BS * kPitch, "potf2 panels fit in lbuf behind dd / rdv");
   static_assert(kBufBytes >= BS * BS * 8, "lbuf holds a TMA-prefetched BS x BS C block");
   static constexpr int RW = BS / kComputeWarps;    // rows per warp in the solves
   static constexpr int CPL = BS / 32;              // columns per lane in the solves
@@ -65,12 +71,12 @@ struct Ctx {
     const uint32_t mis = static_cast<uint32_t>(__cvta_generic_to_shared(smem_raw)) & 1023u;
     return smem_raw + ((1024u - mis) & 1023u);
   }
-  __device__ static char* bars() { return base() + Cfg<BS>::kPipeBytes + Cfg<BS>::kBufBytes + Cfg<BS>::kPanBytes; }
+  __device__ static char* bars() { return base() + Cfg<BS>::kPipeBytes + Cfg<BS>::kBufBytes; }
   __device__ char* pipe() const { return base(); }  // kStages x {A, B} operand buffers
   __device__ double* buf() const { return reinterpret_cast<double*>(base()); }  // solve buffer (aliases pipe)
   __device__ double* lbuf() const { return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes); }  // BS x kPitch
-  __device__ double* pans() const {  // two BS x 8 panels for the in-block solves
-    return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes + Cfg<BS>::kBufBytes);
+  __device__ double* pans() const {  // potf2: two BS x 8 panels, in lbuf behind dd (64) / rdv (8)
+    return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes) + 128;
   }
   __device__ uint64_t* full() const { return reinterpret_cast<uint64_t*>(bars()); }  // kStages
   __device__ uint64_t* empty() const { return full() + kStages; }                     // kStages
@@ -168,46 +174,56 @@ __device__ __forceinline__ void prefetch_c(Ctx<BS>& c, int64_t tile, int r0, int
   if (c.issuer()) prefetch_c_issue(c, tile, r0, c0);
 }
 
+// Stage q (ring slot q % kStages): A = rows [ra, ra+BS) x columns [ka, ka+BK) of plane ta of
+// map ma, B likewise (rb, kb, tb, mb) -- two 16-wide boxes each.  A-less (ma null) stages
+// carry only B (the A operand staged in lbuf).
 template <int BS>
-__device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, int ra, int64_t tb, int rb, int kk) {
+__device__ __forceinline__ void issue_stage_ab(Ctx<BS>& c, uint32_t q, const CUtensorMap* ma, int64_t ta, int ra, int ka,
+                                               const CUtensorMap* mb, int64_t tb, int rb, int kb) {
   using C = Cfg<BS>;
   const uint32_t st = q % kStages, ph = (q / kStages) & 1;
   mbar_wait(&c.empty()[st], ph ^ 1);  // the previous use of this buffer was released by all warps
-  mbar_arrive_expect_tx(&c.full()[st], 2 * C::kOpBytes);
-  char* sa = c.pipe() + st * 2 * C::kOpBytes;
-  tma_load_3d(sa, c.map, &c.full()[st], kk, ra, (int)ta);
-  tma_load_3d(sa + C::kOpBytes, c.map, &c.full()[st], kk, rb, (int)tb);
+  mbar_arrive_expect_tx(&c.full()[st], (ma ? 4 : 2) * C::kOpBytes);
+  char* sa = c.pipe() + st * C::kStageBytes;
+  if (ma) {
+    tma_load_3d(sa, ma, &c.full()[st], ka, ra, (int)ta);
+    tma_load_3d(sa + C::kOpBytes, ma, &c.full()[st], ka + kBox, ra, (int)ta);
+  }
+  tma_load_3d(sa + 2 * C::kOpBytes, mb, &c.full()[st], kb, rb, (int)tb);
+  tma_load_3d(sa + 3 * C::kOpBytes, mb, &c.full()[st], kb + kBox, rb, (int)tb);
 }
-
+template <int BS>
+__device__ __forceinline__ void issue_stage(Ctx<BS>& c, uint32_t q, int64_t ta, int ra, int64_t tb, int rb, int kk) {
+  issue_stage_ab(c, q, c.map, ta, ra, kk, c.map, tb, rb, kk);
+}
 // B-only stage (the A operand is staged in lbuf): BS rows x BK of block `blk` of map m
-// (the Dinv workspace of the inverse-form TRSM), into the B half of ring slot q % kStages.
+// (the Dinv workspace of the inverse-form TRSM).
 template <int BS>
 __device__ __forceinline__ void issue_stage_b(Ctx<BS>& c, uint32_t q, const CUtensorMap* m, int blk, int kk) {
-  using C = Cfg<BS>;
-  const uint32_t st = q % kStages, ph = (q / kStages) & 1;
-  mbar_wait(&c.empty()[st], ph ^ 1);
-  mbar_arrive_expect_tx(&c.full()[st], C::kOpBytes);
-  tma_load_3d(c.pipe() + st * 2 * C::kOpBytes + C::kOpBytes, m, &c.full()[st], kk, 0, blk);
+  issue_stage_ab<BS>(c, q, nullptr, 0, 0, 0, m, blk, 0, kk);
 }
 
 // Consume one TMA stage: wait for it, DMMA it into acc, release it to the producer.
-// a_box >= 0: the A operand is box a_box of lbuf instead of the ring stage's A half.
+// a_stage >= 0: the A operand is lbuf (boxes 2 a_stage, 2 a_stage + 1) instead of the
+// ring stage's A boxes.  Quarter qt of a stage = box qt/2, half qt%2: thread (g, t) reads
+// logical 16-byte chunk 2t + h of its row (k = 4t + 2h, +1 within the box); with the 128B
+// swizzle (chunk ^= row & 7) the two rows g, g+1 of one 8-lane phase land on chunks of
+// opposite parity -> conflict-free LDS.128.
 template <int BS>
 __device__ __forceinline__ void consume_stage(Ctx<BS>& c, uint32_t q, Acc<BS>& acc, uint32_t rt_zero,
-                                              int a_box = -1) {
+                                              int a_stage = -1) {
   using C = Cfg<BS>;
   const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
   const uint32_t st = q % kStages, ph = (q / kStages) & 1;
   mbar_wait(&c.full()[st], ph);
-  const uint32_t As = (a_box >= 0 ? smem_u32(c.lbuf()) + (uint32_t)a_box * BS * 128
-                                  : smem_u32(c.pipe()) + st * 2 * C::kOpBytes) + (wm * C::WM + g) * 128;
-  const uint32_t Bs = smem_u32(c.pipe()) + st * 2 * C::kOpBytes + C::kOpBytes + (wn * C::WN + g) * 128;
+  const uint32_t sbase = smem_u32(c.pipe()) + st * C::kStageBytes;
   uint32_t dep = 0;
 #pragma unroll
-  for (int h = 0; h < 2; ++h) {
-    // Thread (g, t) reads logical 16-byte chunk 2t + h of its row (k = 4t + 2h, +1):
-    // with the 128B swizzle (chunk ^= row & 7) the two rows g, g+1 of one 8-lane
-    // phase land on chunks of opposite parity -> conflict-free LDS.128.
+  for (int qt = 0; qt < 4; ++qt) {
+    const int box = qt >> 1, h = qt & 1;
+    const uint32_t As = (a_stage >= 0 ? smem_u32(c.lbuf()) + (uint32_t)(2 * a_stage + box) * BS * 128
+                                      : sbase + box * C::kOpBytes) + (wm * C::WM + g) * 128;
+    const uint32_t Bs = sbase + (2 + box) * C::kOpBytes + (wn * C::WN + g) * 128;
     const int chunk = ((2 * t + h) ^ g) << 4;
     double2 af[C::MI], bf[C::NI];
 #pragma unroll
@@ -245,14 +261,15 @@ __device__ __forceinline__ void zero_acc(Acc<BS>& acc) {
 }
 
 // Consumer side only (warp-specialised kernel: a separate producer issues the stages).
-// Software-pipelined across stages: the fragments of the next stage's first half
-// (k-slots 4t, 4t+1) are loaded -- after its full barrier -- before the DMMAs of this
-// stage's second half, so the shared-memory latency at a stage boundary hides behind
-// ~36 queued DMMAs per warp instead of stalling the pipe (consume_stage paid it every
-// 16 k).  Same DMMA sequence per accumulator as consume_stage (bitwise-identical).
-// A_LBUF: the A operand of stage s is box s of lbuf (a block staged there in the TMA box
-// layout, e.g. the TRSM's Y = X[:, cb] - acc) instead of the ring stage's A half; the ring
-// stages then carry the B operand only.
+// Software-pipelined by quarter stage (16 k each, two per TMA box): the fragments of the
+// next quarter are loaded before the DMMAs of the current one, across stage boundaries
+// too (the next stage's full barrier is waited for before its first quarter's loads, which
+// run under the last quarter's DMMAs) -- the shared-memory latency hides behind ~36 queued
+// DMMAs per warp.  Same DMMA sequence per accumulator as consume_stage (bitwise identical).
+// The stage is released after its last DMMAs, predicated on every fragment register of the
+// stage (XORed right after the DMMAs that consumed it: no extra stall).
+// A_LBUF: the A operand of stage s is lbuf boxes 2s, 2s+1 (a block staged there in the TMA
+// box layout, e.g. the TRSM's Y = X[:, cb] - acc); the ring stages then carry B only.
 template <int BS, bool A_LBUF = false>
 __device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) {
   using C = Cfg<BS>;
@@ -261,65 +278,59 @@ __device__ __forceinline__ void gemm_consume(Ctx<BS>& c, int nst, Acc<BS>& acc) 
   if (nst <= 0) return;
   const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
   const uint32_t base = smem_u32(c.pipe());
-  const uint32_t aoff = (wm * C::WM + g) * 128, boff = C::kOpBytes + (wn * C::WN + g) * 128;
-  const uint32_t ch0 = ((2 * t) ^ g) << 4, ch1 = ((2 * t + 1) ^ g) << 4;  // logical chunks 2t, 2t+1
-  // A operand base of stage s (ring slot st): the ring, or box s of lbuf
-  auto abase = [&](uint32_t st, int s) -> uint32_t {
-    if constexpr (A_LBUF) return smem_u32(c.lbuf()) + (uint32_t)s * BS * 128;
-    else return base + st * 2 * C::kOpBytes;
+  const uint32_t aoff = (wm * C::WM + g) * 128, boff = 2 * C::kOpBytes + (wn * C::WN + g) * 128;
+  const uint32_t chq0 = ((2 * t) ^ g) << 4, chq1 = ((2 * t + 1) ^ g) << 4;  // logical chunks 2t, 2t+1
+  double2 a[2][C::MI], b[2][C::NI];
+  // fragments of quarter qt of stage s (ring slot st) into register slot r
+  auto load = [&](int r, uint32_t st, int s, int qt) {
+    const uint32_t box = (uint32_t)(qt >> 1), ch = (qt & 1) ? chq1 : chq0;
+    uint32_t abase;
+    if constexpr (A_LBUF) abase = smem_u32(c.lbuf()) + (uint32_t)(2 * s) * BS * 128 + box * BS * 128;
+    else abase = base + st * C::kStageBytes + box * C::kOpBytes;
+    const uint32_t bbase = base + st * C::kStageBytes + box * C::kOpBytes;
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) a[r][mi] = lds128(abase + aoff + mi * 8 * 128 + ch);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) b[r][ni] = lds128(bbase + boff + ni * 8 * 128 + ch);
   };
-  double2 a0[C::MI], b0[C::NI];
+  uint32_t dep = 0;
+  auto mma = [&](int r) {
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a[r][mi].x, b[r][ni].x);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a[r][mi].y, b[r][ni].y);
+#pragma unroll
+    for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(a[r][mi].x);
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(b[r][ni].x);
+  };
   uint32_t q = c.it;
   {
     const uint32_t st = q % kStages;
     mbar_wait(&c.full()[st], (q / kStages) & 1);
-    const uint32_t sa = base + st * 2 * C::kOpBytes, sa_a = abase(st, 0);
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(sa_a + aoff + mi * 8 * 128 + ch0);
-#pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) b0[ni] = lds128(sa + boff + ni * 8 * 128 + ch0);
+    load(0, st, 0, 0);
   }
   for (int s = 0; s < nst; ++s, ++q) {
     const uint32_t st = q % kStages;
-    const uint32_t sa = base + st * 2 * C::kOpBytes, sa_a = abase(st, s);
-    double2 a1[C::MI], b1[C::NI];
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) a1[mi] = lds128(sa_a + aoff + mi * 8 * 128 + ch1);
-#pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) b1[ni] = lds128(sa + boff + ni * 8 * 128 + ch1);
-    uint32_t dep = 0;
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi) dep ^= __double2loint(a0[mi].x) ^ __double2loint(a1[mi].x);
-#pragma unroll
-    for (int ni = 0; ni < C::NI; ++ni) dep ^= __double2loint(b0[ni].x) ^ __double2loint(b1[ni].x);
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a0[mi].x, b0[ni].x);
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a0[mi].y, b0[ni].y);
-    // this stage's loads have all returned (dep): hand the buffer back to the producer
-    __syncwarp();
-    if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty()[st]);
-    if (s + 1 < nst) {  // next stage, first half, while the second half's DMMAs run
+    load(1, st, s, 1);
+    mma(0);
+    load(0, st, s, 2);
+    mma(1);
+    load(1, st, s, 3);
+    mma(0);
+    if (s + 1 < nst) {  // next stage, first quarter, while this stage's last DMMAs run
       const uint32_t sn = (q + 1) % kStages;
       mbar_wait(&c.full()[sn], ((q + 1) / kStages) & 1);
-      const uint32_t san = base + sn * 2 * C::kOpBytes, san_a = abase(sn, s + 1);
-#pragma unroll
-      for (int mi = 0; mi < C::MI; ++mi) a0[mi] = lds128(san_a + aoff + mi * 8 * 128 + ch0);
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) b0[ni] = lds128(san + boff + ni * 8 * 128 + ch0);
+      load(0, sn, s + 1, 0);
     }
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a1[mi].x, b1[ni].x);
-#pragma unroll
-    for (int mi = 0; mi < C::MI; ++mi)
-#pragma unroll
-      for (int ni = 0; ni < C::NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a1[mi].y, b1[ni].y);
+    mma(1);
+    // every fragment of this stage has been loaded (dep): hand the buffer back
+    __syncwarp();
+    if (c.lane == (int)(dep & rt_zero)) mbar_arrive(&c.empty()[st]);
   }
   c.it += nst;
 }
