@@ -87,6 +87,14 @@ __device__ __forceinline__ void bulk_store(void* dst, const void* src, uint32_t 
 // every committed bulk store except the newest n has read its shared-memory source
 template <int n>
 __device__ __forceinline__ void bulk_wait_read() { asm volatile("cp.async.bulk.wait_group.read %0;" ::"n"(n) : "memory"); }
+// 3-D tiled TMA reduce-add shared -> global: dst += box, element-wise in the L2 (FP64
+// supported: c + (-v) bit for bit, tools/microbench/tma_red_f64.cu), bulk-group completion
+__device__ __forceinline__ void tma_reduce_add_3d(const CUtensorMap* map, const void* src, int c0, int c1, int c2) {
+  asm volatile("cp.reduce.async.bulk.tensor.3d.global.shared::cta.add.tile.bulk_group [%0, {%2, %3, %4}], [%1];" ::"l"(
+                   map),
+               "r"(smem_u32(src)), "r"(c0), "r"(c1), "r"(c2)
+               : "memory");
+}
 __device__ __forceinline__ void bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
 // the shared-memory source of every committed bulk store has been read
 __device__ __forceinline__ void bulk_wait_read_all() { asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory"); }

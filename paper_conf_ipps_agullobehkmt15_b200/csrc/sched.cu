@@ -308,11 +308,14 @@ __device__ void producer_loop(Ctx<BS>& c, const CUtensorMap* dmap) {
           ra = d1.z * BS; rb = d1.w * BS; kb = d1.y * BS; nst = BS / BK;
           job_cblock(c, type, d0, d1, &tcb, &cr, &cc);
         }
-        // stages first (they only need ring space), then the C prefetch into lbuf once
-        // the previous job has released lbuf, then the rest
+        // the K-loop jobs add -acc to C with TMA reduce-add stores (no C block read);
+        // the fused D(b) update keeps the C prefetch: stages first (they only need ring
+        // space), then the C prefetch into lbuf once the previous job released it
         produce_range(c, pit, nst, ta, ra, tb, rb, kb, 0, kStages);
-        if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
-        prefetch_c_issue(c, tcb, cr, cc);
+        if (fused_diag) {
+          if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
+          prefetch_c_issue(c, tcb, cr, cc);
+        }
         produce_range(c, pit, nst, ta, ra, tb, rb, kb, kStages, nst);
         pit += nst;
       } else if (type == J_TS) {
@@ -364,7 +367,7 @@ __device__ void producer_loop(Ctx<BS>& c, const CUtensorMap* dmap) {
 }
 
 // ---- storer (warp 11, one lane): the TMA-store epilogue of the K-loop jobs.  The compute
-// warps stage C - acc in lbuf (epi_sub_stage), arrive on cready and go on with their next
+// warps stage -acc in lbuf (epi_stage_neg), arrive on cready and go on with their next
 // job; the storer writes the block back with TMA (the same boxes the producer prefetched),
 // releases lbuf once the store has read it (lfree) and completes the job (jdone) once the
 // store has been performed -- only then does the scheduler warp release the successors.
@@ -387,8 +390,13 @@ __device__ void storer_loop(Ctx<BS>& c) {
       mbar_wait(c.cready(), ns & 1);
       ++ns;
       const char* src = reinterpret_cast<const char*>(c.lbuf());
+      if (type == J_TS) {  // overwrite
 #pragma unroll 1
-      for (int b = 0; b < BS / 16; ++b) tma_store_3d(c.map, src + b * BS * 128, c0 + 16 * b, r0, (int)t);
+        for (int b = 0; b < BS / 16; ++b) tma_store_3d(c.map, src + b * BS * 128, c0 + 16 * b, r0, (int)t);
+      } else {  // C += -acc
+#pragma unroll 1
+        for (int b = 0; b < BS / 16; ++b) tma_reduce_add_3d(c.map, src + b * BS * 128, c0 + 16 * b, r0, (int)t);
+      }
       bulk_commit();
       bulk_wait_read_all();
       mbar_arrive(c.lfree());
@@ -541,7 +549,8 @@ void sched_phase_dump() {
 
 // ---- compute warps: run the job's consumer side
 template <int BS>
-__device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int type, const int4& d0, const int4& d1,
+__device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int type, uint32_t q, const int4& d0,
+                                            const int4& d1,
                                             int* info) {
   // accumulators are declared per branch: one function-wide Acc makes ptxas keep its
   // registers reserved across the register-hungry in-block routines (spills)
@@ -562,7 +571,8 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
       PHASE_ADD(6, phase_clock() - p2);
     }
 #endif
-    epi_sub_stage(c, acc, i == j && bm == bn);
+    if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);  // the previous job's staged block has been read
+    epi_stage_neg(c, acc, i == j && bm == bn);
 #ifdef CHOL_PHASES
     const long long p3 = phase_clock();
     PHASE_ADD(1, p1 - p0);
@@ -573,9 +583,10 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     (void)k;
   } else if (type == J_PUPD) {
     Acc<BS> acc;
-    const int r = d1.z, q = d1.w;
+    const int r = d1.z, qb = d1.w;
     gemm_consume(c, BS / BK, acc);
-    epi_sub_stage(c, acc, r == q);
+    if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
+    epi_stage_neg(c, acc, r == qb);
   } else if (type == J_TRSM) {
     // row slab X = A_ik[sl, :] <- X L_kk^{-T} (L200-202), left-looking over the BS-column
     // blocks, inverse form (reading R19): Y = X[:, cb] - X[:, :cb] L_kk[cb, :cb]^T, then
@@ -601,7 +612,8 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
   } else if (type == J_TU) {
     Acc<BS> acc;
     gemm_consume(c, BS / BK, acc);
-    epi_sub_stage(c, acc, false);
+    if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
+    epi_stage_neg(c, acc, false);
   } else if (type == J_TS) {  // X[sl, cb] <- X[sl, cb] Dinv_{k,cb}^T (inverse form, reading R19)
     Acc<BS> z;
     gemm_consume(c, BS / BK, z);
@@ -653,7 +665,7 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
     // prefetched behind lfree anyway) wait until the previous job's TMA store has read it
     if (!skip && q > 0 && (type == J_INV || type == J_TS || type == J_PANEL || type == J_DIAG || type == J_RECV))
       mbar_wait(c.lfree(), (q - 1) & 1);
-    if (!skip) compute_job(c, d, type, d0, d1, info);
+    if (!skip) compute_job(c, d, type, q, d0, d1, info);
     if (!skip && tma_store_job(type)) {
       __syncwarp();
       if (c.lane == 0) mbar_arrive(c.cready());  // C - acc staged: the storer takes over
@@ -663,6 +675,10 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
 #endif
     __syncwarp();
     if (c.lane == 0) {
+      // lfree has one phase per job (compute warps + the storer): a job that ends quickly
+      // (skipped after a failed pivot, no lbuf use) must not arrive into the previous
+      // job's phase while the storer is still reading that job's staged block
+      if (q > 0) mbar_wait(c.lfree(), (q - 1) & 1);
       mbar_arrive(c.lfree());  // lbuf (C block / L block / rdiag) no longer needed
       if (c.warp == 0) {     // end time of the job as seen by warp 0
         const unsigned long long t1 = globaltimer_ns();

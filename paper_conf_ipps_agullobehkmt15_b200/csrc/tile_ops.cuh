@@ -430,6 +430,30 @@ __device__ __forceinline__ void epi_sub_stage(Ctx<BS>& c, const Acc<BS>& acc, bo
   fence_proxy_async_shared();  // generic smem writes -> the TMA store (async proxy)
 }
 
+// Persistent kernel (sched.cu), K-loop jobs C -= A B^T: -acc staged in lbuf in the TMA box
+// layout (BS/16 boxes of BS rows x 128 B, 128B swizzle), which the storer warp adds to C in
+// global memory with TMA reduce-add stores (C + (-acc) == C - acc exactly) -- no C block is
+// read into the SM at all.  lower_only: the strictly upper part of the block gets -0.0
+// (x + -0.0 == x for every x), so the block's upper triangle is left as it is.  Ends with
+// the cross-proxy fence; the caller arrives on cready.
+template <int BS>
+__device__ __forceinline__ void epi_stage_neg(Ctx<BS>& c, const Acc<BS>& acc, bool lower_only) {
+  using C = Cfg<BS>;
+  const int wm = c.warp >> 2, wn = c.warp & 3, g = c.lane >> 2, t = c.lane & 3;
+  const uint32_t cs = smem_u32(c.lbuf());
+#pragma unroll
+  for (int mi = 0; mi < C::MI; ++mi)
+#pragma unroll
+    for (int ni = 0; ni < C::NI; ++ni) {
+      const int r = wm * C::WM + mi * 8 + g, cc = wn * C::WN + ni * 8 + 2 * t;
+      double2 v = make_double2(-acc[mi][ni][0], -acc[mi][ni][1]);
+      if (lower_only && cc > r) v.x = -0.0;
+      if (lower_only && cc + 1 > r) v.y = -0.0;
+      sts128(cs + (cc >> 4) * (BS * 128) + r * 128 + ((((cc & 15) >> 1) ^ (r & 7)) << 4), v);
+    }
+  fence_proxy_async_shared();
+}
+
 // lbuf offset (bytes) of element (r, cc), cc even, of a BS x BS block in the TMA box layout
 // (box cc/16, row r, logical 16-byte chunk (cc%16)/2, 128B swizzle)
 template <int BS>
