@@ -44,3 +44,32 @@ def test_uniform_entries_match_dense():
     i = rng.integers(0, n, 500)
     j = rng.integers(0, n, 500)
     assert np.array_equal(spdgen.uniform_entries(n, 3, i, j), A[i, j])
+
+
+def test_integer_family_block_inverses_are_exact():
+    """DESIGN R19: the inverse-form TRSM keeps the integer family exact because the inverses
+    of L0's diagonal 96-blocks (and whole 960-tiles) are small dyadic numbers.  Checked in
+    exact rational arithmetic on a few blocks (forward substitution with Fractions: every entry
+    is dyadic with a numerator below 2^53, i.e. exactly representable in FP64), and in FP64 on
+    every 96-block: the FP64 inverse times the block is the identity exactly."""
+    from fractions import Fraction
+    import numpy as np
+    for seed in (0, 3, 12):
+        n = 3840
+        L0 = spdgen.integer_L0(n, seed)
+        for b in range(0, n, 96):
+            L = L0[b:b + 96, b:b + 96]
+            X = np.linalg.solve(L, np.eye(96))
+            assert np.array_equal(L @ X, np.eye(96))
+            assert np.abs(X).max() <= 64.0
+        for b in (0, 960, 2880):  # exact rationals: every entry dyadic with a small numerator
+            L = [[Fraction(int(v)) for v in row] for row in L0[b:b + 96, b:b + 96]]
+            for col in range(96):
+                x = [Fraction(0)] * 96
+                for r in range(96):
+                    s = Fraction(1 if r == col else 0) - sum(L[r][m] * x[m] for m in range(max(0, r - 3), r))
+                    x[r] = s / L[r][r]
+                for v in x:
+                    assert v.denominator & (v.denominator - 1) == 0  # power of two
+                    assert abs(v.numerator) < 2 ** 53  # exactly representable in FP64
+                    assert Fraction(float(v)) == v
