@@ -19,7 +19,7 @@ for N in Ns:
         workers = c.chol_get_info(p.h)["workers"]
     t = sum(ts) / len(ts)
     args = types.SimpleNamespace(n=n, nb=nb, policy="cp", seed=0)
-    T_lat, T_thr = bench.calibrate(c, args, workers)
+    T_lat, T_thr = bench.calibrate(c, args)
     b = c.chol_bounds(n, nb, 1, T_lat, T_thr)
     fl = n ** 3 / 3
     print(json.dumps({"N": N, "n": n, "ms": round(t * 1e3, 3), "tflops": round(fl / t / 1e12, 3),
