@@ -234,6 +234,14 @@ int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs);
  * (plus the diagonal-block inverses when they were recomputed), seconds. */
 int chol_last_solve_times(chol_plan_t p, double* total_s, double* sweeps_s);
 
+/* Inject static task priorities into the device scheduler (the paper
+ * injects its CP schedules into StarPU): prio[t] for every Algorithm 1 task in
+ * chol_task_id order (ntasks = n_tasks(N)), higher runs first -- e.g. minus the start rank of
+ * chol_optimal_schedule.  Replaces the bottom-level priority buckets (CHOL_POLICY_CP_PRIORITY /
+ * STATIC; pinning kept) for the following factorizations; the factor is unchanged (R15).
+ * Errors: -4 null, -6 wrong ntasks, -8 not a persistent-scheduler plan. */
+int chol_set_task_priorities(chol_plan_t p, const double* prio, int64_t ntasks);
+
 /* Number of kernel launches the last chol_factor* issued (the persistent scheduler
  * issues 2: queue init + the scheduler kernel). */
 int chol_last_launches(chol_plan_t p, int* launches);
@@ -290,10 +298,14 @@ int chol_lp_bound(int64_t N, int nclasses, const int* workers, const double* tim
 
 /* Scheduler policies of the simulation (StarPU's, L645-660). */
 enum {
-  CHOL_SIM_DMDA = 0, /* ready tasks (release order) go to the worker with the minimum estimated
-                        completion time; each worker runs its queue in FIFO order */
-  CHOL_SIM_DMDAS = 1 /* the same, ready tasks and worker queues in bottom-level priority order
-                        (longest path to an exit task with each type's fastest time, L655-660) */
+  CHOL_SIM_DMDA = 0,  /* ready tasks (release order) go to the worker with the minimum estimated
+                         completion time; each worker runs its queue in FIFO order */
+  CHOL_SIM_DMDAS = 1, /* the same, ready tasks and worker queues in bottom-level priority order
+                         (longest path to an exit task with each type's fastest time, L655-660) */
+  CHOL_SIM_FIXED = 2  /* an injected static schedule (the paper's CP schedule replayed in
+                         simulation, L1056-1072): task t runs on worker fixed_worker[t], each worker
+                         runs its tasks in increasing fixed_rank[t] order, each as soon as its
+                         predecessors have finished and the worker is free */
 };
 typedef struct {
   int nclasses;                            /* 1 .. CHOL_SIM_MAX_CLASSES */
@@ -303,6 +315,8 @@ typedef struct {
   int gemm_syrk_class;                     /* static rule (L1000-1007): SYRK/GEMM only on this class; -1 off */
   int trsm_far_class;                      /* static rule (L1019-1025): TRSM_i_k with i-k >= */
   int trsm_far_distance;                   /*   trsm_far_distance only on trsm_far_class; -1 off */
+  const int32_t* fixed_worker;             /* CHOL_SIM_FIXED: worker per task (chol_task_id order) */
+  const int32_t* fixed_rank;               /* CHOL_SIM_FIXED: order of the task on its worker */
 } chol_sim_opts_t;
 
 /* Discrete-event replay of the Algorithm 1 task DAG for N tiles per side on the
@@ -313,6 +327,23 @@ typedef struct {
  * class (field gpu), worker, and t0/t1 in ns.  Errors: -1 N <= 0, -4 null pointer,
  * -6 bad options or a task no class may run. */
 int chol_simulate(int64_t N, const chol_sim_opts_t* opts, double* makespan, chol_task_rec_t* recs, int64_t cap);
+
+/* Exact minimum-makespan schedule of the Algorithm 1 DAG for small N (the
+ * paper's constraint-programming formulation, P:L409-464 -- one resource class per task,
+ * start times, cumulative resource limits, dependencies, no transfers -- solved to proven
+ * optimality where the paper's CP Optimizer ran 23 hours without a proof).
+ * Method: depth-first branch and bound over semi-active schedules generated in order of start
+ * time (every schedule can be left-shifted to a semi-active one, so one of them is optimal);
+ * identical workers of a class are interchangeable (a task goes to a worker of its class free
+ * earliest); bounds: the longest remaining path with each type's fastest time, the remaining
+ * work over all workers; initial incumbent: the dmdas replay.  The platform, the static rules
+ * and the times are those of *opts (policy and fixed_* ignored).  Outputs: *makespan;
+ * *optimal = 1 if the search completed, 0 if node_limit (0 = 2e8) stopped it first (the best
+ * schedule found is returned); worker / rank (may be NULL; n_tasks entries, chol_task_id
+ * order) -- a schedule CHOL_SIM_FIXED replays; *nodes = search nodes.  Errors: -1 N <= 0,
+ * -4 null pointer, -6 bad options, a task no class may run, or N > 8. */
+int chol_optimal_schedule(int64_t N, const chol_sim_opts_t* opts, int64_t node_limit, double* makespan,
+                          int* optimal, int32_t* worker, int32_t* rank, int64_t* nodes);
 
 #ifdef __cplusplus
 }

@@ -38,14 +38,15 @@ class chol_task_rec_t(ctypes.Structure):
 
 
 SIM_MAX_CLASSES = 4
-SIM_DMDA, SIM_DMDAS = 0, 1
+SIM_DMDA, SIM_DMDAS, SIM_FIXED = 0, 1, 2
 
 
 class chol_sim_opts_t(ctypes.Structure):
     _fields_ = [("nclasses", ctypes.c_int), ("workers", ctypes.c_int * SIM_MAX_CLASSES),
                 ("time", (ctypes.c_double * 4) * SIM_MAX_CLASSES), ("policy", ctypes.c_int),
                 ("gemm_syrk_class", ctypes.c_int), ("trsm_far_class", ctypes.c_int),
-                ("trsm_far_distance", ctypes.c_int)]
+                ("trsm_far_distance", ctypes.c_int), ("fixed_worker", ctypes.POINTER(ctypes.c_int32)),
+                ("fixed_rank", ctypes.POINTER(ctypes.c_int32))]
 
 
 def _load():
@@ -92,6 +93,10 @@ def _load():
         "chol_solve": ([P, vp, i64, i64], i32),
         "chol_last_solve_times": ([P, dp, dp], i32),
         "chol_simulate": ([i64, ctypes.POINTER(chol_sim_opts_t), dp, ctypes.POINTER(chol_task_rec_t), i64], i32),
+        "chol_set_task_priorities": ([P, dp, i64], i32),
+        "chol_optimal_schedule": ([i64, ctypes.POINTER(chol_sim_opts_t), i64, dp, ctypes.POINTER(i32),
+                                   ctypes.POINTER(ctypes.c_int32), ctypes.POINTER(ctypes.c_int32),
+                                   ctypes.POINTER(i64)], i32),
     }
     for name, (args, res) in sig.items():
         f = getattr(L, name)
@@ -107,7 +112,7 @@ EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_dest
             "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
             "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
             "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times", "chol_scatter_tiles",
-            "chol_gather_tiles", "chol_owner_area")
+            "chol_gather_tiles", "chol_owner_area", "chol_optimal_schedule", "chol_set_task_priorities")
 
 
 def _ptr(x) -> int:
@@ -236,6 +241,12 @@ def chol_run_batch(plan: int, type: int, count: int, reps: int = 1) -> float:
     return ms.value
 
 
+def chol_set_task_priorities(plan: int, prio) -> None:
+    """Static priorities per task (chol_task_id order, higher first) for the device scheduler."""
+    arr = (ctypes.c_double * len(prio))(*[float(v) for v in prio])
+    _check(_lib.chol_set_task_priorities(plan, arr, len(prio)), "chol_set_task_priorities")
+
+
 def chol_last_launches(plan: int) -> int:
     n = ctypes.c_int()
     _check(_lib.chol_last_launches(plan, ctypes.byref(n)), "chol_last_launches")
@@ -302,11 +313,7 @@ def chol_lp_bound(N: int, workers, times, mixed: bool = True):
     return l.value, [list(nrt[4 * r:4 * r + 4]) for r in range(R)]
 
 
-def chol_simulate(N: int, workers, times, policy: int = SIM_DMDAS, gemm_syrk_class: int = -1,
-                  trsm_far_class: int = -1, trsm_far_distance: int = 1, records: bool = False):
-    """Replay of the Algorithm 1 DAG on a platform of resource classes under dmda / dmdas
-    and the paper's static rules (chol_simulate in include/chol.h).  Returns the makespan
-    (seconds) and, with records=True, the per-task records (chol_task_id order)."""
+def _sim_opts(workers, times, policy, gemm_syrk_class, trsm_far_class, trsm_far_distance, fixed=None):
     o = chol_sim_opts_t()
     o.nclasses = len(workers)
     for r, (m, row) in enumerate(zip(workers, times)):
@@ -315,6 +322,22 @@ def chol_simulate(N: int, workers, times, policy: int = SIM_DMDAS, gemm_syrk_cla
             o.time[r][t] = float(row[t])
     o.policy, o.gemm_syrk_class, o.trsm_far_class, o.trsm_far_distance = policy, gemm_syrk_class, trsm_far_class, \
         trsm_far_distance
+    keep = None
+    if fixed is not None:
+        w, r = fixed
+        keep = ((ctypes.c_int32 * len(w))(*w), (ctypes.c_int32 * len(r))(*r))
+        o.fixed_worker = ctypes.cast(keep[0], ctypes.POINTER(ctypes.c_int32))
+        o.fixed_rank = ctypes.cast(keep[1], ctypes.POINTER(ctypes.c_int32))
+    return o, keep
+
+
+def chol_simulate(N: int, workers, times, policy: int = SIM_DMDAS, gemm_syrk_class: int = -1,
+                  trsm_far_class: int = -1, trsm_far_distance: int = 1, records: bool = False, fixed=None):
+    """Replay of the Algorithm 1 DAG on a platform of resource classes under dmda / dmdas,
+    the paper's static rules, or an injected schedule (policy SIM_FIXED, fixed = (worker per
+    task, rank per task)) -- chol_simulate in include/chol.h.  Returns the makespan (seconds)
+    and, with records=True, the per-task records (chol_task_id order)."""
+    o, keep = _sim_opts(workers, times, policy, gemm_syrk_class, trsm_far_class, trsm_far_distance, fixed)
     mk = ctypes.c_double()
     nt = N + N * (N - 1) + N * (N - 1) * (N - 2) // 6
     recs = (chol_task_rec_t * nt)() if records else None
@@ -323,6 +346,19 @@ def chol_simulate(N: int, workers, times, policy: int = SIM_DMDAS, gemm_syrk_cla
         return mk.value
     return mk.value, [{"type": r.type, "cls": r.gpu, "worker": r.worker, "i": r.i, "j": r.j, "k": r.k,
                        "t0_ns": r.t0_ns, "t1_ns": r.t1_ns} for r in recs]
+
+
+def chol_optimal_schedule(N: int, workers, times, gemm_syrk_class: int = -1, trsm_far_class: int = -1,
+                          trsm_far_distance: int = 1, node_limit: int = 0):
+    """Exact minimum-makespan schedule (branch and bound, include/chol.h).  Returns
+    (makespan, optimal, worker per task, rank per task, search nodes)."""
+    o, _ = _sim_opts(workers, times, SIM_DMDAS, gemm_syrk_class, trsm_far_class, trsm_far_distance)
+    nt = N + N * (N - 1) + N * (N - 1) * (N - 2) // 6
+    mk, opt, nodes = ctypes.c_double(), ctypes.c_int(), ctypes.c_int64()
+    w, r = (ctypes.c_int32 * nt)(), (ctypes.c_int32 * nt)()
+    _check(_lib.chol_optimal_schedule(N, ctypes.byref(o), node_limit, ctypes.byref(mk), ctypes.byref(opt), w, r,
+                                      ctypes.byref(nodes)), "chol_optimal_schedule")
+    return mk.value, bool(opt.value), list(w), list(r), nodes.value
 
 
 def chol_plan_dist(n: int, nb: int, nranks: int, rank: int, **opts) -> int:

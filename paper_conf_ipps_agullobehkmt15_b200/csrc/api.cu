@@ -1095,6 +1095,18 @@ extern "C" int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* 
   return 0;
 }
 
+extern "C" int chol_set_task_priorities(chol_plan_t p, const double* prio, int64_t ntasks) {
+  if (!p || !prio) return -4;
+  if (is_multi(p)) {
+    for (chol_plan_s* sp : p->subs)
+      if (const int st = chol_set_task_priorities(sp, prio, ntasks)) return st;
+    return 0;
+  }
+  if (!p->sched) return -8;
+  cudaSetDevice(p->device);
+  return sched_set_priorities(p->sched, prio, ntasks);
+}
+
 extern "C" int chol_last_launches(chol_plan_t p, int* launches) {
   if (!p || !launches) return -4;
   *launches = p->last_launches;

@@ -828,6 +828,9 @@ struct SchedState {
   uint64_t* job_trace = nullptr;           // device, 4 per job (trace == 2)
   int* d_abort = nullptr;                  // device abort flag (d.abort_flag), written by sched_abort
   CUtensorMap dmap{};                      // Dinv workspace map (sched_set_dinv)
+  // re-bucketing with injected task priorities (sched_set_priorities)
+  std::vector<int> h_node_paper, h_node_queue;
+  size_t o_nq = 0, o_qbase = 0;
   std::vector<int16_t> h_job_type;         // host copies for chol_job_trace
   std::vector<int> h_job_paper;
 };
@@ -1043,6 +1046,8 @@ static int sched_upload(SchedState** out, SchedState* st, Builder& B, const std:
     if (B.deps[v] == 0) roots.push_back(v);
 
   st->nnodes = nnodes;
+  st->h_node_paper = B.paper;
+  st->h_node_queue = node_queue;
   st->njobs = (int)B.jobs.size();
   st->h_job_type.resize(st->njobs);
   st->h_job_paper.resize(st->njobs);
@@ -1077,6 +1082,8 @@ static int sched_upload(SchedState** out, SchedState* st, Builder& B, const std:
   if (!succ.empty()) memcpy(h.data() + o_succ, succ.data(), succ.size() * 4);
   memcpy(h.data() + o_paper, B.paper.data(), nnodes * 4);
   memcpy(h.data() + o_nq, node_queue.data(), nnodes * 4);
+  st->o_nq = o_nq;
+  st->o_qbase = o_qbase;
   memcpy(h.data() + o_qbase, qbase.data(), kQueues * 4);
   if (!roots.empty()) memcpy(h.data() + o_roots, roots.data(), roots.size() * 4);
   if (!publish.empty()) memcpy(h.data() + o_pub, publish.data(), publish.size() * 4);
@@ -1667,6 +1674,34 @@ int sched_create_batch(SchedState** out, int64_t N, int64_t nb, int bs, int sms,
   std::vector<int> node_queue(B.deps.size(), 0), publish;
   std::vector<int4> watch;
   return sched_upload(out, st, B, node_queue, publish, watch, opts, nb, bs, sms);
+}
+
+// Injected static priorities (NEXT-4: the paper injects its CP schedules into StarPU,
+// P:L1063-1072): prio[paper task id] (higher = earlier) replaces the bottom-level bucket of
+// every task node; pinned classes (STATIC) and the untraced gating nodes (RECV, INV: top
+// bucket) are kept.  Rewrites the node -> queue table and the queue bases on the device.
+int sched_set_priorities(SchedState* st, const double* prio, int64_t ntasks) {
+  if (!st || !prio) return -4;
+  if (ntasks != n_tasks(st->N)) return -6;
+  double lo = prio[0], hi = prio[0];
+  for (int64_t t = 1; t < ntasks; ++t) lo = std::min(lo, prio[t]), hi = std::max(hi, prio[t]);
+  const double span = hi - lo > 0 ? hi - lo : 1.0;
+  std::vector<int> nq(st->nnodes);
+  for (int v = 0; v < st->nnodes; ++v) {
+    const int pinned = st->h_node_queue[v] >= kBuckets ? kBuckets : 0;
+    const int p = st->h_node_paper[v];
+    const int bucket = p < 0 ? kBuckets - 1 : std::min(kBuckets - 1, (int)((kBuckets - 1) * (prio[p] - lo) / span));
+    nq[v] = bucket + pinned;
+  }
+  std::vector<int> qcap(kQueues, 0), qbase(kQueues, 0);
+  for (int v = 0; v < st->nnodes; ++v) qcap[nq[v]] += 1;
+  for (int q = 1; q < kQueues; ++q) qbase[q] = qbase[q - 1] + qcap[q - 1];
+  char* S = static_cast<char*>(st->dev_static);
+  cudaError_t e = cudaMemcpy(S + st->o_nq, nq.data(), nq.size() * 4, cudaMemcpyHostToDevice);
+  if (!e) e = cudaMemcpy(S + st->o_qbase, qbase.data(), kQueues * 4, cudaMemcpyHostToDevice);
+  if (e) return -100 - (int)e;
+  st->h_node_queue = nq;
+  return 0;
 }
 
 int sched_set_dinv(SchedState* st, double* dinv, const CUtensorMap& dmap) {

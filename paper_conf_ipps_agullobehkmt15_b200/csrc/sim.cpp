@@ -188,7 +188,8 @@ extern "C" int chol_simulate(int64_t N, const chol_sim_opts_t* o, double* makesp
                              int64_t cap) {
   if (N <= 0) return -1;
   if (!o || !makespan) return -4;
-  if (o->nclasses < 1 || o->nclasses > CHOL_SIM_MAX_CLASSES || o->policy < 0 || o->policy > 1) return -6;
+  if (o->nclasses < 1 || o->nclasses > CHOL_SIM_MAX_CLASSES || o->policy < 0 || o->policy > 2) return -6;
+  if (o->policy == CHOL_SIM_FIXED && (!o->fixed_worker || !o->fixed_rank)) return -4;
   const int R = o->nclasses;
   // workers, their classes
   std::vector<int> wcls;
@@ -251,7 +252,20 @@ extern "C" int chol_simulate(int64_t N, const chol_sim_opts_t* o, double* makesp
   std::priority_queue<Ev, std::vector<Ev>, std::greater<Ev>> events;
   std::vector<int64_t> running(W, -1);
 
+  if (o->policy == CHOL_SIM_FIXED)
+    for (int64_t t = 0; t < nt; ++t) {
+      const int w = o->fixed_worker[t];
+      if (w < 0 || w >= W || !runs_on(*o, wcls[w], type_of[t], ti[t], tk[t])) return -6;
+    }
   auto assign = [&](std::vector<int64_t>& ready, double now) {
+    if (o->policy == CHOL_SIM_FIXED) {  // the injected schedule's worker
+      for (int64_t t : ready) {
+        wq[o->fixed_worker[t]].push_back(t);
+        twork[t] = o->fixed_worker[t];
+      }
+      ready.clear();
+      return;
+    }
     if (o->policy == 1)  // dmdas: highest priority first (ties: lower id)
       std::stable_sort(ready.begin(), ready.end(), [&](int64_t a, int64_t b) { return prio[a] > prio[b]; });
     for (int64_t t : ready) {
@@ -268,9 +282,31 @@ extern "C" int chol_simulate(int64_t N, const chol_sim_opts_t* o, double* makesp
     }
     ready.clear();
   };
+  // CHOL_SIM_FIXED: position of each worker in its injected order (next rank to run)
+  std::vector<std::vector<int64_t>> worder(W);
+  std::vector<size_t> wnext(W, 0);
+  if (o->policy == CHOL_SIM_FIXED) {
+    for (int64_t t = 0; t < nt; ++t) worder[o->fixed_worker[t]].push_back(t);
+    for (auto& v : worder)
+      std::stable_sort(v.begin(), v.end(), [&](int64_t a, int64_t b) { return o->fixed_rank[a] < o->fixed_rank[b]; });
+  }
   auto start_idle = [&](double now) {
     for (int w = 0; w < W; ++w) {
       if (busy[w] || wq[w].empty()) continue;
+      if (o->policy == CHOL_SIM_FIXED) {  // only the worker's next task in the injected order
+        if (wnext[w] >= worder[w].size()) continue;
+        const int64_t t = worder[w][wnext[w]];
+        auto it = std::find(wq[w].begin(), wq[w].end(), t);
+        if (it == wq[w].end()) continue;  // not ready yet
+        wq[w].erase(it);
+        ++wnext[w];
+        busy[w] = 1;
+        running[w] = t;
+        t0[t] = now;
+        t1[t] = now + o->time[wcls[w]][type_of[t]];
+        events.push(Ev(t1[t], w));
+        continue;
+      }
       size_t pick = 0;
       if (o->policy == 1)
         for (size_t q = 1; q < wq[w].size(); ++q)
@@ -322,5 +358,200 @@ extern "C" int chol_simulate(int64_t N, const chol_sim_opts_t* o, double* makesp
       r.t0_ns = (uint64_t)std::llround(t0[t] * 1e9);
       r.t1_ns = (uint64_t)std::llround(t1[t] * 1e9);
     }
+  return 0;
+}
+
+// ------------------------------------------------------------------ exact schedules (NEXT-4)
+namespace {
+struct ExactSearch {
+  int64_t nt = 0;
+  int W = 0, R = 0;
+  const chol_sim_opts_t* o = nullptr;
+  std::vector<int> type_of, ti, tk, wcls;
+  std::vector<std::vector<int>> succ, pred;
+  std::vector<int> topo;                 // a topological order (task ids are one)
+  std::vector<double> fast, blev;        // fastest time over the allowed classes; bottom level
+  std::vector<std::vector<int>> cls_workers;
+  // state
+  std::vector<double> fin, st;
+  std::vector<int> wk, npred;
+  std::vector<double> wfree;
+  double best = INFINITY;
+  std::vector<double> best_st;
+  std::vector<int> best_wk;
+  int64_t nodes = 0, limit = 0;
+  bool stopped = false;
+  std::vector<double> es;  // scratch: earliest starts
+
+  double lower_bound(double cur_mk) {
+    // longest remaining path: earliest start of every unscheduled task (scheduled
+    // predecessors: their finish; unscheduled ones: their earliest start + fastest time)
+    double lb = cur_mk, work = 0.0;
+    for (int t : topo) {
+      if (fin[t] >= 0.0) continue;
+      double e = 0.0;
+      for (int p : pred[t]) e = std::max(e, fin[p] >= 0.0 ? fin[p] : es[p] + fast[p]);
+      es[t] = e;
+      lb = std::max(lb, e + blev[t]);
+      work += fast[t];
+    }
+    double busy = 0.0;
+    for (int w = 0; w < W; ++w) busy += wfree[w];
+    return std::max(lb, (busy + work) / W);
+  }
+
+  void dfs(int nsched, double cur_mk, double cursor, int last_task) {
+    if (stopped) return;
+    if (nsched == nt) {
+      if (cur_mk < best) {
+        best = cur_mk;
+        best_st = st;
+        best_wk = wk;
+      }
+      return;
+    }
+    if (++nodes > limit) {
+      stopped = true;
+      return;
+    }
+    if (lower_bound(cur_mk) >= best - 1e-12) return;
+    struct Cand {
+      double est, ect;
+      int t, w;
+    };
+    std::vector<Cand> cand;
+    for (int t = 0; t < nt; ++t) {
+      if (fin[t] >= 0.0 || npred[t] != 0) continue;
+      double ready = 0.0;
+      for (int p : pred[t]) ready = std::max(ready, fin[p]);
+      for (int r = 0; r < R; ++r) {
+        if (cls_workers[r].empty() || !runs_on(*o, r, type_of[t], ti[t], tk[t])) continue;
+        int bw = cls_workers[r][0];
+        for (int w : cls_workers[r])
+          if (wfree[w] < wfree[bw]) bw = w;
+        const double est = std::max(ready, wfree[bw]);
+        // start-time order (ties by task id): every semi-active schedule is generated once
+        if (est < cursor - 1e-12 || (est <= cursor + 1e-12 && t <= last_task && nsched > 0)) continue;
+        cand.push_back({est, est + o->time[r][type_of[t]], t, bw});
+      }
+    }
+    std::sort(cand.begin(), cand.end(), [](const Cand& a, const Cand& b) {
+      return a.ect != b.ect ? a.ect < b.ect : (a.est != b.est ? a.est < b.est : a.t < b.t);
+    });
+    for (const Cand& c : cand) {
+      if (c.ect >= best - 1e-12) continue;
+      const double old_free = wfree[c.w];
+      fin[c.t] = c.ect;
+      st[c.t] = c.est;
+      wk[c.t] = c.w;
+      wfree[c.w] = c.ect;
+      for (int s : succ[c.t]) --npred[s];
+      dfs(nsched + 1, std::max(cur_mk, c.ect), c.est, c.t);
+      for (int s : succ[c.t]) ++npred[s];
+      wfree[c.w] = old_free;
+      fin[c.t] = -1.0;
+      wk[c.t] = -1;
+      if (stopped) return;
+    }
+  }
+};
+}  // namespace
+
+extern "C" int chol_optimal_schedule(int64_t N, const chol_sim_opts_t* o, int64_t node_limit, double* makespan,
+                                     int* optimal, int32_t* worker, int32_t* rank, int64_t* nodes) {
+  if (N <= 0) return -1;
+  if (!o || !makespan) return -4;
+  if (N > 8 || o->nclasses < 1 || o->nclasses > CHOL_SIM_MAX_CLASSES) return -6;
+  ExactSearch S;
+  S.o = o;
+  S.R = o->nclasses;
+  S.cls_workers.resize(S.R);
+  for (int r = 0; r < S.R; ++r) {
+    if (o->workers[r] < 0) return -6;
+    for (int w = 0; w < o->workers[r]; ++w) {
+      S.cls_workers[r].push_back((int)S.wcls.size());
+      S.wcls.push_back(r);
+    }
+  }
+  S.W = (int)S.wcls.size();
+  if (S.W == 0) return -6;
+  std::vector<std::pair<int64_t, int64_t>> E;
+  build_task_dag(N, E, S.type_of);
+  S.nt = n_tasks(N);
+  S.ti.assign(S.nt, 0);
+  S.tk.assign(S.nt, 0);
+  for (int64_t k = 0; k < N; ++k) {
+    S.ti[id_potrf(N, k)] = (int)k, S.tk[id_potrf(N, k)] = (int)k;
+    for (int64_t i = k + 1; i < N; ++i) S.ti[id_trsm(N, i, k)] = (int)i, S.tk[id_trsm(N, i, k)] = (int)k;
+  }
+  S.succ.assign(S.nt, {});
+  S.pred.assign(S.nt, {});
+  for (auto& e : E) {
+    S.succ[e.first].push_back((int)e.second);
+    S.pred[e.second].push_back((int)e.first);
+  }
+  // topological order (Kahn)
+  std::vector<int> indeg(S.nt, 0);
+  for (auto& e : E) ++indeg[e.second];
+  for (int t = 0; t < S.nt; ++t)
+    if (!indeg[t]) S.topo.push_back(t);
+  for (size_t h = 0; h < S.topo.size(); ++h)
+    for (int s : S.succ[S.topo[h]])
+      if (--indeg[s] == 0) S.topo.push_back(s);
+  S.fast.assign(S.nt, INFINITY);
+  for (int t = 0; t < S.nt; ++t) {
+    for (int r = 0; r < S.R; ++r)
+      if (o->workers[r] > 0 && runs_on(*o, r, S.type_of[t], S.ti[t], S.tk[t]))
+        S.fast[t] = std::min(S.fast[t], o->time[r][S.type_of[t]]);
+    if (std::isinf(S.fast[t])) return -6;
+  }
+  S.blev.assign(S.nt, 0.0);
+  for (int h = (int)S.topo.size() - 1; h >= 0; --h) {
+    const int t = S.topo[h];
+    double m = 0.0;
+    for (int s : S.succ[t]) m = std::max(m, S.blev[s]);
+    S.blev[t] = S.fast[t] + m;
+  }
+  // incumbent: the dmdas replay
+  {
+    chol_sim_opts_t od = *o;
+    od.policy = CHOL_SIM_DMDAS;
+    std::vector<chol_task_rec_t> recs(S.nt);
+    double mk = 0.0;
+    if (chol_simulate(N, &od, &mk, recs.data(), S.nt) == 0) {
+      S.best = mk + 1e-9;  // strictly better schedules only; kept if none is found
+      S.best_st.resize(S.nt);
+      S.best_wk.resize(S.nt);
+      for (int t = 0; t < S.nt; ++t) {
+        S.best_st[t] = recs[t].t0_ns * 1e-9;
+        S.best_wk[t] = recs[t].worker;
+      }
+    }
+  }
+  S.fin.assign(S.nt, -1.0);
+  S.st.assign(S.nt, 0.0);
+  S.wk.assign(S.nt, -1);
+  S.npred.assign(S.nt, 0);
+  for (int t = 0; t < S.nt; ++t) S.npred[t] = (int)S.pred[t].size();
+  S.wfree.assign(S.W, 0.0);
+  S.es.assign(S.nt, 0.0);
+  S.limit = node_limit > 0 ? node_limit : (int64_t)200000000;
+  S.dfs(0, 0.0, 0.0, -1);
+  if (S.best_wk.empty()) return -6;
+  // the schedule's exact makespan (the dmdas incumbent carried a 1e-9 guard)
+  double mk = 0.0;
+  for (int t = 0; t < S.nt; ++t) mk = std::max(mk, S.best_st[t] + o->time[S.wcls[S.best_wk[t]]][S.type_of[t]]);
+  *makespan = mk;
+  if (optimal) *optimal = S.stopped ? 0 : 1;
+  if (nodes) *nodes = S.nodes;
+  if (worker || rank) {
+    std::vector<int> ord(S.nt);
+    for (int t = 0; t < S.nt; ++t) ord[t] = t;
+    std::stable_sort(ord.begin(), ord.end(), [&](int a, int b) { return S.best_st[a] < S.best_st[b]; });
+    for (int r = 0; r < S.nt; ++r) {
+      if (worker) worker[ord[r]] = S.best_wk[ord[r]];
+      if (rank) rank[ord[r]] = r;
+    }
+  }
   return 0;
 }

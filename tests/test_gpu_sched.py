@@ -144,3 +144,30 @@ def test_non_spd_leading_columns_final_task_level_path():
         dA = torch.from_numpy(A).cuda()
         assert p.factor(dA) == j0 + 1
         assert torch.equal(dA[:, :j0].cpu(), torch.from_numpy(np.ascontiguousarray(L0[:, :j0])))
+
+
+def test_injected_priorities_keep_the_factor():
+    """NEXT-4: static priorities from an exact task-level schedule (chol_optimal_schedule)
+    injected into the device scheduler change only the order in which ready tasks run, never
+    the factor (R15); wrong lengths are rejected."""
+    c = _lib()
+    N, nb = 4, 960
+    n = N * nb
+    mk, optimal, w, r, _ = c.chol_optimal_schedule(N, [2], [[5e-4, 3.5e-4, 1e-4, 1e-4]])
+    assert optimal
+    outs = []
+    for inject in (False, True):
+        with c.Plan(n, nb, executor=c.EXEC_SCHEDULER) as p:
+            if inject:
+                c.chol_set_task_priorities(p.h, [-x for x in r])
+            c.chol_generate(p.h, 3, 0)
+            assert c.chol_factor_inplace(p.h) == 0
+            L = torch.empty((n, n), dtype=torch.float64, device="cuda")
+            c.chol_gather(p.h, L, n)
+            outs.append(L.cpu().numpy())
+            with pytest.raises(c.CholError) as e:
+                c.chol_set_task_priorities(p.h, [0.0] * (len(r) - 1))
+            assert e.value.status == -6
+    assert np.array_equal(outs[0], outs[1])
+    ref, _ = oracle.chol_tiled(spdgen.uniform_spd(n, 3), nb)
+    assert oracle.rel_diff(outs[1], ref)["max_rel_floored"] <= 1e-10
