@@ -1252,7 +1252,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // N = 12..24 (n=3840 3.76 -> 2.82 ms, n=9600 13.07 -> 12.18, n=19200 71.82 -> 71.57).
   // Single GPU only.  CHOL_BLOCK_TAIL=m overrides (m steps).
   const char* ebt = getenv("CHOL_BLOCK_TAIL");
-  int block_tail = ebt ? atoi(ebt) : (N <= 10 ? 4 : 2);
+  // round-2 sweep (profiles/r02/block_tail_sweep_r02.txt): m = 4 for N <= 6, 3 for N = 7..10
+  // (n=9600 11.78 -> 11.25 ms, n=7680 8.11 -> 7.93), 2 above
+  int block_tail = ebt ? atoi(ebt) : (N <= 6 ? 4 : N <= 10 ? 3 : 2);
   if (dist) block_tail = 0;
   const int k0 = (int)N - std::max(0, std::min(block_tail, (int)N));
   // blocked-region TRSM: per-slab TS/TU chains (0) or one left-looking slab job per
