@@ -80,6 +80,11 @@ typedef struct {
                             2 = also per-job (CTA sub-task) records (chol_job_trace) */
   int executor;          /* CHOL_EXEC_* */
   int workers;           /* persistent CTAs (0 = one per SM) */
+  int cpu_trsm_distance; /* > 0: the host CPU cores are a second resource class -- every
+                            TRSM_i_k with i-k >= d runs on them (the paper's static rule,
+                            P:L1019-1025, executed in Fig. 11; NEXT-3, DESIGN.md
+                            §7f); single-GPU persistent-scheduler plans only (else -6) */
+  int cpu_threads;       /* host threads of that class (0 = all host cores) */
 } chol_opts_t;
 
 /* One trace record per task (Fig. 12). */
@@ -253,6 +258,13 @@ int chol_last_launches(chol_plan_t p, int* launches);
  * dependencies (L213-220); edges[2e], edges[2e+1] = (pred, succ) dense task ids
  * (chol_task_id), at most cap edges written (edges may be NULL). */
 int chol_dag(int64_t N, int64_t* ntasks, int64_t* nedges, int64_t* edges, int64_t cap);
+
+/* The host CPU class's TRSM tile kernel (NEXT-3; host only): X (nb x nb, row-major) <- X L^{-T}
+ * for the lower triangular L (nb x nb, row-major; only its lower triangle is read), in the
+ * inverse form of the device (R19: the inverses of L's bs x bs diagonal blocks by
+ * substitution, then two products per column block), AVX-512 when the CPU has it, one thread.
+ * Errors: -4 null pointer, -6 nb % bs, nb % 4 or bs % 8 != 0. */
+int chol_cpu_trsm(double* X, const double* L, int64_t nb, int bs);
 
 /* Multi-GPU layout of rank `rank` on the p x q grid (host only): *nowned tiles owned,
  * *ncached remote panel tiles received; slot_map[t] (t = i(i+1)/2 + j, at most cap

@@ -8,8 +8,8 @@ import sys
 HERE = os.path.dirname(os.path.abspath(__file__))
 CSRC = os.path.join(HERE, "csrc")
 LIB = os.path.join(HERE, "libchol_b200.so")
-SOURCES = ["api.cu", "kernels.cu", "sched.cu", "solve.cu", "dag.cpp", "sim.cpp"]
-HEADERS = ["dev_common.cuh", "tile_ops.cuh", "kernels.h", "sched.h", "solve.h", "taskid.h", "dag.h"]
+SOURCES = ["api.cu", "kernels.cu", "sched.cu", "solve.cu", "dag.cpp", "sim.cpp", "hetero.cpp"]
+HEADERS = ["dev_common.cuh", "tile_ops.cuh", "kernels.h", "sched.h", "solve.h", "taskid.h", "dag.h", "hetero.h"]
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 FLAGS = ["-O3", "-std=c++17", "-gencode", "arch=compute_100a,code=sm_100a", "-lineinfo",
          "-Xcompiler", "-fPIC", "-Xcompiler", "-O2", "--expt-relaxed-constexpr"]

@@ -28,7 +28,8 @@ class CholError(RuntimeError):
 class chol_opts_t(ctypes.Structure):
     _fields_ = [("policy", ctypes.c_int), ("trsm_pin_distance", ctypes.c_int),
                 ("latency_workers", ctypes.c_int), ("grid_p", ctypes.c_int), ("grid_q", ctypes.c_int),
-                ("trace", ctypes.c_int), ("executor", ctypes.c_int), ("workers", ctypes.c_int)]
+                ("trace", ctypes.c_int), ("executor", ctypes.c_int), ("workers", ctypes.c_int),
+                ("cpu_trsm_distance", ctypes.c_int), ("cpu_threads", ctypes.c_int)]
 
 
 class chol_task_rec_t(ctypes.Structure):
@@ -94,6 +95,7 @@ def _load():
         "chol_last_solve_times": ([P, dp, dp], i32),
         "chol_simulate": ([i64, ctypes.POINTER(chol_sim_opts_t), dp, ctypes.POINTER(chol_task_rec_t), i64], i32),
         "chol_set_task_priorities": ([P, dp, i64], i32),
+        "chol_cpu_trsm": ([vp, vp, i64, i32], i32),
         "chol_optimal_schedule": ([i64, ctypes.POINTER(chol_sim_opts_t), i64, dp, ctypes.POINTER(i32),
                                    ctypes.POINTER(ctypes.c_int32), ctypes.POINTER(ctypes.c_int32),
                                    ctypes.POINTER(i64)], i32),
@@ -112,7 +114,8 @@ EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_dest
             "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
             "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
             "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times", "chol_scatter_tiles",
-            "chol_gather_tiles", "chol_owner_area", "chol_optimal_schedule", "chol_set_task_priorities")
+            "chol_gather_tiles", "chol_owner_area", "chol_optimal_schedule", "chol_set_task_priorities",
+            "chol_cpu_trsm")
 
 
 def _ptr(x) -> int:
@@ -245,6 +248,12 @@ def chol_set_task_priorities(plan: int, prio) -> None:
     """Static priorities per task (chol_task_id order, higher first) for the device scheduler."""
     arr = (ctypes.c_double * len(prio))(*[float(v) for v in prio])
     _check(_lib.chol_set_task_priorities(plan, arr, len(prio)), "chol_set_task_priorities")
+
+
+def chol_cpu_trsm(X, L, bs: int = 96) -> None:
+    """X <- X L^{-T} on the host CPU (the NEXT-3 class's tile kernel); X, L numpy (nb x nb)."""
+    nb = X.shape[0]
+    _check(_lib.chol_cpu_trsm(_ptr(X), _ptr(L), nb, bs), "chol_cpu_trsm")
 
 
 def chol_last_launches(plan: int) -> int:

@@ -15,6 +15,7 @@
 
 #include "../../include/chol.h"
 #include "dag.h"
+#include "hetero.h"
 #include "kernels.h"
 #include "sched.h"
 #include "solve.h"
@@ -57,7 +58,10 @@ struct chol_plan_s {
   unsigned epoch = 0;
   // ---- single GPU, persistent scheduler: streamed host input / output (chol_factor)
   int* d_in_flags = nullptr;   // per tile: epoch in which its input copy landed (device)
-  int* h_out_flags = nullptr;  // per tile: epoch in which it became final (host-mapped)
+  int* h_out_flags = nullptr;  // per tile: epoch in which it became final (host-mapped); second half:
+                               // epoch in which a host-class TRSM's inputs became final
+  int* d_host_flags = nullptr; // per tile: epoch in which the host class wrote L_ik back (device)
+  HostTrsm* host = nullptr;    // host CPU class (opts.cpu_trsm_distance > 0)
   int* d_out_flags = nullptr;  // device alias of h_out_flags
   int* h_epoch = nullptr;      // pinned source of the 4-byte arrival-flag copies
   cudaStream_t s_in = nullptr, s_out = nullptr;
@@ -158,6 +162,7 @@ extern "C" int chol_destroy(chol_plan_t p) {
     delete p;
     return 0;
   }
+  if (p->host) host_trsm_destroy(p->host);
   if (p->sched) sched_destroy(p->sched);
   cudaSetDevice(p->device);
   sched_phase_dump();
@@ -176,6 +181,7 @@ extern "C" int chol_destroy(chol_plan_t p) {
   cudaFree(p->d_peer_slots);
   cudaFree(p->d_peer_flags);
   cudaFree(p->d_in_flags);
+  cudaFree(p->d_host_flags);
   if (p->h_out_flags) cudaFreeHost(p->h_out_flags);
   if (p->h_epoch) cudaFreeHost(p->h_epoch);
   if (p->s_in) cudaStreamDestroy(p->s_in);
@@ -206,8 +212,9 @@ extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t*
   if (o) opts = *o;
   if (opts.policy < 0 || opts.policy > 2 || opts.executor < 0 || opts.executor > 1 || opts.trsm_pin_distance < 0 ||
       opts.latency_workers < 0 || opts.workers < 0 || opts.grid_p < 0 || opts.grid_q < 0 || opts.trace < 0 ||
-      opts.trace > 2)
+      opts.trace > 2 || opts.cpu_trsm_distance < 0 || opts.cpu_threads < 0)
     return -6;
+  if (opts.cpu_trsm_distance > 0 && (ngpus != 1 || opts.executor != CHOL_EXEC_SCHEDULER)) return -6;
   int ndev = 0;
   if (cudaGetDeviceCount(&ndev) != cudaSuccess) {
     cudaGetLastError();
@@ -270,17 +277,24 @@ extern "C" int chol_plan_ex(int64_t n, int64_t nb, int ngpus, const chol_opts_t*
     sched_set_dinv(p->sched, p->d_dinv, p->dmap);
     // arrival flags (device), publish flags (host-mapped, polled by chol_factor), copy streams
     if ((e = cudaMalloc(&p->d_in_flags, p->ntiles * sizeof(int))) ||
-        (e = cudaHostAlloc(&p->h_out_flags, p->ntiles * sizeof(int), cudaHostAllocMapped)) ||
+        (e = cudaHostAlloc(&p->h_out_flags, 2 * p->ntiles * sizeof(int), cudaHostAllocMapped)) ||
         (e = cudaHostGetDevicePointer(&p->d_out_flags, p->h_out_flags, 0)) ||
         (e = cudaHostAlloc(&p->h_epoch, sizeof(int), cudaHostAllocDefault)) ||
-        (e = cudaMalloc(&p->d_peer_flags, sizeof(int*))) ||
+        (e = cudaMalloc(&p->d_host_flags, p->ntiles * sizeof(int))) ||
+        (e = cudaMalloc(&p->d_peer_flags, 2 * sizeof(int*))) ||
         (e = cudaStreamCreateWithFlags(&p->s_in, cudaStreamNonBlocking)) ||
         (e = cudaStreamCreateWithFlags(&p->s_out, cudaStreamNonBlocking)))
       return fail(-100 - (int)e);
-    memset(p->h_out_flags, 0, p->ntiles * sizeof(int));
+    memset(p->h_out_flags, 0, 2 * p->ntiles * sizeof(int));
     cudaMemset(p->d_in_flags, 0, p->ntiles * sizeof(int));
-    cudaMemcpy(p->d_peer_flags, &p->d_in_flags, sizeof(int*), cudaMemcpyHostToDevice);
+    cudaMemset(p->d_host_flags, 0, p->ntiles * sizeof(int));
+    int* watched[2] = {p->d_in_flags, p->d_host_flags};  // watch owner 0: input arrival, 1: host class
+    cudaMemcpy(p->d_peer_flags, watched, 2 * sizeof(int*), cudaMemcpyHostToDevice);
     sched_set_dist(p->sched, nullptr, nullptr, nullptr, p->d_peer_flags, p->d_out_flags);
+    if (!sched_host_tasks(p->sched).empty() &&
+        (st = host_trsm_create(&p->host, p->device, (int)nb, p->bs, opts.cpu_threads, p->ntiles, p->tiles, p->d_dinv,
+                               p->d_host_flags, p->h_out_flags + p->ntiles, sched_host_tasks(p->sched))))
+      return fail(st);
   }
   *out = p;
   return 0;
@@ -831,6 +845,7 @@ static int factor_launch(chol_plan_s* p) {
   else
     st = sched_run(p->sched, p->map, base_params(p), p->stream, &nl, p->epoch);
   if (st) return st;
+  if (p->host) host_trsm_start(p->host, p->epoch);  // the host class follows the kernel's flags
   CUDA_TRY(cudaEventRecord(p->ev1, p->stream));
   p->last_launches = nl;
   return 0;
@@ -906,7 +921,12 @@ static int wait_plan(chol_plan_s* p) {
 
 static int finish_info(chol_plan_s* p, int* info) {
   int h = 0;
-  if (const int w = wait_plan(p)) return w;
+  if (const int w = wait_plan(p)) {
+    if (p->host) host_trsm_finish(p->host, true);
+    return w;
+  }
+  if (p->host)
+    if (const int hs = host_trsm_finish(p->host, false)) return hs;
   CUDA_TRY(cudaMemcpyAsync(&h, p->d_info, sizeof(int), cudaMemcpyDeviceToHost, p->stream));
   CUDA_TRY(cudaStreamSynchronize(p->stream));
   float ms = 0.f;
@@ -1086,9 +1106,19 @@ extern "C" int chol_factor(chol_plan_t p, const double* A, int64_t lda, double* 
   int st = scatter_impl(p, A, lda);
   if (st) return st;
   if ((st = factor_launch(p))) return st;
-  if ((st = gather_impl(p, L, ldl))) return st;
-  CUDA_TRY(cudaEventRecord(p->ev3, p->stream));
-  if ((st = finish_info(p, info))) return st;
+  if (p->host) {
+    // with the host CPU class nothing may wait behind the kernel on p->stream while it runs:
+    // copies queued there share the copy engines' hardware queues with the host driver's
+    // copies, which the kernel itself waits for (false serialization -> deadlock)
+    if ((st = finish_info(p, info))) return st;
+    if ((st = gather_impl(p, L, ldl))) return st;
+    CUDA_TRY(cudaEventRecord(p->ev3, p->stream));
+    CUDA_TRY(cudaStreamSynchronize(p->stream));
+  } else {
+    if ((st = gather_impl(p, L, ldl))) return st;
+    CUDA_TRY(cudaEventRecord(p->ev3, p->stream));
+    if ((st = finish_info(p, info))) return st;
+  }
   float tot = 0.f;
   CUDA_TRY(cudaEventElapsedTime(&tot, p->ev2, p->ev3));
   p->last_layout_s = tot * 1e-3 - p->last_factor_s;

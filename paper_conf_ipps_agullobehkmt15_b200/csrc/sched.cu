@@ -42,7 +42,8 @@ constexpr int kQStride = 32;           // ints between queue heads (separate 128
 // Multi-GPU: J_RECV copies row slab a of remote panel tile (i, j) from its owner b (peer
 // memory over NVLink) into this rank's cache slot.
 enum JobType : int16_t {
-  J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6, J_RECV = 7, J_INV = 8
+  J_UPD = 0, J_TRSM = 1, J_DIAG = 2, J_PANEL = 3, J_PUPD = 4, J_TS = 5, J_TU = 6, J_RECV = 7, J_INV = 8,
+  J_NOP = 9  // no work: a node that only publishes (host-class TRSM "inputs ready", hetero.cpp)
 };
 struct Job {
   int16_t type, i, j, k, a, b, c, pad;
@@ -828,6 +829,7 @@ struct SchedState {
   uint64_t* job_trace = nullptr;           // device, 4 per job (trace == 2)
   int* d_abort = nullptr;                  // device abort flag (d.abort_flag), written by sched_abort
   CUtensorMap dmap{};                      // Dinv workspace map (sched_set_dinv)
+  std::vector<std::pair<int, int>> host_tasks;  // TRSM_i_k run by the host CPU class (i, k)
   // re-bucketing with injected task priorities (sched_set_priorities)
   std::vector<int> h_node_paper, h_node_queue;
   size_t o_nq = 0, o_qbase = 0;
@@ -1274,6 +1276,9 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // inverse-form TRSM row slabs of each step and the D(b) nodes of each local POTRF
   // (build_inverses, after the task edges)
   std::vector<std::vector<int>> slab_nodes(N), dnodes(N);
+  // host CPU class: TRSMs at least cpu_d tiles below the diagonal (0 = off; single GPU)
+  const int cpu_d = dist ? 0 : opts->cpu_trsm_distance;
+  std::vector<int> host_in, host_out;
   std::vector<std::vector<std::vector<int>>> ts_nodes(N, std::vector<std::vector<int>>(nbb));
   const int nbb2 = nbb * nbb;
   auto gate_of = [&](int tid, int type, int i, int k) {
@@ -1348,6 +1353,22 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     }
     for (int i = k + 1; i < N && !blk; ++i) {
       if (!mine(i, k)) continue;
+      if (cpu_d > 0 && i - k >= cpu_d) {
+        // host CPU class (NEXT-3, the paper's TRSM-distance rule, L1019-1025): OUT (one no-op
+        // job) publishes "inputs final" to the host; IN (job-less) is fired by the watcher when
+        // the host has written L_ik back; IN is the task's last node (publishes the tile)
+        const int tid = (int)id_trsm(N, i, k);
+        const int outn = B.add_node(tid, T_TRSM, i, k);
+        B.add_job(outn, Job{J_NOP, (int16_t)i, (int16_t)k, (int16_t)k, 0, 0, 0, 0});
+        const int inn = B.add_node(-1, T_TRSM, i, k);
+        host_in.push_back(inn);
+        host_out.push_back(outn);
+        st->host_tasks.emplace_back(i, k);
+        first_node[tid] = outn;
+        last_node[tid] = inn;
+        slab_nodes[k].push_back(outn);  // waits for the inverses Dinv_k too
+        continue;
+      }
       const bool trsm_slab = trsm_slab_all && k < N - 1 - trsm_tail && i - k > trsm_dist;
       if (trsm_slab) {  // one left-looking row-slab job per BS rows
         const int tid = (int)id_trsm(N, i, k);
@@ -1518,6 +1539,17 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     for (int64_t k = 0; k < N; ++k) {
       publish[last_node[id_potrf(N, k)]] = (int)tile_index(k, k);
       for (int64_t i = k + 1; i < N; ++i) publish[last_node[id_trsm(N, i, k)]] = (int)tile_index(i, k);
+    }
+    // host CPU class: OUT publishes into the second half of the host-mapped flag array
+    // ("inputs of tile t final"); IN waits for the host's flag (peer_flags[1], watch order
+    // after every input-arrival entry)
+    const int64_t ntl = N * (N + 1) / 2;
+    for (size_t h = 0; h < host_in.size(); ++h) {
+      const int i = st->host_tasks[h].first, k = st->host_tasks[h].second;
+      const int t = (int)tile_index(i, k);
+      publish[host_out[h]] = (int)(ntl + t);
+      B.deps[host_in[h]] += 1;
+      watch.push_back(make_int4(host_in[h], 1, t, (int)(ntl + h)));
     }
   } else {
     // Same last-writer rule over the tiles an owned task touches: an owned tile's last
@@ -1748,6 +1780,7 @@ int sched_run(SchedState* st, const CUtensorMap& map, const StepParams& base, cu
 }
 
 int sched_workers(const SchedState* st) { return st ? st->workers : 0; }
+const std::vector<std::pair<int, int>>& sched_host_tasks(const SchedState* st) { return st->host_tasks; }
 const int* sched_progress(const SchedState* st) { return st ? st->d.done_nodes : nullptr; }
 void sched_abort(SchedState* st) {
   // from the host, while the kernel runs: a copy on a stream of its own

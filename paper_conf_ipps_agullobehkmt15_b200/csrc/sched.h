@@ -28,6 +28,8 @@ int sched_create_batch(SchedState** out, int64_t N, int64_t nb, int bs, int sms,
 // Dinv workspace of the inverse-form TRSM slabs: [N][nb/bs] bs x bs blocks (plan-owned) and
 // its TMA map (dims {bs, bs, N nb/bs}, box {16, bs, 1}, 128B swizzle)
 int sched_set_dinv(SchedState* st, double* dinv, const CUtensorMap& dmap);
+// the TRSM_i_k (i, k) this plan runs on the host CPU class (opts->cpu_trsm_distance)
+const std::vector<std::pair<int, int>>& sched_host_tasks(const SchedState* st);
 // injected static priorities per Algorithm 1 task (higher first; NEXT-4)
 int sched_set_priorities(SchedState* st, const double* prio, int64_t ntasks);
 // device pointers of the distributed plan, known after the IPC handle exchange

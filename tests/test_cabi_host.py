@@ -80,3 +80,28 @@ def test_owner_area_matches_oracle(chol):
         rmx, rper = obounds.owner_area(N, p, q, dict(zip(keys, T_thr)))
         assert abs(mx - rmx) <= 1e-12 * rmx
         assert all(abs(a - b) <= 1e-12 * max(b, 1e-30) for a, b in zip(per, rper))
+
+
+@pytest.mark.parametrize("nb,bs", [(96, 96), (192, 96), (960, 96), (128, 64), (64, 32)])
+def test_cpu_class_trsm_kernel_matches_oracle(nb, bs, chol):
+    """NEXT-3: the host CPU class's tile TRSM (inverse form, AVX-512 dot-product kernel)
+    against the oracle's substitution, and exact on the integer family (R19)."""
+    import numpy as np
+    import oracle
+    import spdgen
+    c = chol
+    M = spdgen.uniform_spd(2 * nb, nb + bs)
+    L = np.ascontiguousarray(np.linalg.cholesky(M[:nb, :nb]))
+    X = np.ascontiguousarray(M[nb:, :nb])
+    ref = oracle.tile_trsm(L, X)
+    got = X.copy()
+    c.chol_cpu_trsm(got, L, bs)
+    scale = np.max(np.abs(ref))
+    assert np.max(np.abs(got - ref) / np.maximum(np.abs(ref), 1e-6 * scale)) <= 1e-10
+    L0 = spdgen.integer_L0(2 * nb, 7)
+    A = spdgen.integer_spd(2 * nb, 7)
+    Xi = np.ascontiguousarray(A[nb:, :nb])
+    c.chol_cpu_trsm(Xi, np.ascontiguousarray(L0[:nb, :nb]), bs)
+    assert np.array_equal(Xi, L0[nb:, :nb])
+    with pytest.raises(c.CholError):
+        c.chol_cpu_trsm(X.copy(), L, 7)

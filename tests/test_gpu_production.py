@@ -144,3 +144,25 @@ def test_forced_decompositions_match_oracle(N, switch, monkeypatch):
     c = _lib()
     A, ref = _oracle(N * NB, N)
     _check(A, _factor_device(c, A), ref)
+
+
+@pytest.mark.parametrize("N,d", [(8, 3), (12, 6)])
+def test_host_cpu_class_trsms_match_oracle(N, d, monkeypatch):
+    """NEXT-3: the TRSMs at least d tiles below the diagonal run on the host CPU cores (the
+    paper's static rule); the factor still matches the oracle, device and streamed host
+    pointers, and the integer family stays exact."""
+    c = _lib()
+    A, ref = _oracle(N * NB, N + 100)
+    n = A.shape[0]
+    with c.Plan(n, NB, cpu_trsm_distance=d) as p:
+        dA = torch.from_numpy(A).cuda()
+        assert p.factor(dA) == 0
+        _check(A, dA.cpu().numpy(), ref)
+        L = np.full_like(A, np.nan)
+        assert c.chol_factor(p.h, A, n, L, n) == 0
+        _check(A, L, ref)
+        c.chol_generate(p.h, 4, 1)
+        assert c.chol_factor_inplace(p.h) == 0
+        out = torch.empty((n, n), dtype=torch.float64, device="cuda")
+        c.chol_gather(p.h, out, n)
+        assert np.array_equal(out.cpu().numpy(), spdgen.integer_L0(n, 4))

@@ -7,7 +7,7 @@ cd "$(dirname "$0")/.."
 mkdir -p variants/obj_$name
 CS=paper_conf_ipps_agullobehkmt15_b200/csrc
 F="-O3 -std=c++17 -gencode arch=compute_100a,code=sm_100a -lineinfo -Xcompiler -fPIC -Xcompiler -O2 --expt-relaxed-constexpr $@"
-for s in api.cu kernels.cu sched.cu solve.cu dag.cpp sim.cpp; do
+for s in api.cu kernels.cu sched.cu solve.cu dag.cpp sim.cpp hetero.cpp; do
   nvcc $F -c $CS/$s -o variants/obj_$name/${s%.*}.o &
 done
 wait

@@ -9,7 +9,7 @@ n = int(sys.argv[1]) if len(sys.argv) > 1 else 19200
 pol = int(sys.argv[2]) if len(sys.argv) > 2 else 0  # 0 = CP_PRIORITY
 binus = float(sys.argv[3]) if len(sys.argv) > 3 else 250.0
 nb = 960
-JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU", "RECV", "INV"]
+JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU", "RECV", "INV", "NOP"]
 with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=pol, trace=2) as p:
     for rep in range(2):
         c.chol_generate(p.h, 0, 0)
@@ -29,7 +29,7 @@ for lo, hi in zip(edges[:-1], edges[1:]):
     ov = np.clip(np.minimum(t1, hi) - np.maximum(t0, lo), 0, None)
     idle = W * (hi - lo) - ov.sum()
     tot_idle += idle
-    by = {JT[k]: round(float(ov[typ == k].sum() / (hi - lo)), 1) for k in range(9) if ov[typ == k].sum() > 0}
+    by = {JT[k]: round(float(ov[typ == k].sum() / (hi - lo)), 1) for k in range(10) if ov[typ == k].sum() > 0}
     rows.append((round(float((lo - T0) / 1e6), 2), round(float(idle / 1e6), 3), by))
 print(json.dumps({"n": n, "factor_ms": round(t_f * 1e3, 3), "workers": int(W), "idle_worker_ms": round(tot_idle / 1e6, 1),
                   "idle_frac": round(tot_idle / (W * (T1 - T0)), 4)}))

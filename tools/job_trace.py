@@ -7,7 +7,7 @@ import paper_conf_ipps_agullobehkmt15_b200 as c
 n = int(sys.argv[1]) if len(sys.argv) > 1 else 19200
 pol = int(sys.argv[2]) if len(sys.argv) > 2 else 0  # 0 = CP_PRIORITY
 nb = 960
-JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU", "RECV", "INV"]
+JT = ["UPD", "TRSM", "DIAG", "PANEL", "PUPD", "TS", "TU", "RECV", "INV", "NOP"]
 with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=pol, trace=2) as p:
     for rep in range(2):
         c.chol_generate(p.h, 0, 0)
