@@ -233,6 +233,10 @@ __device__ __forceinline__ int try_pop(const DevSched& d, bool latency_worker, i
 // completion bookkeeping off the compute warps; the producer walks the same job
 // sequence through a 2-deep shared-memory job ring and issues every TMA load,
 // running ahead into the next job as soon as ring stages free up.
+// idle scheduler warp: exponential __nanosleep backoff up to this many ns (A/B via -D)
+#ifndef CHOL_SCHED_BACKOFF_MAX
+#define CHOL_SCHED_BACKOFF_MAX 256
+#endif
 constexpr int kWsThreads = 384;
 constexpr int kProdWarp = 8, kSchedWarp = 9, kStoreWarp = 11;
 constexpr int kRegsCompute = 232, kRegsControl = 40;
@@ -777,7 +781,7 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
       break;
     }
     __nanosleep(backoff);
-    backoff = backoff < 256 ? backoff * 2 : 256;
+    backoff = backoff < CHOL_SCHED_BACKOFF_MAX ? backoff * 2 : CHOL_SCHED_BACKOFF_MAX;
   }
 }
 

@@ -5,6 +5,7 @@ with the right info under every policy."""
 import numpy as np
 import pytest
 
+import oracle
 import spdgen
 from oracle import dag as odag
 

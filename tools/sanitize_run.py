@@ -7,9 +7,14 @@ import torch
 import spdgen
 import paper_conf_ipps_agullobehkmt15_b200 as c
 
-for n, nb, pol in [(1920, 96, 1), (960, 96, 2), (3840, 960, 0)]:
+CASES = [(1920, 96, dict(policy=c.POLICY_CP_PRIORITY)), (960, 96, dict(policy=c.POLICY_STATIC)),
+         (3840, 960, dict(policy=c.POLICY_DYNAMIC)),  # all-TS/TU TRSMs, block DAG
+         (7680, 960, dict()),                         # slab TRSMs in inverse form + J_INV
+         (5760, 960, dict(cpu_trsm_distance=3))]      # host CPU class (OUT/NOP/IN, host flags)
+for n, nb, opts in CASES:
+    pol = opts.get("policy", 0)
     A = spdgen.uniform_spd(n, 5)
-    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=pol) as p:
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, **opts) as p:
         dA = torch.from_numpy(A.copy()).cuda()
         assert p.factor(dA) == 0
         torch.cuda.synchronize()
