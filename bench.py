@@ -55,6 +55,7 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-bounds", action="store_true")
+    ap.add_argument("--no-solve", action="store_true")
     ap.add_argument("--cpu-sample-n", type=int, default=7680)
     ap.add_argument("--grid", default="", help="process grid PxQ (default 1xN; SURVEY §8e prefers p <= q)")
     ap.add_argument("--logical-ranks", type=int, default=0)
@@ -536,6 +537,25 @@ def run_ours(args, ws, rank, local):
                                "factorization, final tiles of L streamed out as published, upper part zeroed "
                                "on the host; wall time"}
         del H
+    # the use of the factor: A X = B with the plan's factor, sweeps only
+    # (device time of the two triangular sweeps; B resident), one and 960 right-hand sides
+    if not args.no_solve and ex == c.EXEC_SCHEDULER:
+        import numpy as np
+        c.chol_generate(plan.h, args.seed, 0)
+        assert c.chol_factor_inplace(plan.h) == 0
+        sol = {}
+        for nrhs in (1, 960):
+            B = torch.ones((n, nrhs), dtype=torch.float64, device="cuda")
+            best = None
+            for _ in range(4):
+                c.chol_solve(plan.h, B, nrhs, nrhs)
+                sw = c.chol_last_solve_times(plan.h)[1]
+                best = sw if best is None else min(best, sw)
+            sol[str(nrhs)] = {"sweeps_ms": 1e3 * best, "fp64_tflops": 2.0 * n * n * nrhs / best / 1e12,
+                              "factor_read_GBps": 2 * (n * n / 2) * 8 / best / 1e9}
+            del B
+        line["solve"] = {"what": "chol_solve sweeps (L Y = B, L^T X = Y) with this factor, B on the device",
+                         "nrhs": sol}
     plan.close()
 
     # configs[1] beside the headline (parity cases and the r01 headline)

@@ -502,35 +502,39 @@ static cudaError_t solve_vec(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
 // the right-hand-side block with pitch 36, so every fragment load of a half-warp hits 16
 // distinct banks (forward: A[g][t] = L[8R+g][k+t]; backward, transposed: L[k+t][8R+g];
 // B[t][g] = Y[k+t][8C+g]).
-template <bool FWD>
+// RC = 64 (round 2, nrhs > 32): twice the columns per item, so each staged 96 x 96 matrix
+// feeds twice the DMMA work and the factor is streamed half as often (warp: 3 x 4 blocks,
+// pitch 68 keeps the half-warp fragment loads conflict-free: 68 mod 16 = 4 like 36).
+template <bool FWD, int RC>
 __global__ void __launch_bounds__(kSolveThreads, 1)
     k_sweep_mma(const double* tiles, int nb, int nblocks, const double* aux, double* W, int ldw, int nchunks,
                 int* flags, int* counter, int epoch) {
-  constexpr int SB = 96, RC = 32, LP = 100, YP = 36;
+  constexpr int SB = 96, LP = 100, YP = RC + 4, NI = RC / 16;
+  static_assert(RC == 32 || RC == 64, "chunk width");
   extern __shared__ __align__(16) double sm[];
   double* Lb[2] = {sm, sm + SB * LP};
   double* Ys = sm + 2 * SB * LP;
   int* s_item = reinterpret_cast<int*>(Ys + SB * YP);
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, g = lane >> 2, t = lane & 3;
-  const int R0 = 3 * (warp & 3), C0 = 2 * (warp >> 2);
+  const int R0 = 3 * (warp & 3), C0 = NI * (warp >> 2);
   const int total = nblocks * nchunks;
   const int64_t bsz = (int64_t)SB * SB;
   const double* inv = aux;
   const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
   // acc (+)= Op(Ls) Ys over k = 0..SB-1
-  auto block_mma = [&](const double* Ls, double (&acc)[3][2][2]) {
+  auto block_mma = [&](const double* Ls, double (&acc)[3][NI][2]) {
 #pragma unroll 4
     for (int k0 = 0; k0 < SB; k0 += 4) {
-      double a[3], bv[2];
+      double a[3], bv[NI];
 #pragma unroll
       for (int mi = 0; mi < 3; ++mi)
         a[mi] = FWD ? Ls[(8 * (R0 + mi) + g) * LP + k0 + t] : Ls[(k0 + t) * LP + 8 * (R0 + mi) + g];
 #pragma unroll
-      for (int ni = 0; ni < 2; ++ni) bv[ni] = Ys[(k0 + t) * YP + 8 * (C0 + ni) + g];
+      for (int ni = 0; ni < NI; ++ni) bv[ni] = Ys[(k0 + t) * YP + 8 * (C0 + ni) + g];
 #pragma unroll
       for (int mi = 0; mi < 3; ++mi)
 #pragma unroll
-        for (int ni = 0; ni < 2; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a[mi], bv[ni]);
+        for (int ni = 0; ni < NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a[mi], bv[ni]);
     }
   };
   while (true) {
@@ -557,11 +561,11 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
       cp_async_commit();
     };
     double* Wb = W + (int64_t)b * SB * ldw + ch * RC;
-    double rhs[3][2][2], acc[3][2][2];
+    double rhs[3][NI][2], acc[3][NI][2];
 #pragma unroll
     for (int mi = 0; mi < 3; ++mi)
 #pragma unroll
-      for (int ni = 0; ni < 2; ++ni) {
+      for (int ni = 0; ni < NI; ++ni) {
         const double2 v = __ldcg(reinterpret_cast<const double2*>(Wb + (int64_t)(8 * (R0 + mi) + g) * ldw +
                                                                   8 * (C0 + ni) + 2 * t));
         rhs[mi][ni][0] = v.x;
@@ -587,7 +591,7 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
 #pragma unroll
         for (int mi = 0; mi < 3; ++mi)
 #pragma unroll
-          for (int ni = 0; ni < 2; ++ni) {
+          for (int ni = 0; ni < NI; ++ni) {
             *reinterpret_cast<double2*>(Ys + (8 * (R0 + mi) + g) * YP + 8 * (C0 + ni) + 2 * t) =
                 make_double2(rhs[mi][ni][0] - acc[mi][ni][0], rhs[mi][ni][1] - acc[mi][ni][1]);
             acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
@@ -602,16 +606,16 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
       }
       __syncthreads();
       if (q == nold + 1) {  // acc = U - M y
-        double m[3][2][2];
+        double m[3][NI][2];
 #pragma unroll
         for (int mi = 0; mi < 3; ++mi)
 #pragma unroll
-          for (int ni = 0; ni < 2; ++ni) m[mi][ni][0] = m[mi][ni][1] = 0.0;
+          for (int ni = 0; ni < NI; ++ni) m[mi][ni][0] = m[mi][ni][1] = 0.0;
         block_mma(Lb[buf], m);
 #pragma unroll
         for (int mi = 0; mi < 3; ++mi)
 #pragma unroll
-          for (int ni = 0; ni < 2; ++ni) {
+          for (int ni = 0; ni < NI; ++ni) {
             acc[mi][ni][0] -= m[mi][ni][0];
             acc[mi][ni][1] -= m[mi][ni][1];
           }
@@ -623,7 +627,7 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
 #pragma unroll
     for (int mi = 0; mi < 3; ++mi)
 #pragma unroll
-      for (int ni = 0; ni < 2; ++ni)
+      for (int ni = 0; ni < NI; ++ni)
         __stcg(reinterpret_cast<double2*>(Wb + (int64_t)(8 * (R0 + mi) + g) * ldw + 8 * (C0 + ni) + 2 * t),
                make_double2(acc[mi][ni][0], acc[mi][ni][1]));
     __syncthreads();
@@ -632,13 +636,14 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
   }
 }
 
+template <int RC>
 static cudaError_t solve_mma(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   constexpr int SB = 96;
-  const int smem = (2 * SB * 100 + SB * 36) * 8 + 16, smem_inv = 2 * SB * kInvPitch * 8;
+  const int smem = (2 * SB * 100 + SB * (RC + 4)) * 8 + 16, smem_inv = 2 * SB * kInvPitch * 8;
   cudaError_t e;
   if ((e = cudaFuncSetAttribute(k_diag_aux<SB>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_inv))) return e;
-  if ((e = cudaFuncSetAttribute(k_sweep_mma<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
-  if ((e = cudaFuncSetAttribute(k_sweep_mma<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep_mma<true, RC>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep_mma<false, RC>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
   const int nblocks = (int)(a.n / SB);
   if (!a.inv_valid) {
     k_diag_aux<SB><<<std::min(nblocks, a.sms), kSolveThreads, smem_inv, s>>>(a.tiles, a.nb, nblocks, a.inv);
@@ -647,10 +652,10 @@ static cudaError_t solve_mma(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   const int total = nblocks * a.nchunks;
   const int grid = std::min(total, a.sms);
   if ((e = cudaMemsetAsync(a.ctl, 0, (2 + 2 * (size_t)total) * sizeof(int), s))) return e;
-  k_sweep_mma<true><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
-                                                       a.ctl + 2, a.ctl, 1);
-  k_sweep_mma<false><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
-                                                        a.ctl + 2 + total, a.ctl + 1, 1);
+  k_sweep_mma<true, RC><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                           a.ctl + 2, a.ctl, 1);
+  k_sweep_mma<false, RC><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                            a.ctl + 2 + total, a.ctl + 1, 1);
   *nlaunch += 2;
   return cudaGetLastError();
 }
@@ -694,7 +699,8 @@ cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   }
   // 32-column chunks at SB = 96 on DMMA (CHOL_SOLVE_SIMT=1: the SIMT sweeps; development switch)
   const char* esimt = getenv("CHOL_SOLVE_SIMT");
-  if (a.rc == 32 && a.sb == 96 && !(esimt && esimt[0] == '1')) return solve_mma(a, s, nlaunch);
+  if (a.rc == 64 && a.sb == 96) return solve_mma<64>(a, s, nlaunch);
+  if (a.rc == 32 && a.sb == 96 && !(esimt && esimt[0] == '1')) return solve_mma<32>(a, s, nlaunch);
   const bool narrow = a.rc == 8;
   switch (a.sb) {
     case 96: return narrow ? solve_sb<96, 8>(a, s, nlaunch) : solve_sb<96, 32>(a, s, nlaunch);
