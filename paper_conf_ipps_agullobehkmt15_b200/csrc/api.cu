@@ -316,7 +316,7 @@ extern "C" int chol_plan_dist(int64_t n, int64_t nb, int nranks, int rank, const
   if (o) opts = *o;
   if (opts.policy < 0 || opts.policy > 2 || opts.executor != CHOL_EXEC_SCHEDULER || opts.trsm_pin_distance < 0 ||
       opts.latency_workers < 0 || opts.workers < 0 || opts.grid_p < 0 || opts.grid_q < 0 || opts.trace < 0 ||
-      opts.trace > 2)
+      opts.trace > 2 || opts.cpu_trsm_distance != 0 || opts.cpu_threads < 0)  // host class: single GPU only
     return -6;
   if (opts.grid_p == 0 && opts.grid_q == 0) {
     opts.grid_p = 1;

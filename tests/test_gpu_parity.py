@@ -227,6 +227,13 @@ def test_argument_errors():
     with pytest.raises(c.CholError) as e:
         c.chol_plan_ex(96, 32, 1, policy=7)
     assert e.value.status == -6
+    for bad in (dict(cpu_trsm_distance=-1), dict(cpu_threads=-2), dict(cpu_trsm_distance=2, executor=c.EXEC_HOST)):
+        with pytest.raises(c.CholError) as e:
+            c.chol_plan_ex(960, 96, 1, **bad)
+        assert e.value.status == -6
+    with pytest.raises(c.CholError) as e:  # the host CPU class is single-GPU only
+        c.chol_plan_dist(960, 96, 2, 0, cpu_trsm_distance=2)
+    assert e.value.status == -6
     with c.Plan(96, 32) as p:
         with pytest.raises(c.CholError) as e:
             c.chol_factor(p.h, 0, 96, 0, 96)
