@@ -172,7 +172,7 @@ def run_reference(args, ws, rank):
     import oracle
     import spdgen
     n_w = workload_n(args, ws)
-    n_s = min(n_w, 3840)
+    n_s = min(n_w, 7680)  # 8 x 8 tiles: enough tasks per step for the oracle's OpenMP fork-join
     A = spdgen.uniform_spd(n_s, args.seed)
     times = []
     for it in range(args.warmup + args.steps):
