@@ -1256,12 +1256,13 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   // the whole SYRK.  A larger block region costs efficiency (K = BS TRSM updates, more
   // nodes): measured best m (tools/tail_sweep.py, nb = 960) is 4 for N = 4..10 and 2 for
   // N = 12..24 (n=3840 3.76 -> 2.82 ms, n=9600 13.07 -> 12.18, n=19200 71.82 -> 71.57).
-  // Single GPU only.  CHOL_BLOCK_TAIL=m overrides (m steps).
+  // Distributed plans too (round 2): a remote panel tile enters the blocked region through
+  // its RECV node, which every block node reading it waits for.  CHOL_BLOCK_TAIL=m overrides
+  // (m steps).
   const char* ebt = getenv("CHOL_BLOCK_TAIL");
   // round-2 sweep (profiles/r02/block_tail_sweep_r02.txt): m = 4 for N <= 6, 3 for N = 7..10
   // (n=9600 11.78 -> 11.25 ms, n=7680 8.11 -> 7.93), 2 above
   int block_tail = ebt ? atoi(ebt) : (N <= 6 ? 4 : N <= 10 ? 3 : 2);
-  if (dist) block_tail = 0;
   const int k0 = (int)N - std::max(0, std::min(block_tail, (int)N));
   // blocked-region TRSM: per-slab TS/TU chains (0) or one left-looking slab job per
   // slab node (1).  CHOL_TAIL_TRSM.
@@ -1285,6 +1286,26 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
   std::vector<int> host_in, host_out;
   std::vector<std::vector<std::vector<int>>> ts_nodes(N, std::vector<std::vector<int>>(nbb));
   const int nbb2 = nbb * nbb;
+  std::vector<int4> watch;  // multi-GPU: {RECV node, owner, tile, step}
+  std::vector<int> recv_node((size_t)(N * (N + 1) / 2), -1);  // multi-GPU: RECV node of a remote tile
+  // multi-GPU: this rank's RECV node for remote panel tile (i, j), created on first use (its
+  // jobs copy the tile's row slabs from the owner's store; the watcher fires it when the
+  // owner publishes the tile)
+  auto recv_of = [&](int64_t i, int64_t j) -> int {
+    const int64_t t = tile_index(i, j);
+    if (recv_node[t] < 0) {
+      const int owner = tile_owner((int)i, (int)j, dist->p, dist->q);
+      const int rn = B.add_node(-1, -1, (int)i, (int)j);
+      for (int sl = 0; sl < nbb; ++sl)
+        B.add_job(rn, Job{J_RECV, (int16_t)i, (int16_t)j, 0, (int16_t)sl, (int16_t)owner, 0, 0});
+      B.deps[rn] += 1;  // fired by the watcher (remote readiness)
+      recv_node[t] = rn;
+      watch.push_back(make_int4(rn, owner, (int)t, (int)j));
+    }
+    return recv_node[t];
+  };
+  // the node that makes block (r, c) of L_kk final: local D / P node, or the RECV of L_kk
+  auto lkk_block = [&](int k, int pid, int r, int c) { return mine(k, k) ? tfin[pid][r * nbb + c] : recv_of(k, k); };
   auto gate_of = [&](int tid, int type, int i, int k) {
     // job-less node in front of a blocked task's entry nodes: the target of task-level
     // dependencies (streamed tile arrival at k = 0)
@@ -1314,6 +1335,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       // blocked TRSM_i_k: per row slab sl, TS(c, sl) / TU(c, sl, c') single-job nodes
       // (or one slab job per node), edges from the POTRF_k blocks each one reads:
       // TS(c, sl) <- L_kk[c,c] = D(c); TU(c, sl, c') <- L_kk[c',c] = P(c',c)
+      if (!mine(i, k)) continue;
       const int tid = (int)id_trsm(N, i, k);
       tentry[tid].assign(nbb2, -1);
       tfin[tid].assign(nbb2, -1);
@@ -1323,7 +1345,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
         if (tail_trsm_slab) {
           const int sn = B.add_node(tid, T_TRSM, i, k);
           B.add_job(sn, Job{J_TRSM, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)sl, 0, 0, 0});
-          B.edge(tfin[pid][(nbb - 1) * nbb + nbb - 1], sn);  // D(nbb-1): all of L_kk
+          B.edge(lkk_block(k, pid, nbb - 1, nbb - 1), sn);  // D(nbb-1): all of L_kk
           slab_nodes[k].push_back(sn);
           for (int c = 0; c < nbb; ++c) tentry[tid][sl * nbb + c] = tfin[tid][sl * nbb + c] = sn;
           tslab[tid][sl] = sn;
@@ -1335,7 +1357,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
           const int ts = B.add_node(tid, T_TRSM, i, k);
           B.add_job(ts, Job{J_TS, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, 0, 0});
           ts_nodes[k][cb].push_back(ts);
-          B.edge(tfin[pid][cb * nbb + cb], ts);
+          B.edge(lkk_block(k, pid, cb, cb), ts);
           if (cb > 0) B.edge(lastTU[cb], ts);
           else tentry[tid][sl * nbb] = ts;
           tfin[tid][sl * nbb + cb] = ts;
@@ -1343,7 +1365,7 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
             const int tu = B.add_node(tid, T_TRSM, i, k);
             B.add_job(tu, Job{J_TU, (int16_t)i, (int16_t)k, (int16_t)k, (int16_t)cb, (int16_t)sl, (int16_t)c2, 0});
             B.edge(ts, tu);
-            B.edge(tfin[pid][c2 * nbb + cb], tu);
+            B.edge(lkk_block(k, pid, c2, cb), tu);
             if (lastTU[c2] >= 0) B.edge(lastTU[c2], tu);
             else tentry[tid][sl * nbb + c2] = tu;
             lastTU[c2] = tu;
@@ -1420,17 +1442,20 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
     for (int j = k + 1; j < N && blk; ++j) {
       // blocked SYRK_j_k / GEMM_i_j_k: one node per output block, K = nb
       const int sid = (int)id_syrk(N, j, k);
-      tentry[sid].assign(nbb2, -1);
-      for (int bm = 0; bm < nbb; ++bm)
-        for (int bn = 0; bn <= bm; ++bn) {
-          const int n = B.add_node(sid, T_SYRK, j, k);
-          B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
-          tentry[sid][bm * nbb + bn] = n;
-        }
-      tfin[sid] = tentry[sid];
-      if (k == 0) gate_of(sid, T_SYRK, j, k);
+      if (mine(j, j)) {
+        tentry[sid].assign(nbb2, -1);
+        for (int bm = 0; bm < nbb; ++bm)
+          for (int bn = 0; bn <= bm; ++bn) {
+            const int n = B.add_node(sid, T_SYRK, j, k);
+            B.add_job(n, Job{J_UPD, (int16_t)j, (int16_t)j, (int16_t)k, (int16_t)bm, (int16_t)bn, 0, 0});
+            tentry[sid][bm * nbb + bn] = n;
+          }
+        tfin[sid] = tentry[sid];
+        if (k == 0) gate_of(sid, T_SYRK, j, k);
+      }
 
       for (int i = j + 1; i < N; ++i) {
+        if (!mine(i, j)) continue;
         const int gid = (int)id_gemm(N, i, j, k);
         tentry[gid].assign(nbb2, -1);
         for (int bm = 0; bm < nbb; ++bm)
@@ -1466,54 +1491,71 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
 
   // ---- task edges: direct data dependencies of Algorithm 1 (dag.cpp, L213-220),
   // mapped onto the nodes (POTRF_k enters at its first inner node, leaves at its last).
-  std::vector<int4> watch;  // multi-GPU: {RECV node, owner, tile, step}
-  std::vector<int> recv_node((size_t)(N * (N + 1) / 2), -1);  // multi-GPU: RECV node of a remote tile
-  if (!dist) {
-    std::vector<std::pair<int64_t, int64_t>> E;
-    std::vector<int> type_of;
-    build_task_dag(N, E, type_of);
-    // tile written by a task (i, j) -- Algorithm 1 visit order of taskid.h
-    std::vector<int2> wtile(n_tasks(N));
-    for (int64_t k = 0; k < N; ++k) {
-      wtile[id_potrf(N, k)] = make_int2((int)k, (int)k);
-      for (int64_t i = k + 1; i < N; ++i) wtile[id_trsm(N, i, k)] = make_int2((int)i, (int)k);
-      for (int64_t j = k + 1; j < N; ++j) {
-        wtile[id_syrk(N, j, k)] = make_int2((int)j, (int)j);
-        for (int64_t i = j + 1; i < N; ++i) wtile[id_gemm(N, i, j, k)] = make_int2((int)i, (int)j);
-      }
+  std::vector<std::pair<int64_t, int64_t>> E;
+  std::vector<int> type_of;
+  build_task_dag(N, E, type_of);
+  // tile written by a task (i, j) -- Algorithm 1 visit order of taskid.h
+  std::vector<int2> wtile(n_tasks(N));
+  for (int64_t k = 0; k < N; ++k) {
+    wtile[id_potrf(N, k)] = make_int2((int)k, (int)k);
+    for (int64_t i = k + 1; i < N; ++i) wtile[id_trsm(N, i, k)] = make_int2((int)i, (int)k);
+    for (int64_t j = k + 1; j < N; ++j) {
+      wtile[id_syrk(N, j, k)] = make_int2((int)j, (int)j);
+      for (int64_t i = j + 1; i < N; ++i) wtile[id_gemm(N, i, j, k)] = make_int2((int)i, (int)j);
     }
-    for (auto& e : E) {
-      const int64_t a = e.first, b = e.second;
-      if (tentry[b].empty()) {  // task-level consumer (k < k0)
-        B.edge(last_node[a], first_node[b]);
-        continue;
-      }
-      const int2 tb = wtile[b];
-      const bool diag = tb.x == tb.y;
-      if (tentry[a].empty()) {  // task-level producer of a blocked consumer: every entry waits
+  }
+  // Multi-GPU: a rank builds the edges into the tasks it owns; a producer on another rank
+  // (always the task that made a panel tile L_kk / L_ik final) is reached through this
+  // rank's RECV node for that tile, which every node of the consumer waits for.
+  auto owned = [&](int64_t task) { return mine(wtile[task].x, wtile[task].y); };
+  for (auto& e : E) {
+    const int64_t a = e.first, b = e.second;
+    if (dist && !owned(b)) continue;
+    if (dist && !owned(a)) {
+      const int rn = recv_of(wtile[a].x, wtile[a].y);
+      if (tentry[b].empty()) {
+        B.edge(rn, first_node[b]);
+      } else if (!(type_of[a] == T_POTRF && type_of[b] == T_TRSM)) {  // TRSM blocks: made with the nodes
         std::vector<int> seen;
         for (int x : tentry[b])
           if (x >= 0 && std::find(seen.begin(), seen.end(), x) == seen.end()) {
-            B.edge(last_node[a], x);
+            B.edge(rn, x);
             seen.push_back(x);
           }
-        continue;
       }
-      if (type_of[a] == T_POTRF && type_of[b] == T_TRSM) continue;  // block edges made with the TRSM nodes
-      for (int bm = 0; bm < nbb; ++bm)
-        for (int bn = 0; bn < nbb; ++bn) {
-          if (diag && bn > bm) continue;  // lower blocks of a diagonal tile
-          const int x = tentry[b][bm * nbb + bn];
-          if (x < 0) continue;
-          if (type_of[a] == T_TRSM) {  // L_ik read by SYRK / GEMM: row slabs bm and / or bn
-            const int pi = wtile[a].x;
-            if (pi == tb.x) B.edge(tslab[a][bm], x);
-            if (pi == tb.y && !(pi == tb.x && bm == bn)) B.edge(tslab[a][bn], x);
-          } else {  // the same tile, block by block (SYRK->POTRF, SYRK->SYRK, GEMM->GEMM, GEMM->TRSM)
-            B.edge(tfin[a][bm * nbb + bn], x);
-          }
-        }
+      continue;
     }
+    if (tentry[b].empty()) {  // task-level consumer (k < k0)
+      B.edge(last_node[a], first_node[b]);
+      continue;
+    }
+    const int2 tb = wtile[b];
+    const bool diag = tb.x == tb.y;
+    if (tentry[a].empty()) {  // task-level producer of a blocked consumer: every entry waits
+      std::vector<int> seen;
+      for (int x : tentry[b])
+        if (x >= 0 && std::find(seen.begin(), seen.end(), x) == seen.end()) {
+          B.edge(last_node[a], x);
+          seen.push_back(x);
+        }
+      continue;
+    }
+    if (type_of[a] == T_POTRF && type_of[b] == T_TRSM) continue;  // block edges made with the TRSM nodes
+    for (int bm = 0; bm < nbb; ++bm)
+      for (int bn = 0; bn < nbb; ++bn) {
+        if (diag && bn > bm) continue;  // lower blocks of a diagonal tile
+        const int x = tentry[b][bm * nbb + bn];
+        if (x < 0) continue;
+        if (type_of[a] == T_TRSM) {  // L_ik read by SYRK / GEMM: row slabs bm and / or bn
+          const int pi = wtile[a].x;
+          if (pi == tb.x) B.edge(tslab[a][bm], x);
+          if (pi == tb.y && !(pi == tb.x && bm == bn)) B.edge(tslab[a][bn], x);
+        } else {  // the same tile, block by block (SYRK->POTRF, SYRK->SYRK, GEMM->GEMM, GEMM->TRSM)
+          B.edge(tfin[a][bm * nbb + bn], x);
+        }
+      }
+  }
+  if (!dist) {
     // Streamed input (chol_factor from host memory): the first task touching a tile
     // waits for the tile's arrival flag (the copy engine writes it after the tile).
     // Tiles arrive in row-major tile order (row i: tiles (i,0..i)); the watch list
@@ -1556,48 +1598,6 @@ int sched_create(SchedState** out, int64_t N, int64_t nb, int bs, int sms, const
       watch.push_back(make_int4(host_in[h], 1, t, (int)(ntl + h)));
     }
   } else {
-    // Same last-writer rule over the tiles an owned task touches: an owned tile's last
-    // writer is an owned task; a remote tile (always a final panel tile L_kk / L_ik) is
-    // reached through this rank's RECV node for it, fired by the watcher when the owner
-    // publishes the tile.
-    std::vector<int64_t> last_writer((size_t)(N * (N + 1) / 2), -1);
-    std::vector<int> preds;
-    auto visit = [&](int64_t task, std::initializer_list<std::pair<int64_t, int64_t>> touched, int64_t wi,
-                     int64_t wj) {
-      const int64_t wt = tile_index(wi, wj);
-      if (mine(wi, wj)) {
-        preds.clear();
-        for (auto& ij : touched) {
-          const int64_t t = tile_index(ij.first, ij.second);
-          int pn = -1;
-          if (mine(ij.first, ij.second)) {
-            if (last_writer[t] >= 0) pn = last_node[last_writer[t]];
-          } else {
-            if (recv_node[t] < 0) {
-              const int owner = tile_owner(ij.first, ij.second, dist->p, dist->q);
-              const int rn = B.add_node(-1, -1, (int)ij.first, (int)ij.second);
-              for (int sl = 0; sl < nbb; ++sl)
-                B.add_job(rn, Job{J_RECV, (int16_t)ij.first, (int16_t)ij.second, 0, (int16_t)sl, (int16_t)owner, 0, 0});
-              B.deps[rn] += 1;  // fired by the watcher (remote readiness)
-              recv_node[t] = rn;
-              watch.push_back(make_int4(rn, owner, (int)t, (int)ij.second));
-            }
-            pn = recv_node[t];
-          }
-          if (pn >= 0 && std::find(preds.begin(), preds.end(), pn) == preds.end()) preds.push_back(pn);
-        }
-        for (int pn : preds) B.edge(pn, first_node[task]);
-      }
-      last_writer[wt] = task;
-    };
-    for (int64_t k = 0; k < N; ++k) {
-      visit(id_potrf(N, k), {{k, k}}, k, k);
-      for (int64_t i = k + 1; i < N; ++i) visit(id_trsm(N, i, k), {{k, k}, {i, k}}, i, k);
-      for (int64_t j = k + 1; j < N; ++j) {
-        visit(id_syrk(N, j, k), {{j, k}, {j, j}}, j, j);
-        for (int64_t i = j + 1; i < N; ++i) visit(id_gemm(N, i, j, k), {{i, k}, {j, k}, {i, j}}, i, j);
-      }
-    }
     std::stable_sort(watch.begin(), watch.end(), [](const int4& a, const int4& b) { return a.w < b.w; });
     // panel tiles this rank finalises are published (their final node)
     publish.assign(B.deps.size(), -1);
