@@ -1134,6 +1134,7 @@ extern "C" int chol_set_task_priorities(chol_plan_t p, const double* prio, int64
   }
   if (!p->sched) return -8;
   cudaSetDevice(p->device);
+  CUDA_TRY(cudaStreamSynchronize(p->stream));  // no factorization in flight reads the tables
   return sched_set_priorities(p->sched, prio, ntasks);
 }
 
