@@ -89,6 +89,24 @@ struct DevSched {
 };
 
 // ------------------------------------------------------------------ device queue ops
+// -DCHOL_HOPS: the scheduler warp of every CTA accumulates clock64 sections of the hand-off
+// path (a worker whose completion readies a single-job successor runs it next): [0] jdone
+// seen -> node counter decremented, [1] -> successors decremented / taker chosen, [2] ->
+// other successors pushed, [3] -> node counted / trace, [4] -> descriptor written (jfull),
+// [5] hand-off count, [6] compute end (globaltimer) -> jdone seen (ns).
+#ifdef CHOL_HOPS
+__device__ unsigned long long g_hop[8];
+__device__ long long g_hopt[1024][4];  // per CTA: stamps inside node_done_warp
+#define HOP_T(v) const long long v = clock64()
+#define HOP_MARK(i) \
+  if (lane == 0) g_hopt[blockIdx.x][i] = clock64()
+#define HOP_ADD(i, v) \
+  if (lane == 0) atomicAdd(&g_hop[i], (unsigned long long)(v))
+#else
+#define HOP_T(v)
+#define HOP_MARK(i)
+#define HOP_ADD(i, v)
+#endif
 __device__ __forceinline__ int ld_volatile(const int* p) { return *reinterpret_cast<const volatile int*>(p); }
 
 // A ready node is enqueued ONCE (one queue item per node); workers then claim its jobs
@@ -118,17 +136,13 @@ __device__ __forceinline__ void push_node(const DevSched& d, int node) {
 // queue round trips on chains of single-job nodes (the POTRF block DAG's critical path
 // D(b) -> P(b+1,b) -> U(b+1,b+1,b) -> D(b+1)).  Returns that node or -1 (warp-uniform).
 template <int Depth>
-__device__ int node_done_warp(const DevSched& d, int node, int lane, bool can_take) {
-  __threadfence();
-  if (lane == 0 && d.node_publish) {
-    const int pt = d.node_publish[node];
-    if (pt >= 0) {  // panel tile final: release it to every rank (system scope, NVLink)
-      __threadfence_system();
-      asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(d.my_flags + pt), "r"(d.epoch) : "memory");
-    }
-  }
+__device__ int node_done_warp(const DevSched& d, int node, int lane, bool can_take);
+
+// Release the successors succ[beg, end) of a completed node, one lane per edge (see
+// node_done_warp); returns the hand-off node or -1 (warp-uniform).
+template <int Depth>
+__device__ int release_range(const DevSched& d, int beg, int end, int lane, bool can_take) {
   int take = -1;
-  const int beg = d.succ_off[node], end = d.succ_off[node + 1];
   for (int e0 = beg; e0 < end; e0 += 32) {
     const int e = e0 + lane;
     int s = -1, cnt = -1;
@@ -140,10 +154,15 @@ __device__ int node_done_warp(const DevSched& d, int node, int lane, bool can_ta
     const unsigned ms = __ballot_sync(0xffffffffu, can_take && take < 0 && cnt == 1);
     const int taker = ms ? __ffs(ms) - 1 : -1;
     if (taker >= 0) {
+      HOP_MARK(0);
       take = __shfl_sync(0xffffffffu, s, taker);
       if (lane == taker && d.job_trace) d.job_trace[4 * (size_t)d.node_job_begin[s] + 3] = globaltimer_ns() - *d.tr_base;
     }
     if (cnt > 0 && lane != taker) push_node(d, s);
+    if (taker >= 0) {
+      __syncwarp();
+      HOP_MARK(1);
+    }
     if constexpr (Depth > 0) {
       unsigned m = __ballot_sync(0xffffffffu, join);
       while (m) {
@@ -154,11 +173,35 @@ __device__ int node_done_warp(const DevSched& d, int node, int lane, bool can_ta
       }
     }
   }
+  return take;
+}
+
+// The node's tile is final: release it to every rank (system scope, NVLink) / the host.
+__device__ __forceinline__ void publish_node(const DevSched& d, int node, int lane) {
+  if (lane == 0 && d.node_publish) {
+    const int pt = d.node_publish[node];
+    if (pt >= 0) {
+      __threadfence_system();
+      asm volatile("st.release.sys.global.u32 [%0], %1;" ::"l"(d.my_flags + pt), "r"(d.epoch) : "memory");
+    }
+  }
+}
+
+__device__ __forceinline__ void count_node_done(const DevSched& d, int lane) {
   if (lane == 0 && atomicAdd(d.done_nodes, 1) == d.total_nodes - 1) {
     __threadfence();
     atomicExch(d.finished, 1);
   }
   __syncwarp();
+}
+
+template <int Depth>
+__device__ int node_done_warp(const DevSched& d, int node, int lane, bool can_take) {
+  __threadfence();
+  publish_node(d, node, lane);
+  const int take = release_range<Depth>(d, d.succ_off[node], d.succ_off[node + 1], lane, can_take);
+  count_node_done(d, lane);
+  HOP_MARK(2);
   return take;
 }
 
@@ -540,6 +583,18 @@ __device__ __forceinline__ long long phase_clock() { return clock64(); }
 #define PHASE_ADD(i, v)
 #endif
 void sched_phase_dump() {
+#ifdef CHOL_HOPS
+  {
+    unsigned long long h[8];
+    cudaMemcpyFromSymbol(h, g_hop, sizeof(h));
+    const double nh = h[5] ? (double)h[5] : 1.0;
+    fprintf(stderr, "CHOL_HOPS handoffs %llu  cycles: node_left %.0f  succ %.0f  pushes %.0f  count/trace %.0f  "
+            "claim %.0f  (compute end -> jdone seen %.0f ns)\n", h[5], h[0] / nh, h[1] / nh, h[2] / nh, h[3] / nh,
+            h[4] / nh, h[6] / nh);
+    const unsigned long long z[8] = {};
+    cudaMemcpyToSymbol(g_hop, z, sizeof(z));
+  }
+#endif
 #ifdef CHOL_PHASES
   unsigned long long h[8];
   cudaMemcpyFromSymbol(h, g_phase, sizeof(h));
@@ -699,18 +754,10 @@ __device__ void compute_loop(Ctx<BS>& c, const DevSched& d, int* info) {
   }
 }
 
-// ---- scheduler warp (all lanes): job counter, node completion, trace
-__device__ __forceinline__ int complete_job(const DevSched& d, const StepParams& sp, int job, uint64_t t0_abs,
-                                            uint64_t t1_abs, int lane, bool can_take) {
-  const int node = d.job_node[job];
-  int last = 0;
-  if (lane == 0) {
-    __threadfence();  // the compute warps' stores (acquired through jdone) before the counters
-    last = atomicSub(&d.node_left[node], 1) == 1;
-  }
-  const int take = __shfl_sync(0xffffffffu, last, 0) ? node_done_warp<1>(d, node, lane, can_take) : -1;
-  // trace records after the release: every job of a task updates the same two words,
-  // and that contention must not delay the successors
+// Trace records of a completed job (after the releases: every job of a task updates the
+// same two words, and that contention must not delay the successors).
+__device__ __forceinline__ void trace_job(const DevSched& d, const StepParams& sp, int node, int job, uint64_t t0_abs,
+                                          uint64_t t1_abs, int lane) {
   if (lane == 0 && sp.tr_t0 && d.node_paper[node] >= 0) {
     const uint64_t base = *sp.tr_base;
     const uint64_t t0 = t0_abs - base, t_end = t1_abs - base;
@@ -723,6 +770,118 @@ __device__ __forceinline__ int complete_job(const DevSched& d, const StepParams&
       d.job_trace[4 * (size_t)job + 2] = ((uint64_t)blockIdx.x << 32) | smid();
     }
   }
+}
+
+// ---- hand-off fast path.  While a job runs alone on its worker, the scheduler warp
+// preloads the successor list of the job's node into shared memory: successor ids, their
+// job counts and, for single-job successors, the job descriptor (all of these tables are
+// constant during a launch).  At completion the successors are released with one round of
+// atomics and a ready single-job successor is written into the job ring straight from the
+// preloaded descriptor, before the other successors are queued and the node is counted --
+// none of the dependent global loads of the generic path (node, successor list, job count,
+// job begin, descriptor) are left between the end of one job and the start of the next on
+// a chain of single-job nodes (the POTRF block DAG's D(b) -> P(b+1,b) -> D(b+1)).
+struct SuccPre {
+  int4 sjob[32];                   // Job of single-job successor l (raw 16 bytes)
+  int succ[32], scnt[32], sbeg[32];
+  int job, node, jc, ns;           // preloaded job (-1: none), its node, job count, successors
+};
+static_assert(sizeof(Job) == 16, "Job is loaded as one int4");
+
+#ifndef CHOL_PRE_MODE
+#define CHOL_PRE_MODE 2  // development switch: 0 no preload, 1 after claims only, 2 also while idle
+#endif
+__device__ __forceinline__ void fence_acq_rel_gpu() { asm volatile("fence.acq_rel.gpu;" ::: "memory"); }
+
+__device__ void preload_succ(const DevSched& d, SuccPre* P, int job, int lane) {
+  const int node = __ldg(d.job_node + job);
+  const int beg = __ldg(d.succ_off + node), ns = __ldg(d.succ_off + node + 1) - beg;
+  int sc = 1;
+  if (lane < ns) {
+    const int sn = __ldg(d.succ + beg + lane);
+    sc = __ldg(d.node_job_count + sn);
+    const int sb = __ldg(d.node_job_begin + sn);
+    P->succ[lane] = sn;
+    P->scnt[lane] = sc;
+    P->sbeg[lane] = sb;
+    if (sc == 1) P->sjob[lane] = __ldg(reinterpret_cast<const int4*>(d.jobs) + sb);
+  }
+  // a node with more than 32 successors or a job-less successor keeps the generic path
+  const bool ok = ns <= 32 && __all_sync(0xffffffffu, sc > 0);
+  if (lane == 0) {
+    P->node = node;
+    P->jc = __ldg(d.node_job_count + node);
+    P->ns = ns;
+    P->job = ok ? job : -2 - job;
+  }
+  __syncwarp();
+}
+
+// Completion of the preloaded job.  Returns the job written into the ring slot (slot /
+// jfull_e: the next free entry) or -1.  Same releases and counts as complete_job +
+// node_done_warp (the preloaded nodes have no job-less successor), hand-off first.
+__device__ int complete_job_pre(const DevSched& d, const StepParams& sp, const SuccPre* P, uint64_t t0_abs,
+                                uint64_t t1_abs, int lane, bool can_take, int4* slot, uint64_t* jfull_e) {
+  const int node = P->node, job = P->job;
+  int last = 1;
+  if (P->jc != 1) {  // several jobs: the node is done when its counter runs out
+    if (lane == 0) {
+      __threadfence();  // the compute warps' stores (acquired through jdone) before the counter
+      last = atomicSub(&d.node_left[node], 1) == 1;
+    }
+    last = __shfl_sync(0xffffffffu, last, 0);
+  }
+  HOP_MARK(3);
+  int issued = -1;
+  if (last) {
+    fence_acq_rel_gpu();  // every job of the node (this worker's stores, the other jobs' releases) before the edges
+    const int inf = ld_volatile(sp.info);
+    const int ns = P->ns;
+    int sn = -1, cnt = -1;
+    if (lane < ns) {
+      sn = P->succ[lane];
+      if (atomicSub(&d.node_deps[sn], 1) == 1) cnt = P->scnt[lane];
+    }
+    const unsigned ms = __ballot_sync(0xffffffffu, can_take && cnt == 1);
+    const int taker = ms ? __ffs(ms) - 1 : -1;
+    if (taker >= 0) {
+      HOP_MARK(0);
+      if (lane == taker) {
+        fence_acq_rel_gpu();  // acquire: the other predecessors' releases, before the job's loads
+        const int4 raw = P->sjob[lane];
+        const Job jb = *reinterpret_cast<const Job*>(&raw);
+        const int jid = P->sbeg[lane];
+        write_desc(slot, jid, jb, inf != INT_MAX && jb.k >= (inf - 1) / sp.nb);
+        mbar_arrive(jfull_e);
+        if (d.job_trace) d.job_trace[4 * (size_t)jid + 3] = globaltimer_ns() - *d.tr_base;
+      }
+      issued = P->sbeg[taker];
+    }
+    __syncwarp();
+    HOP_MARK(1);
+    publish_node(d, node, lane);
+    if (cnt > 0 && lane != taker) push_node(d, sn);
+    count_node_done(d, lane);
+    HOP_MARK(2);
+  }
+  trace_job(d, sp, node, job, t0_abs, t1_abs, lane);
+  return issued;
+}
+
+// ---- scheduler warp (all lanes): job counter, node completion, trace
+__device__ __forceinline__ int complete_job(const DevSched& d, const StepParams& sp, int job, uint64_t t0_abs,
+                                            uint64_t t1_abs, int lane, bool can_take) {
+  const int node = d.job_node[job];
+  int last = 0;
+  if (lane == 0) {
+    __threadfence();  // the compute warps' stores (acquired through jdone) before the counters
+    last = atomicSub(&d.node_left[node], 1) == 1;
+  }
+  HOP_MARK(3);
+  const int take = __shfl_sync(0xffffffffu, last, 0) ? node_done_warp<1>(d, node, lane, can_take) : -1;
+  // trace records after the release: every job of a task updates the same two words,
+  // and that contention must not delay the successors
+  trace_job(d, sp, node, job, t0_abs, t1_abs, lane);
   return take;
 }
 template <int BS>
@@ -732,16 +891,63 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
   int pending[2] = {-1, -1};
   int take = -1;  // single-job successor handed to this worker by its own completion
   unsigned backoff = 32;
+  SuccPre* P = reinterpret_cast<SuccPre*>(Ctx<BS>::pre());
+  if (lane == 0) P->job = -1;
+  __syncwarp();
+#ifdef CHOL_HOPS
+  long long h_claim_from = 0;
+#endif
   while (true) {
     // 1. retire finished jobs in order
     while (q_done < q_issue) {
       const int e = q_done & 1;
       if (!mbar_try_wait(smem_u32(&c.jdone()[e]), (q_done >> 1) & 1)) break;
+      HOP_T(h_seen);
+#ifdef CHOL_HOPS
+      const unsigned long long h_gt = globaltimer_ns();
+#endif
       const int4 tt = c.jdesc()[e * 3 + 2];
       const uint64_t t0 = (uint64_t)(uint32_t)tt.x | ((uint64_t)(uint32_t)tt.y << 32);
       const uint64_t t1 = (uint64_t)(uint32_t)tt.z | ((uint64_t)(uint32_t)tt.w << 32);
-      const int t = complete_job(d, sp, pending[e], t0, t1, lane, take < 0 && q_done + 1 == q_issue);
+      const bool can_take = take < 0 && q_done + 1 == q_issue;
+      if (P->job == pending[e]) {  // successors preloaded: hand-off fast path
+        const int ne = q_issue & 1;
+        const int iss = complete_job_pre(d, sp, P, t0, t1, lane, can_take, &c.jdesc()[ne * 3], &c.jfull()[ne]);
+#ifdef CHOL_HOPS
+        HOP_T(h_ret);
+        if (iss >= 0) {
+          const long long* m = g_hopt[blockIdx.x];
+          HOP_ADD(0, m[3] - h_seen);
+          HOP_ADD(1, m[0] - m[3]);
+          HOP_ADD(4, m[1] - m[0]);
+          HOP_ADD(3, h_ret - m[1]);
+          HOP_ADD(6, h_gt - t1);
+          HOP_ADD(5, 1);
+        }
+#endif
+        ++q_done;
+        if (iss >= 0) {  // the successor is running already: preload its successors
+          pending[ne] = iss;
+          ++q_issue;
+          backoff = 32;
+          preload_succ(d, P, iss, lane);
+        }
+        continue;
+      }
+      const int t = complete_job(d, sp, pending[e], t0, t1, lane, can_take);
       if (t >= 0) take = t;
+#ifdef CHOL_HOPS
+      HOP_T(h_ret);
+      if (t >= 0) {
+        const long long* m = g_hopt[blockIdx.x];
+        HOP_ADD(0, m[3] - h_seen);
+        HOP_ADD(1, m[0] - m[3]);
+        HOP_ADD(2, m[1] - m[0]);
+        HOP_ADD(3, h_ret - m[1]);
+        HOP_ADD(6, h_gt - t1);
+      }
+      h_claim_from = t >= 0 ? h_ret : 0;
+#endif
       ++q_done;
     }
     // 2. claim the next job once the ring has room and the producer is done with the
@@ -762,13 +968,29 @@ __device__ void scheduler_loop(Ctx<BS>& c, const DevSched& d, const StepParams& 
           const int inf = ld_volatile(sp.info);
           write_desc(&c.jdesc()[e * 3], job, jb, inf != INT_MAX && jb.k >= (inf - 1) / sp.nb);
           mbar_arrive(&c.jfull()[e]);
+#ifdef CHOL_HOPS
+          if (h_claim_from) {
+            atomicAdd(&g_hop[4], (unsigned long long)(clock64() - h_claim_from));
+            atomicAdd(&g_hop[5], 1ull);
+          }
+#endif
         }
+#ifdef CHOL_HOPS
+        h_claim_from = 0;
+#endif
         __syncwarp();
         pending[e] = job;
         ++q_issue;
         backoff = 32;
+        if (CHOL_PRE_MODE >= 1 && q_issue == q_done + 1) preload_succ(d, P, job, lane);
         continue;
       }
+    }
+    // the job running alone (its successor list may be needed for a hand-off)
+    if (CHOL_PRE_MODE >= 2 && q_issue == q_done + 1 && P->job != pending[q_done & 1] &&
+        P->job != -2 - pending[q_done & 1]) {
+      preload_succ(d, P, pending[q_done & 1], lane);
+      continue;
     }
     // 3. done?
     if (q_done == q_issue && (ld_volatile(d.finished) || ld_volatile(d.abort_flag))) {

@@ -45,7 +45,8 @@ struct Cfg {
   static constexpr int kPitch = BS + 2;            // doubles; keeps double2 alignment
   static constexpr int kBufBytes = BS * kPitch * 8;
   static constexpr int kBarBytes = 320;               // 21 mbarriers (176 B) + job ring descriptors + progress word
-  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kBarBytes + 1024;
+  static constexpr int kPreBytes = 1024;           // scheduler warp: successors of the running job (sched.cu)
+  static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kBarBytes + kPreBytes + 1024;
   static_assert(2 * BS * 10 + 128 <= BS * kPitch, "potf2 panels fit in lbuf behind dd / rdv");
   static_assert(kBufBytes >= BS * BS * 8, "lbuf holds a TMA-prefetched BS x BS C block");
   static constexpr int RW = BS / kComputeWarps;    // rows per warp in the solves
@@ -91,6 +92,9 @@ struct Ctx {
   __device__ uint64_t* rbar() const { return sfree() + 1; }   // [2] RECV bulk-copy buffers (thread 0 only)
   // 2*kStages + 11 = 21 barriers = 168 bytes; then 2 x 3 int4 job descriptors + producer progress word
   __device__ int4* jdesc() const { return reinterpret_cast<int4*>(bars() + 176); }
+  // scheduler warp only: the successor list of the running job's node, preloaded while the
+  // job runs (sched.cu SuccPre)
+  __device__ static char* pre() { return bars() + Cfg<BS>::kBarBytes; }
   uint32_t it;     // stages consumed so far
   uint32_t cphase; // parity of the next cbar completion
   uint32_t rcount; // RECV bulk copies (thread 0): bit h = parity of the next completion of rbar[h]
