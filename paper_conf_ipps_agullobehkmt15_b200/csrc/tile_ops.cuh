@@ -33,6 +33,8 @@ constexpr int kBox = 16;  // doubles per TMA box row (128 bytes)
 constexpr int kBarCompute = 1;  // named barrier id: compute warps only
 constexpr int kBarAll = 2;      // named barrier id: all warps
 constexpr int kBarDiag = 3;     // named barrier id: panel owner warp -> diagonal-factor warp (potf2_block)
+constexpr int kBarPivot = 4;    // potf2_block: factored diagonal block published (factor warp -> row warps)
+constexpr int kBarPanel = 5;    // potf2_block: solved panel published (row warps only)
 
 
 template <int BS>
@@ -47,7 +49,7 @@ struct Cfg {
   static constexpr int kBarBytes = 320;               // 21 mbarriers (176 B) + job ring descriptors + progress word
   static constexpr int kPreBytes = 1024;           // scheduler warp: successors of the running job (sched.cu)
   static constexpr int kSmemBytes = kPipeBytes + kBufBytes + kBarBytes + kPreBytes + 1024;
-  static_assert(2 * BS * 10 + 128 <= BS * kPitch, "potf2 panels fit in lbuf behind dd / rdv");
+  static_assert(2 * BS * 10 + 160 <= BS * kPitch, "potf2 panels fit in lbuf behind dd / rdv");
   static_assert(kBufBytes >= BS * BS * 8, "lbuf holds a TMA-prefetched BS x BS C block");
   static constexpr int RW = BS / kComputeWarps;    // rows per warp in the solves
   static constexpr int CPL = BS / 32;              // columns per lane in the solves
@@ -76,8 +78,8 @@ struct Ctx {
   __device__ char* pipe() const { return base(); }  // kStages x {A, B} operand buffers
   __device__ double* buf() const { return reinterpret_cast<double*>(base()); }  // solve buffer (aliases pipe)
   __device__ double* lbuf() const { return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes); }  // BS x kPitch
-  __device__ double* pans() const {  // potf2: two BS x 8 panels, in lbuf behind dd (64) / rdv (8)
-    return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes) + 128;
+  __device__ double* pans() const {  // potf2: two BS x 8 panels, in lbuf behind two dd (64) / rdv (8) slots
+    return reinterpret_cast<double*>(base() + Cfg<BS>::kPipeBytes) + 160;
   }
   __device__ uint64_t* full() const { return reinterpret_cast<uint64_t*>(bars()); }  // kStages
   __device__ uint64_t* empty() const { return full() + kStages; }                     // kStages
@@ -827,22 +829,6 @@ __device__ __forceinline__ void factor_8x8(double* dd, double* rdv, int* info, i
     for (int q = 0; q <= r; ++q) dd[r * 8 + q] = v[r][q];
 }
 
-// Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
-// L196-199), blocked right-looking over 8-column panels p, register resident in a
-// row layout with paired row blocks: warp w < NB/2 owns the 8-row blocks rb = w and
-// rb = NB-1-w (13 of the 78 lower 8x8 blocks each for BS = 96: balanced work, and
-// NB+1 fragment slots per thread instead of 2*NB -- column cb of the first block in
-// slot cb, of the second in slot NB-cb, disjoint since cb <= w < NB-cb).  Per panel:
-//   (1) the owner of the diagonal block updates it first and hands it to the idle
-//       warp 7 (named barrier kBarDiag), which factors it with one thread in
-//       registers (column algorithm of SURVEY §8c, one rsqrt per column) while the
-//       other warps finish their updates (one-panel lookahead);
-//   (2) after a compute barrier every warp solves its rows below against L_pp (quad
-//       shuffles) and publishes them to shared memory;
-//   (3) after a second barrier every warp applies the rank-8 update to its lower
-//       blocks with FP64 DMMA (A operand = its own solved fragments).
-// A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
-// reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
 #ifndef POTF2_STAMP
 #define POTF2_STAMP(id)  // microbenchmark hook (tools/microbench/potf2_phases.cu)
 #endif
@@ -862,120 +848,135 @@ struct Potf2Regs {
 
 // One 8-column panel P of potf2_block.  P is a template parameter so that every index
 // into x is a compile-time constant (a runtime panel index puts x in local memory:
-// 208-byte stack frame, 3x slower).
+// 208-byte stack frame, 3x slower).  dd / rdv: the slot of panel P (double-buffered by
+// parity: the owner of block P+1 hands it over while the other row warps still read L_PP).
 template <int BS, int P>
-__device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, double* dd, double* rdv) {
+__device__ __forceinline__ void potf2_panel(const Ctx<BS>& c, Potf2Regs<BS>& s, double* dd0) {
   using R = Potf2Regs<BS>;
   constexpr int NB = R::NB, kHalf = NB / 2;
+  constexpr int kRowThreads = kHalf * 32;         // row warps 0 .. NB/2-1
   constexpr int pm = P < kHalf ? 0 : 1;           // which of its blocks holds row block P
   constexpr int pw = P < kHalf ? P : NB - 1 - P;  // the warp owning row block P
   double* pan = c.pans() + (P & 1) * BS * kPanelPitch;
+  const double* dd = dd0 + (P & 1) * 72;
+  const double* rdv = dd + 64;
   const int g = s.g, t = s.t;
-  bar_sync(kBarCompute, kComputeThreads);  // L_pp and 1/L[j][j] published
+  bar_sync(kBarPivot, kRowThreads + 32);  // L_PP and 1/L[j][j] published by the factor warp
   POTF2_STAMP(0);
-  if (s.active) {
-    if (c.warp == pw) {
-      const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
-      s.x[R::sl(pm, P)][0] = l.x;
-      s.x[R::sl(pm, P)][1] = l.y;
-    }
-    // (2) rows below the diagonal block: L[r, panel] = A[r, panel] L_pp^{-T}
-#pragma unroll
-    for (int j = 0; j < 8; ++j) {
-      const double rd = rdv[j];
-      const double l0 = dd[(2 * t) * 8 + j], l1 = dd[(2 * t + 1) * 8 + j];
-#pragma unroll
-      for (int mi = 0; mi < 2; ++mi) {
-        if (s.rb(mi) <= P) continue;  // warp-uniform
-        double* xs = s.x[R::sl(mi, P)];
-        const double xj = __shfl_sync(0xffffffffu, xs[j & 1], s.qbase | (j >> 1)) * rd;
-        if (t == (j >> 1)) xs[j & 1] = xj;
-        if (2 * t > j) xs[0] = fma(-xj, l0, xs[0]);
-        if (2 * t + 1 > j) xs[1] = fma(-xj, l1, xs[1]);
-      }
-    }
-#pragma unroll
-    for (int mi = 0; mi < 2; ++mi)
-      if (s.rb(mi) > P)
-        *reinterpret_cast<double2*>(pan + (8 * s.rb(mi) + g) * kPanelPitch + 2 * t) =
-            make_double2(s.x[R::sl(mi, P)][0], s.x[R::sl(mi, P)][1]);
+  if (c.warp == pw) {
+    const double2 l = *reinterpret_cast<const double2*>(dd + g * 8 + 2 * t);
+    s.x[R::sl(pm, P)][0] = l.x;
+    s.x[R::sl(pm, P)][1] = l.y;
   }
+  // (2) rows below the diagonal block: L[r, panel] = A[r, panel] L_PP^{-T}
+#pragma unroll
+  for (int j = 0; j < 8; ++j) {
+    const double rd = rdv[j];
+    const double l0 = dd[(2 * t) * 8 + j], l1 = dd[(2 * t + 1) * 8 + j];
+#pragma unroll
+    for (int mi = 0; mi < 2; ++mi) {
+      if (s.rb(mi) <= P) continue;  // warp-uniform
+      double* xs = s.x[R::sl(mi, P)];
+      const double xj = __shfl_sync(0xffffffffu, xs[j & 1], s.qbase | (j >> 1)) * rd;
+      if (t == (j >> 1)) xs[j & 1] = xj;
+      if (2 * t > j) xs[0] = fma(-xj, l0, xs[0]);
+      if (2 * t + 1 > j) xs[1] = fma(-xj, l1, xs[1]);
+    }
+  }
+  if constexpr (P + 1 < NB) {
+    // (3a) the owner of row block P+1 updates its diagonal block first -- both operands are
+    // its own solved fragments (B[t][g] = L[8(P+1)+g][c0+2t] is the thread's A value) -- and
+    // hands it to the factor warp before the panel barrier: the next pivot does not wait
+    // for the other row warps' solves
+    constexpr int nm = (P + 1) < kHalf ? 0 : 1;
+    constexpr int nw = (P + 1) < kHalf ? P + 1 : NB - 2 - P;
+    if (c.warp == nw) {
+      const double a0 = s.x[R::sl(nm, P)][0], a1 = s.x[R::sl(nm, P)][1];
+      double* xd = s.x[R::sl(nm, P + 1)];
+      dmma884(xd[0], xd[1], -a0, a0);
+      dmma884(xd[0], xd[1], -a1, a1);
+      *reinterpret_cast<double2*>(dd0 + ((P + 1) & 1) * 72 + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
+      bar_arrive(kBarDiag, 64);
+      POTF2_STAMP(3);
+    }
+  }
+#pragma unroll
+  for (int mi = 0; mi < 2; ++mi)
+    if (s.rb(mi) > P)
+      *reinterpret_cast<double2*>(pan + (8 * s.rb(mi) + g) * kPanelPitch + 2 * t) =
+          make_double2(s.x[R::sl(mi, P)][0], s.x[R::sl(mi, P)][1]);
   POTF2_STAMP(1);
-  bar_sync(kBarCompute, kComputeThreads);  // panel p published; dd / rdv free
+  bar_sync(kBarPanel, kRowThreads);  // panel P published
   POTF2_STAMP(2);
   if constexpr (P + 1 < NB) {
-    if (s.active) {
-      // (3) rank-8 update of this warp's lower blocks (rb >= cb > p); block (p+1, p+1)
-      // first, handed to the factor warp before the rest
-      constexpr int nm = (P + 1) < kHalf ? 0 : 1;
-      constexpr int nw = (P + 1) < kHalf ? P + 1 : NB - 2 - P;
-      if (c.warp == nw) {
-        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * (P + 1) + g) * kPanelPitch + 2 * t);
-        double* xd = s.x[R::sl(nm, P + 1)];
-        dmma884(xd[0], xd[1], -s.x[R::sl(nm, P)][0], bv.x);
-        dmma884(xd[0], xd[1], -s.x[R::sl(nm, P)][1], bv.y);
-        *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(xd[0], xd[1]);
-        bar_arrive(kBarDiag, 64);
-        POTF2_STAMP(3);
-      }
+    // (3b) rank-8 update of this warp's other lower blocks (rb >= cb > P)
+    constexpr int nm = (P + 1) < kHalf ? 0 : 1;
+    constexpr int nw = (P + 1) < kHalf ? P + 1 : NB - 2 - P;
 #pragma unroll
-      for (int cb = P + 1; cb < NB; ++cb) {
-        if (cb > s.rb1) continue;  // warp-uniform (rb1 >= rb0)
-        const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * cb + g) * kPanelPitch + 2 * t);
+    for (int cb = P + 1; cb < NB; ++cb) {
+      if (cb > s.rb1) continue;  // warp-uniform (rb1 >= rb0)
+      const double2 bv = *reinterpret_cast<const double2*>(pan + (8 * cb + g) * kPanelPitch + 2 * t);
 #pragma unroll
-        for (int mi = 0; mi < 2; ++mi) {
-          if (s.rb(mi) < cb) continue;
-          if (cb == P + 1 && mi == nm && c.warp == nw) continue;  // done above
-          dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][0], bv.x);
-          dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][1], bv.y);
-        }
+      for (int mi = 0; mi < 2; ++mi) {
+        if (s.rb(mi) < cb) continue;
+        if (cb == P + 1 && mi == nm && c.warp == nw) continue;  // done above
+        dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][0], bv.x);
+        dmma884(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1], -s.x[R::sl(mi, P)][1], bv.y);
       }
-      POTF2_STAMP(4);
     }
+    POTF2_STAMP(4);
   }
 }
 
 template <int BS, int... P>
-__device__ __forceinline__ void potf2_panels(const Ctx<BS>& c, Potf2Regs<BS>& s, double* dd, double* rdv,
+__device__ __forceinline__ void potf2_panels(const Ctx<BS>& c, Potf2Regs<BS>& s, double* dd0,
                                              std::integer_sequence<int, P...>) {
-  (potf2_panel<BS, P>(c, s, dd, rdv), ...);
+  (potf2_panel<BS, P>(c, s, dd0), ...);
 }
 
 // Cholesky of the BS x BS diagonal block A (ld lda), lower, in place (POTRF,
 // L196-199), blocked right-looking over 8-column panels p, register resident in a
-// row layout with paired row blocks: warp w < NB/2 owns the 8-row blocks rb = w and
+// row layout with paired row blocks: row warp w < NB/2 owns the 8-row blocks rb = w and
 // rb = NB-1-w (13 of the 78 lower 8x8 blocks each for BS = 96: balanced work, and
 // NB+1 fragment slots per thread instead of 2*NB).  Per panel (potf2_panel):
-//   (1) the owner of the diagonal block updates it first and hands it to the idle
-//       warp 7 (named barrier kBarDiag), which factors it with one thread in
-//       registers (column algorithm of SURVEY §8c, one rsqrt per column) while the
-//       other warps finish their updates (one-panel lookahead);
-//   (2) after a compute barrier every warp solves its rows below against L_pp (quad
-//       shuffles) and publishes them to shared memory;
-//   (3) after a second barrier every warp applies the rank-8 update to its lower
-//       blocks with FP64 DMMA (A operand = its own solved fragments).
+//   (1) warp 7 factors the diagonal block p with one thread in registers (column
+//       algorithm of SURVEY §8c, one rsqrt per column) and publishes it (kBarPivot);
+//   (2) every row warp solves its rows below against L_pp (quad shuffles); the owner of
+//       row block p+1 at once updates its diagonal block (p+1, p+1) with its own
+//       fragments and hands it to warp 7 (kBarDiag) -- the next pivot does not wait for
+//       the other row warps' solves or the panel barrier;
+//   (3) the row warps publish the panel (kBarPanel, row warps only) and apply the
+//       rank-8 update to their other lower blocks with FP64 DMMA.
+// The 8x8 diagonal block and its reciprocals are double-buffered by panel parity.
+// (Measured and not taken, round 2: the factor warp alone on its SM sub-partition with the
+// row warps on warps 0-2 / 4-6, the owner solving its hand-off row block first, and an
+// mbarrier instead of kBarPivot -- potf2 alone 39.2K -> 37.0K cycles, but the factorization
+// slower: the update DMMAs of six row warps on three sub-partitions.)
 // A pivot !(d > 0) records info = col0 + c + 1 with atomicMin (LAPACK convention,
 // reading R6).  The block is stored whole: L on and below the diagonal, zeros above.
 template <int BS>
 __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda, int col0, int* info) {
-  constexpr int NB = BS / 8;
+  constexpr int NB = BS / 8, kHalf = NB / 2;
   static_assert(NB % 2 == 0 && NB / 2 <= 7, "paired row blocks; warp 7 factors the diagonal blocks");
   using R = Potf2Regs<BS>;
-  double* dd = c.lbuf();        // 8 x 8 diagonal block (pitch 8) + 8 reciprocals
-  double* rdv = c.lbuf() + 64;
+  double* dd0 = c.lbuf();  // two slots of 8 x 8 diagonal block (pitch 8) + 8 reciprocals (72 doubles)
   bar_sync(kBarCompute, kComputeThreads);  // lbuf / pans reuse
   if (c.warp == 7) {
     // factor warp: its own loop, disjoint from the row-block code (register pressure)
 #pragma unroll 1
     for (int p = 0; p < NB; ++p) {
-      bar_sync(kBarDiag, 64);  // diagonal block p is in dd
+      bar_sync(kBarDiag, 64);  // diagonal block p is in its slot
       POTF2_STAMP(5);
-      if (c.lane == 0) factor_8x8(dd, rdv, info, col0 + 8 * p);
+      double* dd = dd0 + (p & 1) * 72;
+      if (c.lane == 0) factor_8x8(dd, dd + 64, info, col0 + 8 * p);
       POTF2_STAMP(6);
-      __syncwarp();  // bar.sync is .aligned: the warp reconverges after lane 0's factor first
-      bar_sync(kBarCompute, kComputeThreads);  // L_pp published
-      bar_sync(kBarCompute, kComputeThreads);  // panel p published
+      __syncwarp();
+      bar_arrive(kBarPivot, kHalf * 32 + 32);  // L_pp published to the row warps
     }
+    bar_sync(kBarCompute, kComputeThreads);
+    return;
+  }
+  if (c.warp >= kHalf) {  // no row blocks
     bar_sync(kBarCompute, kComputeThreads);
     return;
   }
@@ -983,45 +984,41 @@ __device__ __forceinline__ void potf2_block(const Ctx<BS>& c, double* A, int lda
   s.g = c.lane >> 2;
   s.t = c.lane & 3;
   s.qbase = c.lane & ~3;
-  s.active = c.warp < NB / 2;
+  s.active = true;
   s.rb0 = c.warp;
   s.rb1 = NB - 1 - c.warp;
   const int g = s.g, t = s.t;
-  if (s.active) {
 #pragma unroll
-    for (int mi = 0; mi < 2; ++mi)
+  for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
-      for (int cb = 0; cb < NB; ++cb) {
-        if (cb > s.rb(mi)) continue;  // strictly upper blocks: never needed
-        const double2 v =
-            __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t));
-        s.x[R::sl(mi, cb)][0] = v.x;
-        s.x[R::sl(mi, cb)][1] = v.y;
-      }
-    if (c.warp == 0) {  // hand over the first diagonal block (rb0 = 0, slot 0)
-      *reinterpret_cast<double2*>(dd + g * 8 + 2 * t) = make_double2(s.x[0][0], s.x[0][1]);
-      bar_arrive(kBarDiag, 64);
+    for (int cb = 0; cb < NB; ++cb) {
+      if (cb > s.rb(mi)) continue;  // strictly upper blocks: never needed
+      const double2 v =
+          __ldcg(reinterpret_cast<const double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t));
+      s.x[R::sl(mi, cb)][0] = v.x;
+      s.x[R::sl(mi, cb)][1] = v.y;
     }
+  if (c.warp == 0) {  // hand over the first diagonal block (rb0 = 0, slot 0)
+    *reinterpret_cast<double2*>(dd0 + g * 8 + 2 * t) = make_double2(s.x[0][0], s.x[0][1]);
+    bar_arrive(kBarDiag, 64);
   }
-  potf2_panels<BS>(c, s, dd, rdv, std::make_integer_sequence<int, NB>{});
-  if (s.active) {
-    // the whole block is written: L on and below the diagonal, zeros above it (the
-    // strictly upper triangle of the factor is zero; written here so a diagonal tile
-    // can be copied out as soon as its POTRF completes)
+  potf2_panels<BS>(c, s, dd0, std::make_integer_sequence<int, NB>{});
+  // the whole block is written: L on and below the diagonal, zeros above it (the
+  // strictly upper triangle of the factor is zero; written here so a diagonal tile
+  // can be copied out as soon as its POTRF completes)
 #pragma unroll
-    for (int mi = 0; mi < 2; ++mi)
+  for (int mi = 0; mi < 2; ++mi)
 #pragma unroll
-      for (int cb = 0; cb < NB; ++cb) {
-        double2 v = make_double2(0.0, 0.0);
-        if (cb < s.rb(mi)) {
-          v = make_double2(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1]);
-        } else if (cb == s.rb(mi)) {
-          v.x = 2 * t <= g ? s.x[R::sl(mi, cb)][0] : 0.0;
-          v.y = 2 * t + 1 <= g ? s.x[R::sl(mi, cb)][1] : 0.0;
-        }
-        __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t), v);
+    for (int cb = 0; cb < NB; ++cb) {
+      double2 v = make_double2(0.0, 0.0);
+      if (cb < s.rb(mi)) {
+        v = make_double2(s.x[R::sl(mi, cb)][0], s.x[R::sl(mi, cb)][1]);
+      } else if (cb == s.rb(mi)) {
+        v.x = 2 * t <= g ? s.x[R::sl(mi, cb)][0] : 0.0;
+        v.y = 2 * t + 1 <= g ? s.x[R::sl(mi, cb)][1] : 0.0;
       }
-  }
+      __stcg(reinterpret_cast<double2*>(A + (int64_t)(8 * s.rb(mi) + g) * lda + 8 * cb + 2 * t), v);
+    }
   bar_sync(kBarCompute, kComputeThreads);
 }
 

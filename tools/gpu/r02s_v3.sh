@@ -1,0 +1,5 @@
+export PYTHONUNBUFFERED=1
+for i in 1 2; do variants/bin/pt_old; variants/bin/pt_new; variants/bin/pt_v3; done > gpurun_out/potf2_total_v3.txt 2>&1
+variants/bin/pp2_v3 > gpurun_out/pp2_v3.txt 2>&1
+timeout 600 python -m pytest tests/test_gpu_parity.py tests/test_gpu_production.py -m gpu -x -q > gpurun_out/pytest_v3.txt 2>&1
+timeout 900 python tools/libab.py 960,3840,7680,9600,11520,19200 variants/s2keep.so variants/pf.so variants/v3.so --rounds 2 --reps 5 > gpurun_out/ab7.txt 2>&1
