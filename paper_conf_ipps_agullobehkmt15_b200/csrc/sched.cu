@@ -579,6 +579,11 @@ __device__ unsigned long long g_phase[8];
 __device__ __forceinline__ long long phase_clock() { return clock64(); }
 #define PHASE_ADD(i, v) \
   if (threadIdx.x == 0) atomicAdd(&g_phase[i], (unsigned long long)(v))
+// TRSM row-slab jobs, per column block (warp 0): [0] Y mainloop (issue), [1] drain of its DMMA
+// queue, [2] Y mainloop + stage_y, [3] Z mainloop, [4] stage_z, [5] blocks, [6] block 1's Y
+__device__ unsigned long long g_tphase[8];
+#define TPHASE_ADD(i, v) \
+  if (threadIdx.x == 0) atomicAdd(&g_tphase[i], (unsigned long long)(v))
 #else
 #define PHASE_ADD(i, v)
 #endif
@@ -604,6 +609,13 @@ void sched_phase_dump() {
           h[3] / nj, h[4] / nj, h[6] / nj);
   const unsigned long long z[8] = {};
   cudaMemcpyToSymbol(g_phase, z, sizeof(z));
+  unsigned long long tp[8];
+  cudaMemcpyFromSymbol(tp, g_tphase, sizeof(tp));
+  const double nbk = tp[5] ? (double)tp[5] : 1.0;
+  fprintf(stderr, "CHOL_PHASES trsm blocks %llu  cycles/block: Y mainloop %.0f (drain %.0f)  Y+stage_y %.0f  Z %.0f  "
+          "stage_z %.0f  block-1 Y %.0f\n", tp[5], tp[0] / nbk, tp[1] / nbk, tp[2] / nbk, tp[3] / nbk, tp[4] / nbk,
+          tp[6] / (nbk / 10.0));
+  cudaMemcpyToSymbol(g_tphase, z, sizeof(z));
 #endif
 }
 
@@ -654,16 +666,43 @@ __device__ __forceinline__ void compute_job(Ctx<BS>& c, const DevSched& d, int t
     const int i = d0.z, k = d1.x, slab = d1.y, nbb = c.nb / BS;
     prefetch_l2_rows<BS>(c.tile(i, k) + (int64_t)slab * BS * c.nb, c.nb, BS, c.nb);
     for (int cb = 0; cb < nbb; ++cb) {
+#ifdef CHOL_PHASES
+      const long long q0 = phase_clock();
+#endif
       {
         Acc<BS> acc;
         gemm_consume(c, cb * BS / BK, acc);  // zero for cb = 0
+#ifdef CHOL_PHASES
+        const long long q1 = phase_clock();
+        TPHASE_ADD(0, q1 - q0);
+        {
+          volatile double sink = acc[Cfg<BS>::MI - 1][Cfg<BS>::NI - 1][1] + acc[0][0][0];
+          (void)sink;
+        }
+        const long long q2 = phase_clock();
+        TPHASE_ADD(1, q2 - q1);
+#endif
         trsm_stage_y(c, acc);
       }
+#ifdef CHOL_PHASES
+      const long long q3 = phase_clock();
+#endif
       Acc<BS> z;
       gemm_consume<BS, true>(c, BS / BK, z);
+#ifdef CHOL_PHASES
+      const long long q4 = phase_clock();
+#endif
       trsm_stage_z(c, z);
       __syncwarp();
       if (c.lane == 0) mbar_arrive(c.cready());  // the storer writes Z_cb back
+#ifdef CHOL_PHASES
+      const long long q5 = phase_clock();
+      TPHASE_ADD(2, q3 - q0);
+      TPHASE_ADD(3, q4 - q3);
+      TPHASE_ADD(4, q5 - q4);
+      if (cb == 1) TPHASE_ADD(6, q3 - q0);
+      TPHASE_ADD(5, 1);
+#endif
     }
   } else if (type == J_INV) {
     const int k = d1.x, b = d1.y, nbb = c.nb / BS;

@@ -31,6 +31,7 @@ with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, policy=c.POLICY_CP_PRIORITY, trace
         if rep and (best is None or t < best[0]):
             best = (t, jt.copy())
 t_f, jt = best
+jt = jt[jt[:, 1] > 0]  # untraced jobs (INV: no paper task) carry no times
 t0, t1, tq = (jt[:, x].astype(np.int64) for x in (0, 1, 4))
 typ = (jt[:, 3] >> np.uint64(32)).astype(np.int64)
 base = min(tq.min(), t0.min())

@@ -1,0 +1,3 @@
+export PYTHONUNBUFFERED=1
+CHOL_LIB_OVERRIDE=variants/sv4.so timeout 600 python -m pytest tests/test_gpu_solve.py -m gpu -x -q > gpurun_out/pytest_sv4.txt 2>&1
+for lib in variants/pf2.so variants/sv4.so; do echo $lib; CHOL_LIB_OVERRIDE=$lib timeout 300 python tools/solve_bench.py 19200 1,96,192,960; CHOL_LIB_OVERRIDE=$lib timeout 300 python tools/solve_bench.py 46080 96,960; done > gpurun_out/solve_ab4.txt 2>&1
