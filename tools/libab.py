@@ -37,16 +37,18 @@ a = ap.parse_args()
 res = {}
 for rnd in range(a.rounds):
     for n in [int(x) for x in a.ns.split(",")]:
-        for lib in a.libs:
+        for spec in a.libs:  # path[:VAR=value,...] (extra environment for that build)
+            lib, _, extra = spec.partition(":")
             env = dict(os.environ, CHOL_LIB_OVERRIDE=os.path.abspath(lib))
+            env.update(kv.split("=", 1) for kv in extra.split(",") if kv)
             out = subprocess.run([sys.executable, "-c", CHILD, str(n), str(a.reps)], env=env, capture_output=True,
                                  text=True, timeout=600)
             if out.returncode:
-                print(json.dumps({"lib": lib, "n": n, "error": out.stderr[-400:]}), flush=True)
+                print(json.dumps({"lib": spec, "n": n, "error": out.stderr[-400:]}), flush=True)
                 continue
             d = json.loads(out.stdout.strip().splitlines()[-1])
-            res.setdefault((lib, n), []).append(d)
-            print(json.dumps({"round": rnd, "lib": os.path.basename(lib), "n": n, **d}), flush=True)
+            res.setdefault((spec, n), []).append(d)
+            print(json.dumps({"round": rnd, "lib": os.path.basename(spec), "n": n, **d}), flush=True)
 for (lib, n), v in sorted(res.items(), key=lambda x: (x[0][1], x[0][0])):
-    print(f"{n:6d} {os.path.basename(lib):16s} median {min(x['ms'] for x in v):9.3f} ms  best {min(x['best'] for x in v):9.3f}"
+    print(f"{n:6d} {os.path.basename(lib):24s} median {min(x['ms'] for x in v):9.3f} ms  best {min(x['best'] for x in v):9.3f}"
           f"  hash {v[0]['hash']}")
