@@ -1167,11 +1167,14 @@ extern "C" int chol_solve(chol_plan_t p, double* B, int64_t ldb, int64_t nrhs) {
   // columns per work item: 1 (register-streamed matrix-vector sweeps), 32 (DMMA sweeps
   // at block 96 -- also for 2..8 columns: one padded 32-column chunk beats the 8-column
   // SIMT item), 8 or 32 (SIMT sweeps at blocks 64 / 32)
-  // 64 at block 96 from 160 columns on: half the factor re-reads per right-hand side (n=19200:
-  // nrhs 192 7.9 -> 7.1 ms, 960 35.8 -> 28.6 ms); below, 32-column chunks keep more items in
-  // flight (nrhs 96: 4.5 vs 5.4 ms).  CHOL_SOLVE_RC=32 / 64 forces one (development switch)
+  // 48 at block 96 whenever that takes fewer chunks than 32 (k_sweep_db: both operands
+  // double-buffered; a 48-column chunk costs about as much as a 32-column one: n = 19200, nrhs
+  // 48 3.03 vs 3.46 ms, 96 3.98 vs 4.54, 192 6.37 vs 7.09 (64-column k_sweep_mma), n = 46080,
+  // nrhs 960 152.6 vs 159.4 ms; nrhs 64: 3.94 vs 3.46 -- two chunks either way -- keeps 32;
+  // profiles/r02/solve_db_r02s.txt).  CHOL_SOLVE_RC=32 / 48 / 64 forces one (development switch)
   const char* erc = getenv("CHOL_SOLVE_RC");
-  const int rc_mma = erc ? (atoi(erc) == 64 ? 64 : 32) : (nrhs >= 160 ? 64 : 32);
+  const int rc_mma = erc ? (atoi(erc) == 64 ? 64 : atoi(erc) == 48 ? 48 : 32)
+                         : ((nrhs + 47) / 48 < (nrhs + 31) / 32 ? 48 : 32);
   const int rc = nrhs == 1 ? 1 : (nrhs <= 8 && p->bs != 96) ? 8 : (p->bs == 96 ? rc_mma : 32);
   const int nchunks = (int)((nrhs + rc - 1) / rc), ldw = rc * nchunks;
   const int64_t nblocks = n / p->bs;

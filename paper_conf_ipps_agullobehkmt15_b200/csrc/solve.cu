@@ -636,6 +636,200 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
   }
 }
 
+// Round 2 (second session): 48-column items with both operands double-buffered.  k_sweep_mma
+// fetches each stage's right-hand-side block after the previous stage's product (one exposed
+// L2 round trip per 96 x 96 x RC product: 70% of the DMMA pipe, ncu); here the next stage's
+// matrix AND right-hand-side block stream in under the current product.  To fit two 96 x 96
+// matrices and two 96 x 48 blocks (221 KB) the rows are unpadded and XOR-swizzled -- element
+// (r, c) at r * pitch + (c ^ 4 (r & 3)), which keeps every half-warp fragment load
+// conflict-free for both sweeps -- and each thread copies a fixed 16-byte column chunk down a
+// row stride (no per-chunk index arithmetic).  A right-hand-side block whose producer flag is
+// not up when the prefetch is due (the newest rows of the wavefront; the chain stage always)
+// is fetched at its own stage as before.  Same DMMA sequence per accumulator as k_sweep_mma.
+__device__ __forceinline__ int swz(int r, int c) { return c ^ ((r & 3) << 2); }
+
+// rows x (2 * CH) block at G (ld) -> dst (pitch, swizzled): thread tid < TPR * CH copies
+// column chunk tid % CH of rows tid / CH, tid / CH + TPR, ...
+template <int ROWS, int CH, int PITCH>
+__device__ __forceinline__ void stage_swz(double* dst, const double* G, int64_t ld) {
+  constexpr int TPR = kSolveThreads / CH;  // rows per pass
+  const int tid = threadIdx.x;
+  if (tid >= TPR * CH) return;
+  const int c2 = 2 * (tid % CH);
+  int r = tid / CH;
+  const double* src = G + (int64_t)r * ld + c2;
+  for (; r < ROWS; r += TPR, src += TPR * ld) cp_async16(dst + r * PITCH + swz(r, c2), src);
+}
+
+template <bool FWD>
+__global__ void __launch_bounds__(kSolveThreads, 1)
+    k_sweep_db(const double* tiles, int nb, int nblocks, const double* aux, double* W, int ldw, int nchunks,
+               int* flags, int* counter, int epoch) {
+  constexpr int SB = 96, RC = 48, NI = 3;
+  extern __shared__ __align__(16) double sm[];
+  auto Lb = [&](int buf) { return sm + buf * SB * SB; };
+  auto Yb = [&](int buf) { return sm + 2 * SB * SB + buf * SB * RC; };
+  int* s_item = reinterpret_cast<int*>(sm + 2 * SB * SB + 2 * SB * RC);
+  int* s_pref = s_item + 1;  // [2] right-hand-side block of the stage with this parity prefetched
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, g = lane >> 2, t = lane & 3;
+  const int R0 = 3 * (warp & 3), C0 = NI * (warp >> 2);
+  const int total = nblocks * nchunks;
+  const int64_t bsz = (int64_t)SB * SB;
+  const double* inv = aux;
+  const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
+  auto block_mma = [&](const double* Ls, const double* Ys, double (&acc)[3][NI][2]) {
+#pragma unroll 4
+    for (int k0 = 0; k0 < SB; k0 += 4) {
+      double a[3], bv[NI];
+#pragma unroll
+      for (int mi = 0; mi < 3; ++mi) {
+        const int r = 8 * (R0 + mi) + g;
+        a[mi] = FWD ? Ls[r * SB + ((k0 + t) ^ ((g & 3) << 2))] : Ls[(k0 + t) * SB + (r ^ (t << 2))];
+      }
+#pragma unroll
+      for (int ni = 0; ni < NI; ++ni) bv[ni] = Ys[(k0 + t) * RC + ((8 * (C0 + ni) + g) ^ (t << 2))];
+#pragma unroll
+      for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+        for (int ni = 0; ni < NI; ++ni) dmma884(acc[mi][ni][0], acc[mi][ni][1], a[mi], bv[ni]);
+    }
+  };
+  while (true) {
+    __syncthreads();
+    if (threadIdx.x == 0) *s_item = atomicAdd(counter, 1);
+    __syncthreads();
+    const int item = *s_item;
+    if (item >= total) break;
+    const int ch = item % nchunks;
+    const int b = FWD ? item / nchunks : nblocks - 1 - item / nchunks;
+    const int nc = FWD ? b : nblocks - 1 - b;
+    const int nold = nc > 0 ? nc - 1 : 0;
+    const int nst = nold + 1 + (nc > 0 ? 1 : 0);
+    auto cof = [&](int q) { return FWD ? q : nblocks - 1 - q; };
+    auto ysrc = [&](int q) { return q < nold ? cof(q) : (FWD ? b - 1 : b + 1); };
+    auto flag_up = [&](int q) {
+      int v;
+      asm volatile("ld.acquire.gpu.global.b32 %0, [%1];" : "=r"(v) : "l"(flags + ysrc(q) * nchunks + ch) : "memory");
+      return v == epoch;
+    };
+    auto issue_L = [&](int q) {
+      if (q < nold) {
+        const int c = cof(q);
+        stage_swz<SB, SB / 2, SB>(Lb(q & 1), FWD ? lblock(tiles, nb, SB, b, c) : lblock(tiles, nb, SB, c, b), nb);
+      } else {
+        stage_swz<SB, SB / 2, SB>(Lb(q & 1), (q == nold ? inv : Mch) + b * bsz, SB);
+      }
+    };
+    auto issue_Y = [&](int q) {
+      stage_swz<SB, RC / 2, RC>(Yb(q & 1), W + (int64_t)ysrc(q) * SB * ldw + ch * RC, ldw);
+    };
+    double* Wb = W + (int64_t)b * SB * ldw + ch * RC;
+    double rhs[3][NI][2], acc[3][NI][2];
+#pragma unroll
+    for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < NI; ++ni) {
+        const double2 v = __ldcg(reinterpret_cast<const double2*>(Wb + (int64_t)(8 * (R0 + mi) + g) * ldw +
+                                                                  8 * (C0 + ni) + 2 * t));
+        rhs[mi][ni][0] = v.x;
+        rhs[mi][ni][1] = v.y;
+        acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
+      }
+    // stage 0 (its right-hand-side block only if its producer is done) and the decision for stage 1
+    if (threadIdx.x == 0) {
+      s_pref[0] = 0 < nold && flag_up(0);
+      s_pref[1] = 1 < nold && flag_up(1);
+    }
+    __syncthreads();
+    issue_L(0);
+    if (s_pref[0]) issue_Y(0);
+    cp_async_commit();
+    for (int q = 0; q < nst; ++q) {
+      const int buf = q & 1;
+      if (q != nold && !s_pref[buf]) {  // the right-hand-side block is fetched now
+        if (threadIdx.x == 0)
+          while (!flag_up(q)) {
+          }
+        __syncthreads();
+        issue_Y(q);
+        cp_async_commit();
+      }
+      if (q + 1 < nst) {  // the next stage streams in under this one (its buffers are free)
+        issue_L(q + 1);
+        if (s_pref[buf ^ 1]) issue_Y(q + 1);
+        cp_async_commit();
+        cp_async_wait<1>();
+      } else {
+        cp_async_wait<0>();
+      }
+      if (q == nold) {  // Y = rhs - acc for the inverse; acc restarts
+#pragma unroll
+        for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+          for (int ni = 0; ni < NI; ++ni) {
+            const int r = 8 * (R0 + mi) + g;
+            *reinterpret_cast<double2*>(Yb(buf) + r * RC + swz(r, 8 * (C0 + ni) + 2 * t)) =
+                make_double2(rhs[mi][ni][0] - acc[mi][ni][0], rhs[mi][ni][1] - acc[mi][ni][1]);
+            acc[mi][ni][0] = acc[mi][ni][1] = 0.0;
+          }
+      }
+      __syncthreads();
+      if (q == nold + 1) {  // acc = U - M y
+        double m[3][NI][2];
+#pragma unroll
+        for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+          for (int ni = 0; ni < NI; ++ni) m[mi][ni][0] = m[mi][ni][1] = 0.0;
+        block_mma(Lb(buf), Yb(buf), m);
+#pragma unroll
+        for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+          for (int ni = 0; ni < NI; ++ni) {
+            acc[mi][ni][0] -= m[mi][ni][0];
+            acc[mi][ni][1] -= m[mi][ni][1];
+          }
+      } else {
+        block_mma(Lb(buf), Yb(buf), acc);
+      }
+      // stage q+2 reuses these buffers: prefetch its block only if its producer is done now
+      if (threadIdx.x == 0) s_pref[buf] = q + 2 < nold && flag_up(q + 2);
+      __syncthreads();
+    }
+#pragma unroll
+    for (int mi = 0; mi < 3; ++mi)
+#pragma unroll
+      for (int ni = 0; ni < NI; ++ni)
+        __stcg(reinterpret_cast<double2*>(Wb + (int64_t)(8 * (R0 + mi) + g) * ldw + 8 * (C0 + ni) + 2 * t),
+               make_double2(acc[mi][ni][0], acc[mi][ni][1]));
+    __syncthreads();
+    if (threadIdx.x == 0)
+      asm volatile("st.release.gpu.global.b32 [%0], %1;" ::"l"(flags + b * nchunks + ch), "r"(epoch) : "memory");
+  }
+}
+
+static cudaError_t solve_db(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
+  constexpr int SB = 96;
+  const int smem = (2 * SB * SB + 2 * SB * 48) * 8 + 16, smem_inv = 2 * SB * kInvPitch * 8;
+  cudaError_t e;
+  if ((e = cudaFuncSetAttribute(k_diag_aux<SB>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_inv))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep_db<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  if ((e = cudaFuncSetAttribute(k_sweep_db<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, smem))) return e;
+  const int nblocks = (int)(a.n / SB);
+  if (!a.inv_valid) {
+    k_diag_aux<SB><<<std::min(nblocks, a.sms), kSolveThreads, smem_inv, s>>>(a.tiles, a.nb, nblocks, a.inv);
+    ++*nlaunch;
+  }
+  const int total = nblocks * a.nchunks;
+  const int grid = std::min(total, a.sms);
+  if ((e = cudaMemsetAsync(a.ctl, 0, (2 + 2 * (size_t)total) * sizeof(int), s))) return e;
+  k_sweep_db<true><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks, a.ctl + 2,
+                                                     a.ctl, 1);
+  k_sweep_db<false><<<grid, kSolveThreads, smem, s>>>(a.tiles, a.nb, nblocks, a.inv, a.W, a.ldw, a.nchunks,
+                                                      a.ctl + 2 + total, a.ctl + 1, 1);
+  *nlaunch += 2;
+  return cudaGetLastError();
+}
+
 template <int RC>
 static cudaError_t solve_mma(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   constexpr int SB = 96;
@@ -699,6 +893,7 @@ cudaError_t solve_run(const SolveArgs& a, cudaStream_t s, int* nlaunch) {
   }
   // 32-column chunks at SB = 96 on DMMA (CHOL_SOLVE_SIMT=1: the SIMT sweeps; development switch)
   const char* esimt = getenv("CHOL_SOLVE_SIMT");
+  if (a.rc == 48 && a.sb == 96) return solve_db(a, s, nlaunch);
   if (a.rc == 64 && a.sb == 96) return solve_mma<64>(a, s, nlaunch);
   if (a.rc == 32 && a.sb == 96 && !(esimt && esimt[0] == '1')) return solve_mma<32>(a, s, nlaunch);
   const bool narrow = a.rc == 8;

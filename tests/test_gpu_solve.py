@@ -153,6 +153,22 @@ def test_solve_dmma_and_simt_sweeps_agree(nrhs, monkeypatch):
     assert np.max(np.abs(X1 - X2)) <= 1e-12 * max(1.0, float(np.max(np.abs(X1))))
 
 
+@pytest.mark.parametrize("rc", ["32", "48", "64"])
+@pytest.mark.parametrize("n,nrhs", [(3840, 101), (9600, 49)])
+def test_solve_chunk_widths_match_oracle(rc, n, nrhs, monkeypatch):
+    """Every chunk width of the block-96 DMMA sweeps -- 32 / 64 (k_sweep_mma) and 48
+    (k_sweep_db, both operands double-buffered, swizzled shared layout) -- forced with
+    CHOL_SOLVE_RC, ragged last chunk, against the oracle."""
+    c = _lib()
+    monkeypatch.setenv("CHOL_SOLVE_RC", rc)
+    p, A, L = _factor(c, n, 960, seed=4)
+    B = spdgen.rhs(n, nrhs, 11)
+    X = B.copy()
+    p.solve(X)
+    p.close()
+    _check(A, L, B, X)
+
+
 def test_solve_refuses_a_factor_that_was_overwritten_or_failed():
     """Every call that writes the tile store (generate, scatter, run_batch / run_task, a
     factorization that fails) invalidates the factor: chol_solve returns -10 instead of
