@@ -37,10 +37,10 @@ a = ap.parse_args()
 res = {}
 for rnd in range(a.rounds):
     for n in [int(x) for x in a.ns.split(",")]:
-        for spec in a.libs:  # path[:VAR=value,...] (extra environment for that build)
+        for spec in a.libs:  # path[:VAR=value+VAR2=value...] (extra environment for that build)
             lib, _, extra = spec.partition(":")
             env = dict(os.environ, CHOL_LIB_OVERRIDE=os.path.abspath(lib))
-            env.update(kv.split("=", 1) for kv in extra.split(",") if kv)
+            env.update(kv.split("=", 1) for kv in extra.split("+") if kv)
             out = subprocess.run([sys.executable, "-c", CHILD, str(n), str(a.reps)], env=env, capture_output=True,
                                  text=True, timeout=600)
             if out.returncode:
