@@ -133,9 +133,19 @@ int chol_trace(chol_plan_t p, chol_task_rec_t* recs, int64_t cap, int64_t* nrecs
  * job was enqueued (its node became ready), out[5j+3] = job type
  * << 32 | dense task id (job types: 0 SYRK/GEMM block, 1 TRSM row slab, 2 POTRF
  * diagonal block, 3 POTRF panel block, 4 POTRF update block, 5 TRSM block solve,
- * 6 TRSM block update).  At most cap jobs;
- * *njobs = number of jobs.  -7 if not available. */
+ * 6 TRSM block update, 7 remote-tile receive, 8 diagonal-block inverse (untraced: zero
+ * times), 9 no-op).  At most cap jobs; *njobs = number of jobs.  -7 if not available. */
 int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t* njobs);
+
+/* The persistent scheduler's job descriptors, in chol_job_trace's job order (available once
+ * the plan exists; tests check the block-level dependencies of the trace with them): per job
+ * j, out[8j .. 8j+7] = type (as chol_job_trace), i, j, k (the paper task's tile indices),
+ * a, b, c (type-specific: 0 block (bm, bn); 1 row slab; 2 diagonal block b, fused-update
+ * flag; 3 inner step b, block row r; 4 inner step b, block (r, q); 5 column block cb, row
+ * slab; 6 column block, row slab, target column block; 8 diagonal block b), scheduler node
+ * id.  At most cap jobs; *njobs = number of jobs.  -7 without a persistent scheduler, -8 for
+ * a multi-GPU plan. */
+int chol_job_desc(chol_plan_t p, int32_t* out, int64_t cap, int64_t* njobs);
 
 int chol_destroy(chol_plan_t p);
 const char* chol_strerror(int status);

@@ -81,6 +81,7 @@ def _load():
         "chol_task_id": ([i64, i32, i32, i32, i32, ctypes.POINTER(i64)], i32),
         "chol_bounds": ([i64, i64, i32, dp, dp, dp], i32),
         "chol_job_trace": ([P, ctypes.POINTER(ctypes.c_uint64), i64, ctypes.POINTER(i64)], i32),
+        "chol_job_desc": ([P, ctypes.POINTER(ctypes.c_int32), i64, ctypes.POINTER(i64)], i32),
         "chol_plan_dist": ([i64, i64, i32, i32, ctypes.POINTER(chol_opts_t), ctypes.POINTER(P)], i32),
         "chol_dist_export": ([P, vp, i64, ctypes.POINTER(i64)], i32),
         "chol_dist_connect": ([P, vp, i64], i32),
@@ -111,7 +112,7 @@ _lib = _load()
 EXPORTED = ("chol_plan", "chol_plan_ex", "chol_factor", "chol_trace", "chol_destroy", "chol_strerror",
             "chol_generate", "chol_scatter", "chol_gather", "chol_factor_inplace", "chol_last_times",
             "chol_get_stream", "chol_get_info", "chol_run_task", "chol_run_batch", "chol_last_launches",
-            "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_plan_dist", "chol_dist_export",
+            "chol_dag", "chol_task_id", "chol_bounds", "chol_job_trace", "chol_job_desc", "chol_plan_dist", "chol_dist_export",
             "chol_dist_connect", "chol_get_dist", "chol_factor_async", "chol_wait", "chol_dist_layout",
             "chol_lp_bound", "chol_simulate", "chol_solve", "chol_last_solve_times", "chol_scatter_tiles",
             "chol_gather_tiles", "chol_owner_area", "chol_optimal_schedule", "chol_set_task_priorities",
@@ -183,6 +184,17 @@ def chol_job_trace(plan: int):
     out = np.zeros((max(n.value, 1), 5), dtype=np.uint64)
     _check(_lib.chol_job_trace(plan, out.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)), n.value,
                                ctypes.byref(n)), "chol_job_trace")
+    return out[:n.value]
+
+
+def chol_job_desc(plan: int):
+    """numpy array (njobs, 8) int32: type, i, j, k, a, b, c, node (include/chol.h)."""
+    import numpy as np
+    n = ctypes.c_int64(0)
+    _check(_lib.chol_job_desc(plan, None, 0, ctypes.byref(n)), "chol_job_desc")
+    out = np.zeros((max(n.value, 1), 8), dtype=np.int32)
+    _check(_lib.chol_job_desc(plan, out.ctypes.data_as(ctypes.POINTER(ctypes.c_int32)), n.value,
+                              ctypes.byref(n)), "chol_job_desc")
     return out[:n.value]
 
 

@@ -1365,6 +1365,13 @@ extern "C" int chol_job_trace(chol_plan_t p, uint64_t* out, int64_t cap, int64_t
   return sched_job_trace(p->sched, out, cap, njobs);  // 5 u64 per job
 }
 
+extern "C" int chol_job_desc(chol_plan_t p, int32_t* out, int64_t cap, int64_t* njobs) {
+  if (!p) return -4;
+  if (is_multi(p)) return -8;
+  if (!p->sched) return -7;
+  return sched_job_desc(p->sched, out, cap, njobs);
+}
+
 // ------------------------------------------------------------------ calibration / single tasks
 extern "C" int chol_run_task(chol_plan_t p, int type, int i, int j, int k, int reps, double* ms) {
   if (!p) return -4;

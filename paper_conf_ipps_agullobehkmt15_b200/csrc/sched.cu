@@ -1099,6 +1099,8 @@ struct SchedState {
   std::vector<int> h_node_paper, h_node_queue;
   size_t o_nq = 0, o_qbase = 0;
   std::vector<int16_t> h_job_type;         // host copies for chol_job_trace
+  std::vector<Job> h_jobs;                 // ... and chol_job_desc
+  std::vector<int> h_job_node;
   std::vector<int> h_job_paper;
 };
 
@@ -1318,6 +1320,8 @@ static int sched_upload(SchedState** out, SchedState* st, Builder& B, const std:
   st->njobs = (int)B.jobs.size();
   st->h_job_type.resize(st->njobs);
   st->h_job_paper.resize(st->njobs);
+  st->h_jobs = B.jobs;
+  st->h_job_node = B.job_node;
   for (int j = 0; j < st->njobs; ++j) {
     st->h_job_type[j] = B.jobs[j].type;
     st->h_job_paper[j] = B.paper[B.job_node[j]];
@@ -2071,6 +2075,24 @@ int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* n
     out[5 * j + 2] = h[4 * j + 2];
     out[5 * j + 3] = ((uint64_t)(uint16_t)st->h_job_type[j] << 32) | (uint32_t)st->h_job_paper[j];
     out[5 * j + 4] = h[4 * j + 3];
+  }
+  return 0;
+}
+
+int sched_job_desc(const SchedState* st, int32_t* out, int64_t cap, int64_t* njobs) {
+  if (njobs) *njobs = st->njobs;
+  if (!out || cap <= 0) return 0;
+  for (int64_t j = 0; j < st->njobs && j < cap; ++j) {
+    const Job& jb = st->h_jobs[j];
+    int32_t* o = out + 8 * j;
+    o[0] = jb.type;
+    o[1] = jb.i;
+    o[2] = jb.j;
+    o[3] = jb.k;
+    o[4] = jb.a;
+    o[5] = jb.b;
+    o[6] = jb.c;
+    o[7] = st->h_job_node[j];
   }
   return 0;
 }

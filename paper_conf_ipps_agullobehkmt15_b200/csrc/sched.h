@@ -46,6 +46,7 @@ void sched_abort(SchedState* st);
 // in, which the scheduler's watch list follows (fixed when the plan is built).
 void sched_arrival_order(const SchedState* st, std::vector<std::pair<int, int>>& tiles);
 int sched_job_trace(const SchedState* st, uint64_t* out, int64_t cap, int64_t* njobs);
+int sched_job_desc(const SchedState* st, int32_t* out, int64_t cap, int64_t* njobs);
 void sched_destroy(SchedState* st);
 // development: print the CHOL_PHASES job-phase counters (no-op in normal builds)
 void sched_phase_dump();

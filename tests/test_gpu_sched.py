@@ -172,3 +172,118 @@ def test_injected_priorities_keep_the_factor():
     assert np.array_equal(outs[0], outs[1])
     ref, _ = oracle.chol_tiled(spdgen.uniform_spd(n, 3), nb)
     assert oracle.rel_diff(outs[1], ref)["max_rel_floored"] <= 1e-10
+
+
+@pytest.mark.parametrize("n,env", [(3840, {}), (7680, {}), (9600, {"CHOL_POTRF_BLOCKDAG": "0"}),
+                                   (19200, {}), (5760, {"CHOL_TRSM_TAIL": "0", "CHOL_TRSM_BLOCKS": "1"})])
+def test_job_trace_respects_block_level_dag(n, env, monkeypatch):
+    """The job trace against the block-level dependencies of Algorithm 1's tile operations
+    (chol_job_desc gives each job's blocks): a job starts only after every job that wrote a
+    block it reads or overwrites has ended -- in the hybrid block tail, inside the POTRF block
+    DAG, across the task-level steps, and for every TRSM decomposition (row slabs, the
+    right-looking column steps).  t0 / t1: globaltimer at the compute warps' start / end."""
+    c = _lib()
+    for k_, v_ in env.items():
+        monkeypatch.setenv(k_, v_)
+    nb = 960
+    with c.Plan(n, nb, executor=c.EXEC_SCHEDULER, trace=2) as p:
+        c.chol_generate(p.h, 1, 0)
+        assert c.chol_factor_inplace(p.h) == 0
+        jt = c.chol_job_trace(p.h)
+        jd = c.chol_job_desc(p.h)
+    assert len(jt) == len(jd)
+    t0, t1 = jt[:, 0].astype(np.int64), jt[:, 1].astype(np.int64)
+    typ = (jt[:, 3] >> np.uint64(32)).astype(np.int64)
+    assert np.array_equal(typ, jd[:, 0])
+    UPD, TRSM, DIAG, PANEL, PUPD, TS, TU = 0, 1, 2, 3, 4, 5, 6
+    from collections import defaultdict
+    # last end time of the writers of each block group
+    upd = {}                    # (i, j, k, bm, bn) -> t1
+    slab_w = defaultdict(int)   # (i, k, slab) -> max t1 of the TRSM jobs writing that row slab
+    ts_w = {}                   # (i, k, cb, sl) -> t1
+    tu_w = defaultdict(int)     # (i, k, sl, c2) -> max t1 of the TU jobs writing block (sl, c2)
+    potrf_end = defaultdict(int)  # k -> max t1 of POTRF_k's jobs
+    diag, panel, pupd = {}, {}, {}
+    for x in range(len(jd)):
+        ty, i, j, k, a, b, cc, _ = (int(v) for v in jd[x])
+        if t1[x] == 0:
+            continue  # untraced (diagonal-block inverses)
+        if ty == UPD:
+            upd[(i, j, k, a, b)] = t1[x]
+        elif ty == TRSM:
+            slab_w[(i, k, a)] = max(slab_w[(i, k, a)], t1[x])
+        elif ty == TS:
+            ts_w[(i, k, a, b)] = t1[x]
+            slab_w[(i, k, b)] = max(slab_w[(i, k, b)], t1[x])
+        elif ty == TU:
+            tu_w[(i, k, b, cc)] = max(tu_w[(i, k, b, cc)], t1[x])
+            slab_w[(i, k, b)] = max(slab_w[(i, k, b)], t1[x])
+        elif ty in (DIAG, PANEL, PUPD):
+            potrf_end[k] = max(potrf_end[k], t1[x])
+            if ty == DIAG:
+                diag[(k, a)] = t1[x]
+            elif ty == PANEL:
+                panel[(k, a, b)] = t1[x]
+            else:
+                pupd[(k, a, b, cc)] = t1[x]
+    nbb = nb // 96
+    bad = []
+    nchecked = [0]
+
+    def need(x, t_prev, what):
+        if t_prev is None:
+            return
+        nchecked[0] += 1
+        if t0[x] < t_prev:
+            bad.append((tuple(int(v) for v in jd[x]), what, int(t_prev - t0[x])))
+
+    for x in range(len(jd)):
+        ty, i, j, k, a, b, cc, _ = (int(v) for v in jd[x])
+        if t1[x] == 0:
+            continue
+        if ty == UPD:  # C(i, j)[a, b] -= L(i, k)[a, :] L(j, k)[b, :]^T
+            need(x, slab_w.get((i, k, a)), "operand slab of L_ik")
+            need(x, slab_w.get((j, k, b)), "operand slab of L_jk")
+            need(x, upd.get((i, j, k - 1, a, b)), "previous update of the block")
+        elif ty == TRSM:  # row slab a of A_ik
+            for bn in range(nbb):
+                need(x, upd.get((i, k, k - 1, a, bn)), "last update of the slab")
+            need(x, potrf_end.get(k), "L_kk")
+        elif ty == TS:  # block (b, a) of A_ik, column block a
+            need(x, upd.get((i, k, k - 1, b, a)), "last update of the block")
+            need(x, tu_w.get((i, k, b, a)), "right-looking updates of the block")
+            need(x, diag.get((k, a)), "L_kk diagonal block")
+        elif ty == TU:  # block (b, cc) -= X[b, a] L_kk[cc, a]^T
+            need(x, ts_w.get((i, k, a, b)), "solved block")
+            need(x, upd.get((i, k, k - 1, b, cc)), "last update of the block")
+            need(x, panel.get((k, a, cc)), "L_kk off-diagonal block")
+        elif ty == DIAG:
+            need(x, upd.get((k, k, k - 1, a, a)), "SYRK of the previous step")
+            need(x, panel.get((k, a - 1, a)), "panel block feeding the fused update")
+            for b2 in range(a):
+                need(x, pupd.get((k, b2, a, a)), "inner updates of the block")
+        elif ty == PANEL:
+            need(x, diag.get((k, a)), "diagonal block")
+            need(x, upd.get((k, k, k - 1, b, a)), "SYRK of the previous step")
+            for b2 in range(a):
+                need(x, pupd.get((k, b2, b, a)), "inner updates of the block")
+        elif ty == PUPD:
+            need(x, panel.get((k, a, b)), "panel block r")
+            need(x, panel.get((k, a, cc)), "panel block q")
+            need(x, upd.get((k, k, k - 1, b, cc)), "SYRK of the previous step")
+            for b2 in range(a):
+                need(x, pupd.get((k, b2, b, cc)), "inner updates of the block")
+    assert not bad, bad[:10]
+    assert len(upd) > 0 and len(diag) > 0
+    # every update job checks its two operand slabs; the inner POTRF and TRSM jobs their blocks
+    assert nchecked[0] >= 2 * len(upd) + len(diag), (nchecked[0], len(upd), len(diag))
+    # the checks bite: a trace whose start times are all shifted before the end of the
+    # first traced job fails them
+    t0_saved = t0.copy()
+    t0[:] = t1[t1 > 0].min() - 1
+    bad.clear()
+    for x in range(len(jd)):
+        if int(jd[x, 0]) == UPD and t1[x] > 0:
+            need(x, slab_w.get((int(jd[x, 1]), int(jd[x, 3]), int(jd[x, 4]))), "operand slab of L_ik")
+    t0[:] = t0_saved
+    assert bad
