@@ -3,20 +3,21 @@
 // factor (A = L L^T "is used to solve" the SPD system).
 //
 // B200 form.  The right-hand sides live in a padded device buffer W (n x ldw, row-major,
-// ldw = 32 * nchunks); the unknowns are cut into SB-row blocks (SB = the plan's block, 96
-// at nb = 960) and the right-hand sides into chunks of 32 columns (one per lane).  One
-// work item = (block row b, chunk) computes
+// ldw = RC * nchunks); the unknowns are cut into SB-row blocks (SB = the plan's block, 96
+// at nb = 960) and the right-hand sides into chunks of RC columns (1: register-streamed
+// sweeps; 32 / 48 / 64 at SB = 96 on FP64 DMMA -- k_sweep_mma, k_sweep_db; 8 / 32 for the
+// SIMT sweeps at SB = 64 / 32; chol_solve picks).  One work item = (block row b, chunk)
+// computes
 //     forward:  Y_b = inv(L_bb) (B_b - sum_{c<b} L_bc Y_c)
 //     backward: X_b = inv(L_bb)^T (Y_b - sum_{c>b} L_cb^T X_c)
 // where inv(L_bb) is the inverse of the SB x SB diagonal block, computed once per
 // factorization (k_diag_inv): the sequential substitution inside a block becomes a small
-// product, so the chain from block to block is one flag hop plus one SB x SB x 32 FMA
-// pass.  Items are claimed in dependency order with an atomic counter by a persistent
+// product, so the chain from block to block is one flag hop plus one SB x SB x RC product.  Items are claimed in dependency order with an atomic counter by a persistent
 // grid (a CTA only waits on items claimed before its own, so every wait ends); a block's
 // result is published with a release flag, consumers acquire it.  Each CTA stages the
 // L block it needs in shared memory before waiting for the flag, so the HBM read of L
 // (the dominant traffic: the lower triangle once per sweep) overlaps the wavefront.
-// Arithmetic: FP64 FMA (SIMT; on B200 DFMA and DMMA share the 37 TF/s FP64 peak).
+// Arithmetic: FP64 DMMA (m8n8k4) at SB = 96, FP64 FMA in the SIMT sweeps.
 #include <cuda.h>
 #include <cuda_runtime.h>
 #include <stdint.h>
