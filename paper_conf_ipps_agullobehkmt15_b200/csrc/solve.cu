@@ -679,7 +679,7 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
   const double* inv = aux;
   const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
   auto block_mma = [&](const double* Ls, const double* Ys, double (&acc)[3][NI][2]) {
-#pragma unroll 4
+#pragma unroll  // all 24 k-steps (measured: 0.7-1% faster than unroll 4)
     for (int k0 = 0; k0 < SB; k0 += 4) {
       double a[3], bv[NI];
 #pragma unroll
