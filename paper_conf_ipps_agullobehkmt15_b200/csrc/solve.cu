@@ -524,7 +524,7 @@ __global__ void __launch_bounds__(kSolveThreads, 1)
   const double* Mch = aux + (FWD ? 1 : 2) * (int64_t)nblocks * bsz;
   // acc (+)= Op(Ls) Ys over k = 0..SB-1
   auto block_mma = [&](const double* Ls, double (&acc)[3][NI][2]) {
-#pragma unroll 4
+#pragma unroll
     for (int k0 = 0; k0 < SB; k0 += 4) {
       double a[3], bv[NI];
 #pragma unroll
